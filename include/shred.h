@@ -1,0 +1,160 @@
+/*
+ * shred.h — C ABI of the B200-native content-defined chunker (Shredder's hot path).
+ *
+ * What it computes (PAPER.md, Bhatotia/Rodrigues/Verma, FAST'12):
+ *   * L245-L258 (§2.1, Eq. (1)): a Rabin fingerprint over sliding windows of w contiguous
+ *     bytes — the window, read as a polynomial over GF(2), reduced modulo an irreducible
+ *     polynomial div(x) of degree k ("the remainder r(x) obtained by division of f(x)").
+ *   * L444-L454 (§3.1): w = 48 bytes; a cut where the low-order 13 bits of the fingerprint
+ *     equal a pre-defined marker; slide one byte forward and repeat.
+ *   * L259-L269 (§2.1): min/max chunk sizes; min = 0, max = inf by default.
+ *   * L416-L434 (§3.1): boundaries are handed to the application ("upcall") — here: written
+ *     as ascending absolute u64 offsets into a caller buffer, on a CUDA stream.
+ * Readings where the paper is silent (polynomial, marker value, bit order, cut position,
+ * stream start/end, min/max off-by-ones) are DESIGN.md "Readings" Q1..Q17.
+ *
+ * Cut offset convention: a window ending at byte i (bytes i-w+1..i) that matches yields the
+ * cut c = i+1 (exclusive end of the chunk).  Only full windows are tested (c >= w); c = N
+ * (the stream end) is never emitted.  Forced max-size cuts may be < w.
+ *
+ * Conventions for every call:
+ *   Ownership   The caller owns every pointer it passes (inputs, d_out, n_out); they must stay
+ *               valid and unmodified until the work enqueued on `stream` completes.  The
+ *               library owns the ctx, its device tables, scratch, ring slots, copy stream and
+ *               events.  Fed bytes that must be carried (the last w-1) are copied into
+ *               library memory, so a fed buffer may be reused once the call's work completes.
+ *   Memory      d_* = device memory (cudaMalloc / torch CUDA tensor).  n_out = device memory or
+ *               mapped page-locked host memory (cudaHostAlloc; written by a kernel).
+ *   Async       Calls enqueue on `stream` and return; nothing is synchronised unless stated.
+ *               A ctx is bound to one device and is not re-entrant (one caller thread at a time).
+ *   Errors      Negative return codes are synchronous problems (parameters, enqueue,
+ *               allocation).  Output-capacity overflow is in-band: *n_out receives the TRUE
+ *               count n and min(n, cap) offsets are written (snprintf convention).  In the
+ *               streaming calls an overflow loses emitted offsets, so the ctx turns sticky
+ *               SHRED_ECAPACITY (checked at the next call, which is refused).
+ */
+#ifndef SHRED_H
+#define SHRED_H
+
+#include <stdint.h>
+#include <stddef.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct CUstream_st *shred_stream_t;   /* == cudaStream_t; NULL = legacy default stream */
+
+typedef struct shred_params {
+    uint64_t poly;      /* div(x) over GF(2): bit t = coefficient of x^t; irreducible,
+                           8 <= deg <= 63.  Default 0xbfe6b8a5bf378d83 (deg 63, reading Q1).  */
+    uint32_t window;    /* w bytes, 1 <= w <= 4096.  Default 48 (L444-L446).                   */
+    uint32_t reserved;  /* must be 0                                                           */
+    uint64_t divisor;   /* D, power of two, 2 <= D <= 2^deg.  Default 8192 ("13 bits", L447).   */
+    uint64_t magic;     /* r < D.  Default 0x78 (reading Q6).                                  */
+    uint64_t min_size;  /* 0 = off (paper default)                                  */
+    uint64_t max_size;  /* 0 = off (= inf).  Else max_size >= max(min_size, 1)                 */
+} shred_params;
+
+typedef struct shred_ctx shred_ctx;   /* opaque; bound to one CUDA device */
+
+enum {
+    SHRED_OK        =  0,
+    SHRED_EINVAL    = -1,   /* bad parameter / pointer kind / length                          */
+    SHRED_ENOMEM    = -2,   /* device or host allocation failed                              */
+    SHRED_ECUDA     = -3,   /* a CUDA call failed at enqueue (see shred_last_error)          */
+    SHRED_ESTATE    = -4,   /* misuse of the streaming state                                 */
+    SHRED_ECAPACITY = -5    /* sticky: a streaming call overflowed its output buffer         */
+};
+
+/* Kernel paths the ctx selected for its parameters (shred_path). */
+enum {
+    SHRED_PATH_K63     = 1, /* deg(P) = 63, D <= 2^32: u64 state, TMA-staged, smem LDS.64 tables */
+    SHRED_PATH_K32     = 2, /* deg(P) = 32, D <= 2^32: u32 state, TMA-staged, smem LDS.32 tables */
+    SHRED_PATH_GENERIC = 3  /* any other valid parameters: byte-at-a-time kernel                */
+};
+
+/* Fill *p with the paper defaults (readings Q1, Q5, Q6, Q15): P = 0xbfe6b8a5bf378d83, w = 48,
+   D = 8192, r = 0x78, min = 0, max = 0 (off). */
+void        shred_default_params(shred_params *p);
+
+/* Validate *p (degree, irreducibility of P by Ben-Or's test, D power of two, r < D,
+   min/max), build the push/pop tables (PAPER.md: "shifting a byte forward") on the
+   host, upload them to `device` and create the ctx.  Synchronous.  *out = NULL on error. */
+int         shred_init(const shred_params *p, int device, shred_ctx **out);
+
+/* Synchronise the ctx's own streams and free everything it owns.  NULL is a no-op. */
+void        shred_destroy(shred_ctx *ctx);
+
+const char *shred_strerror(int code);
+const char *shred_last_error(const shred_ctx *ctx);   /* detail incl. the CUDA error string  */
+int         shred_path(const shred_ctx *ctx);         /* SHRED_PATH_* chosen at init          */
+int         shred_get_params(const shred_ctx *ctx, shred_params *out);
+
+/* An output capacity that can never overflow for `len` input bytes:
+   len-1 if min = 0 (a candidate can occur at every position), else floor((len-1)/min) + 1. */
+uint64_t    shred_max_cuts(const shred_ctx *ctx, uint64_t len);
+
+/* One-shot, device-resident chunking of d_in[0..len) as a whole stream.
+   Writes the ascending final cuts (candidates, then the size rule if min > 0 or max > 0) to
+   d_out[0 .. min(n, cap)) and n to *n_out.  d_in may have any alignment.  len = 0 is valid
+   (n = 0).  Enqueues on `stream`, returns after enqueue. */
+int shred_chunk(shred_ctx *ctx, const uint8_t *d_in, uint64_t len,
+                uint64_t *d_out, uint64_t cap, uint64_t *n_out, shred_stream_t stream);
+
+/* Shard primitive for byte-range sharding (multi-GPU: "a small overlap of
+   the size of the sliding window (w bytes) near partition boundaries").
+   d_in points at stream position `start - halo`; the shard's own bytes are
+   d_in[halo .. halo+len) = stream positions [start, start+len).  halo must equal
+   min(w-1, start).  Tests every window ending at i in [start, start+len) with i >= w-1 and
+   writes the cut CANDIDATES c = i+1 with c < total_len (absolute offsets, ascending) — no size
+   rule — to d_out[0 .. min(n, cap)), n to *n_out. */
+int shred_candidates_range(shred_ctx *ctx, const uint8_t *d_in, uint64_t halo, uint64_t start,
+                           uint64_t len, uint64_t total_len,
+                           uint64_t *d_out, uint64_t cap, uint64_t *n_out, shred_stream_t stream);
+
+/* The size rule (readings Q12-Q15) over n_cand ascending candidates of a
+   stream of total_len bytes (e.g. the concatenated per-shard candidate lists).  Uses the
+   ctx's min/max; with both off it copies.  Writes cuts to d_out (cap, n_out as above).
+   d_cand and d_out must not overlap. */
+int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, uint64_t total_len,
+                     uint64_t *d_out, uint64_t cap, uint64_t *n_out, shred_stream_t stream);
+
+/* Streaming with carried window and size-rule state (§4.1-§4.2: pinned
+   buffers, async transfers, multi-buffering).  `in` is device memory or page-locked host
+   memory (pageable host memory -> SHRED_EINVAL).  Host input is copied by the ctx's own copy
+   stream into a ring of device slots (double/triple buffering) while the previous slot is
+   chunked on `stream`.  Offsets are absolute stream positions.  Only final cuts are emitted:
+   a cut at exactly the current stream end is held until the next feed (emitted) or the flush
+   (dropped: c = N is never a cut).  len may be 0. */
+int shred_feed (shred_ctx *ctx, const void *in, uint64_t len,
+                uint64_t *d_out, uint64_t cap, uint64_t *n_out, shred_stream_t stream);
+/* End the stream: emits the remaining forced max-size cuts and resets the stream state. */
+int shred_flush(shred_ctx *ctx, uint64_t *d_out, uint64_t cap, uint64_t *n_out,
+                shred_stream_t stream);
+/* Discard the stream state (synchronises the ctx's streams; clears a sticky error). */
+int shred_reset(shred_ctx *ctx);
+/* Ring configuration for host-fed input: `slots` in {1,2,3,4} device slots of `slot_bytes`
+   each (default 2 x 256 MiB, allocated at the first host feed).  Only between streams. */
+int shred_set_ring(shred_ctx *ctx, int slots, uint64_t slot_bytes);
+
+/* Bench/test helper (not the method): writes bytes [offset, offset+len) of the counter-mode
+   SplitMix64 stream `seed` into d_buf on `stream`. */
+int shred_synth_fill(uint8_t *d_buf, uint64_t len, uint64_t seed, uint64_t offset,
+                     shred_stream_t stream);
+
+/* Diagnostics for the bench: kernel launches enqueued by this ctx since creation. */
+uint64_t shred_launch_count(const shred_ctx *ctx);
+
+/* Diagnostics for the bench's roofline: while enabled, the ctx records a CUDA event pair on the
+   launching stream around every launch of the hot kernel (k1_bulk).  shred_profile_read
+   synchronises on the recorded events and returns the summed device time of those launches,
+   their number and the input bytes they covered (algorithmic bytes = 1 per input byte), then
+   clears the record.  enable = 0 stops recording. */
+int shred_profile(shred_ctx *ctx, int enable);
+int shred_profile_read(shred_ctx *ctx, double *ms, uint64_t *launches, uint64_t *bytes);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* SHRED_H */

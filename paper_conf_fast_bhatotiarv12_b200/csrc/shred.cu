@@ -1,0 +1,725 @@
+// shred.cu — host side of the C ABI declared in include/shred.h.
+//
+// Owns: parameter validation (incl. an irreducibility test of div(x)),
+// host construction of the push/pop tables, the per-ctx device buffers, the launch sequence
+//   K1 (k1_bulk TMA hot loop + k1_generic head/tail) -> k_scan -> k_scatter [-> k_size_bound]
+// and the host-fed streaming ring (§4.1-§4.2: pinned buffers, async H2D on a copy
+// stream, double/triple buffering of device slots).  No CPU fallback: every step of the path
+// runs in the kernels of kernels.cuh.
+#include "kernels.cuh"
+#include "../../include/shred.h"
+
+#include <cstdarg>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <mutex>
+#include <string>
+#include <vector>
+
+using namespace shred;
+
+// ============================================================================ GF(2) on the host
+// Polynomials over GF(2) in a u64 (bit t = coefficient of x^t).  Used only to build tables.
+namespace {
+
+int deg64(uint64_t p) { return p ? 63 - __builtin_clzll(p) : -1; }
+
+// a * x mod P  (deg a < k, P of degree k <= 63)
+inline uint64_t mulx(uint64_t a, uint64_t P, int k) {
+    a <<= 1;
+    if ((a >> k) & 1u) a ^= P;
+    return a;
+}
+// a * b mod P, Horner over the bits of b from the top
+uint64_t mulmod(uint64_t a, uint64_t b, uint64_t P, int k) {
+    uint64_t acc = 0;
+    for (int t = k - 1; t >= 0; --t) {
+        acc = mulx(acc, P, k);
+        if ((b >> t) & 1u) acc ^= a;
+    }
+    return acc;
+}
+uint64_t gcd2(uint64_t a, uint64_t b) {
+    while (b) {
+        while (a && deg64(a) >= deg64(b)) a ^= b << (deg64(a) - deg64(b));
+        std::swap(a, b);
+    }
+    return a;
+}
+// Ben-Or: P of degree k is irreducible iff gcd(x^(2^i) - x mod P, P) = 1 for i = 1..k/2.
+bool irreducible(uint64_t P) {
+    const int k = deg64(P);
+    if (k < 1) return false;
+    uint64_t xp = 2u;                    // x^(2^0) = x  (k >= 2 here)
+    if (k == 1) return true;
+    for (int i = 1; i <= k / 2; ++i) {
+        xp = mulmod(xp, xp, P, k);       // x^(2^i)
+        if (gcd2(P, xp ^ 2u) != 1u) return false;
+    }
+    return true;
+}
+// t(x) * x^e mod P for every byte t, via the 8 basis values x^(e+j) mod P.
+void byte_times_xpow(uint64_t P, int k, uint64_t e, uint64_t out[256]) {
+    uint64_t xe = 1u;                    // x^0
+    for (uint64_t n = 0; n < e; ++n) xe = mulx(xe, P, k);
+    uint64_t basis[8];
+    for (int j = 0; j < 8; ++j) { basis[j] = xe; xe = mulx(xe, P, k); }
+    for (int t = 0; t < 256; ++t) {
+        uint64_t v = 0;
+        for (int j = 0; j < 8; ++j) if ((t >> j) & 1) v ^= basis[j];
+        out[t] = v;
+    }
+}
+
+typedef CUresult (*EncodeTiledFn)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *,
+                                  const cuuint64_t *, const cuuint64_t *, const cuuint32_t *,
+                                  const cuuint32_t *, CUtensorMapInterleave, CUtensorMapSwizzle,
+                                  CUtensorMapL2promotion, CUtensorMapFloatOOBfill);
+
+const char *kErr[] = {"ok", "invalid argument", "out of memory", "CUDA error",
+                      "invalid stream state", "output capacity exceeded (sticky)"};
+
+}  // namespace
+
+// ============================================================================ ctx
+struct shred_ctx {
+    shred_params p{};
+    int device = 0;
+    int path = 0;
+    int k = 0;
+    DevParams dp{};
+    uint4 *d_tab_img = nullptr;          // 64 KiB replicated T|U image (fast paths)
+    GenTables *d_gen = nullptr;          // plain T/U (generic path, recompute)
+    EncodeTiledFn encode = nullptr;
+    int sm_count = 148;
+
+    // scratch (grown on demand, synchronously)
+    uint32_t *d_counts = nullptr; uint64_t counts_cap = 0;
+    uint64_t *d_offsets = nullptr; uint64_t offsets_cap = 0;
+    uint64_t *d_scratch = nullptr; uint64_t scratch_cap = 0;   // in u64 entries
+    uint64_t *d_cand = nullptr; uint64_t cand_cap = 0;         // bounded mode ordered list
+    Aux *d_aux = nullptr;                // [0] one-shot calls, [1] the stream
+    uint64_t *h_pinned = nullptr;        // small pinned readback area
+    uint64_t *h_flag = nullptr;          // mapped pinned word: a streaming call overflowed
+    uint64_t *d_flag = nullptr;          // its device alias
+
+    // streaming state (host mirror)
+    uint64_t pos = 0;                    // bytes fed so far
+    uint8_t *d_carry[2] = {nullptr, nullptr};
+    int carry_idx = 0;
+    uint32_t carry_len = 0;
+    int sticky = SHRED_OK;
+    int ring_n = 2; uint64_t ring_bytes = 256ull << 20;
+    std::vector<uint8_t *> ring;
+    std::vector<cudaEvent_t> ev_free, ev_ready;
+    int ring_next = 0;
+    cudaStream_t copy_stream = nullptr;
+
+    uint64_t launches = 0;
+    std::string last_error;
+
+    // hot-kernel profiling (shred_profile)
+    bool prof = false;
+    std::vector<cudaEvent_t> prof_ev;    // pool, pairs
+    size_t prof_used = 0;
+    uint64_t prof_bytes = 0;
+};
+
+namespace {
+
+int fail(shred_ctx *c, int code, const char *fmt, ...) {
+    if (c) {
+        char buf[512];
+        va_list ap; va_start(ap, fmt); vsnprintf(buf, sizeof buf, fmt, ap); va_end(ap);
+        c->last_error = buf;
+    }
+    return code;
+}
+int cuda_fail(shred_ctx *c, cudaError_t e, const char *what) {
+    return fail(c, SHRED_ECUDA, "%s: %s", what, cudaGetErrorString(e));
+}
+#define CK(call, what) do { cudaError_t _e = (call); if (_e != cudaSuccess) return cuda_fail(ctx, _e, what); } while (0)
+#define LAUNCHED(what) do { ++ctx->launches; cudaError_t _e = cudaGetLastError(); if (_e != cudaSuccess) return cuda_fail(ctx, _e, what); } while (0)
+
+template <class T>
+int grow(shred_ctx *ctx, T *&ptr, uint64_t &cap, uint64_t need, const char *what) {
+    if (need <= cap) return SHRED_OK;
+    uint64_t n = need + need / 4 + 64;
+    if (ptr) { cudaDeviceSynchronize(); cudaFree(ptr); ptr = nullptr; cap = 0; }
+    cudaError_t e = cudaMalloc(&ptr, n * sizeof(T));
+    if (e != cudaSuccess) { cudaGetLastError(); return fail(ctx, SHRED_ENOMEM, "%s: cudaMalloc(%llu B) failed", what, (unsigned long long)(n * sizeof(T))); }
+    cap = n;
+    return SHRED_OK;
+}
+
+// Validation of shred_params (include/shred.h).
+int validate(const shred_params *p, shred_ctx *ctx) {
+    if (!p) return fail(ctx, SHRED_EINVAL, "params is NULL");
+    const int k = deg64(p->poly);
+    if (k < 8 || k > 63) return fail(ctx, SHRED_EINVAL, "deg(poly) = %d, need 8..63", k);
+    if (!irreducible(p->poly)) return fail(ctx, SHRED_EINVAL, "poly 0x%llx is reducible", (unsigned long long)p->poly);
+    if (p->window < 1 || p->window > 4096) return fail(ctx, SHRED_EINVAL, "window %u not in 1..4096", p->window);
+    if (p->reserved != 0) return fail(ctx, SHRED_EINVAL, "reserved field must be 0");
+    if (p->divisor < 2 || (p->divisor & (p->divisor - 1))) return fail(ctx, SHRED_EINVAL, "divisor must be a power of two >= 2");
+    if (deg64(p->divisor) > k) return fail(ctx, SHRED_EINVAL, "divisor exceeds 2^deg(poly)");
+    if (p->magic >= p->divisor) return fail(ctx, SHRED_EINVAL, "magic must be < divisor");
+    if (p->max_size && p->max_size < (p->min_size > 1 ? p->min_size : 1))
+        return fail(ctx, SHRED_EINVAL, "max_size must be >= max(min_size, 1)");
+    return SHRED_OK;
+}
+
+// ---------------------------------------------------------------------------- job planning
+struct Plan {
+    Job J;
+    bool bulk = false;
+    uint32_t nslots = 0;
+    uint32_t bulk_ctas = 0;
+    CUtensorMap tmap;
+};
+
+// Plan candidate detection for window ends [t_begin, t_end) of a job whose bytes start at
+// stream position p_begin (src) with `prefix_len` carried bytes before it.
+int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, const uint8_t *prefix,
+             uint32_t prefix_len, uint64_t t_begin, uint64_t t_end, uint64_t c_limit) {
+    Job &J = pl.J;
+    J = Job{};
+    J.src = src; J.p_begin = p_begin; J.prefix = prefix; J.prefix_len = prefix_len;
+    J.min_i = (uint64_t)ctx->p.window - 1u;
+    J.c_limit = c_limit;
+    SlotMap &m = J.map;
+    m.t_end = t_end;
+    const uint64_t len = t_end > t_begin ? t_end - t_begin : 0;
+    const uint64_t GS = 256;                   // generic head/tail segment
+
+    // bulk region: aligned start b0 >= max(t_begin, p_begin + 64), rows of S bytes
+    pl.bulk = false;
+    uint64_t S = 0, nrows = 0, b0 = t_end;
+    if ((ctx->path == SHRED_PATH_K63 || ctx->path == SHRED_PATH_K32) && len >= 4096) {
+        uint64_t lo = t_begin > p_begin + 64 ? t_begin : p_begin + 64;
+        const uintptr_t a = (uintptr_t)(src + (lo - p_begin));
+        b0 = lo + ((16u - (a & 15u)) & 15u);
+        if (b0 < t_end) {
+            const uint64_t blen = t_end - b0;
+            const uint64_t target = (uint64_t)ctx->sm_count * NT;
+            S = (blen + target - 1) / target;
+            S = (S + ROUND - 1) / ROUND * ROUND;
+            if (S < 256) S = 256;
+            nrows = blen / S;
+            if (nrows > 0 && nrows < (1ull << 31) && S < (1ull << 39)) pl.bulk = true;
+        }
+    }
+    if (!pl.bulk) {
+        // everything generic: segments of about len / (sm_count * 4 * 256) bytes, >= GS
+        uint64_t seg = GS;
+        const uint64_t want = (uint64_t)ctx->sm_count * 4 * GEN_THREADS;
+        if (len / want > seg) seg = (len / want + 63) / 64 * 64;
+        m.head_start = t_begin; m.head_seg = seg;
+        m.n_head = (uint32_t)((len + seg - 1) / seg);
+        m.nrows = 0; m.b0 = t_end; m.S = 0;
+        m.tail_start = t_end; m.tail_seg = GS; m.n_tail = 0;
+    } else {
+        m.head_start = t_begin; m.head_seg = GS;
+        m.n_head = (uint32_t)((b0 - t_begin + GS - 1) / GS);
+        m.b0 = b0; m.S = S; m.nrows = (uint32_t)nrows;
+        m.tail_start = b0 + nrows * S; m.tail_seg = GS;
+        m.n_tail = (uint32_t)((t_end - m.tail_start + GS - 1) / GS);
+        pl.bulk_ctas = (uint32_t)((nrows + NT - 1) / NT);
+        // 2-D tensor map [nrows][S] over the bulk bytes
+        cuuint64_t gdim[2] = {(cuuint64_t)S, (cuuint64_t)nrows};
+        cuuint64_t gstride[1] = {(cuuint64_t)S};
+        cuuint32_t box[2] = {(cuuint32_t)ROUND, (cuuint32_t)BOX_ROWS};
+        cuuint32_t estr[2] = {1, 1};
+        CUresult r = ctx->encode(&pl.tmap, CU_TENSOR_MAP_DATA_TYPE_UINT8, 2,
+                                 (void *)(src + (b0 - p_begin)), gdim, gstride, box, estr,
+                                 CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_64B,
+                                 CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+        if (r != CUDA_SUCCESS) return fail(ctx, SHRED_ECUDA, "cuTensorMapEncodeTiled failed (%d)", (int)r);
+    }
+    pl.nslots = m.n_head + m.nrows + m.n_tail;
+    // per-slot list capacity: twice the expected count of the longest segment + slack
+    const uint64_t maxseg = pl.bulk ? (S > GS ? S : GS) : m.head_seg;
+    uint64_t cap = 2 * maxseg / ctx->p.divisor + 16;
+    if (cap > 256) cap = 256;
+    J.cap = (uint32_t)cap;
+    int rc;
+    if ((rc = grow(ctx, ctx->d_counts, ctx->counts_cap, (uint64_t)pl.nslots + 1, "counts"))) return rc;
+    if ((rc = grow(ctx, ctx->d_offsets, ctx->offsets_cap, (uint64_t)pl.nslots + 1, "offsets"))) return rc;
+    if ((rc = grow(ctx, ctx->d_scratch, ctx->scratch_cap, (uint64_t)pl.nslots * cap + 1, "scratch"))) return rc;
+    J.counts = ctx->d_counts;
+    J.scratch = ctx->d_scratch;
+    return SHRED_OK;
+}
+
+// K1 (bulk + generic) and k_scan.
+int launch_detect(shred_ctx *ctx, Plan &pl, Aux *aux, uint64_t *n_direct, uint64_t direct_cap,
+                  cudaStream_t st) {
+    if (pl.nslots == 0) {
+        // nothing to test: total = 0
+        k_scan<<<1, 1024, 0, st>>>(ctx->d_counts, 0, ctx->d_offsets, aux, n_direct, direct_cap);
+        LAUNCHED("k_scan");
+        return SHRED_OK;
+    }
+    if (pl.bulk) {
+        cudaEvent_t e0 = nullptr, e1 = nullptr;
+        if (ctx->prof) {
+            if (ctx->prof_used + 2 > ctx->prof_ev.size()) {
+                for (int i = 0; i < 64; ++i) {
+                    cudaEvent_t e;
+                    CK(cudaEventCreate(&e), "profile event");
+                    ctx->prof_ev.push_back(e);
+                }
+            }
+            e0 = ctx->prof_ev[ctx->prof_used]; e1 = ctx->prof_ev[ctx->prof_used + 1];
+            ctx->prof_used += 2;
+            ctx->prof_bytes += (uint64_t)pl.J.map.nrows * pl.J.map.S;
+            CK(cudaEventRecord(e0, st), "profile record");
+        }
+        if (ctx->path == SHRED_PATH_K63)
+            k1_bulk<MODE_K63><<<pl.bulk_ctas, NT + 32, BULK_SMEM, st>>>(pl.tmap, ctx->d_tab_img, pl.J,
+                                                                        (uint32_t)ctx->dp.dmask, (uint32_t)ctx->dp.magic);
+        else
+            k1_bulk<MODE_K32><<<pl.bulk_ctas, NT + 32, BULK_SMEM, st>>>(pl.tmap, ctx->d_tab_img, pl.J,
+                                                                        (uint32_t)ctx->dp.dmask, (uint32_t)ctx->dp.magic);
+        LAUNCHED("k1_bulk");
+        if (e1) CK(cudaEventRecord(e1, st), "profile record");
+    }
+    const uint32_t ngen = pl.J.map.n_head + pl.J.map.n_tail;
+    if (ngen) {
+        k1_generic<<<(ngen + GEN_THREADS - 1) / GEN_THREADS, GEN_THREADS, 0, st>>>(pl.J, ctx->dp, ctx->d_gen);
+        LAUNCHED("k1_generic");
+    }
+    k_scan<<<1, 1024, 0, st>>>(ctx->d_counts, pl.nslots, ctx->d_offsets, aux, n_direct, direct_cap);
+    LAUNCHED("k_scan");
+    return SHRED_OK;
+}
+
+int launch_scatter(shred_ctx *ctx, Plan &pl, uint64_t *dst, uint64_t dst_cap, Aux *aux, int streaming,
+                   cudaStream_t st) {
+    if (pl.nslots == 0) return SHRED_OK;
+    k_scatter<<<(pl.nslots + 255) / 256, 256, 0, st>>>(pl.J, ctx->dp, ctx->d_gen, pl.nslots, ctx->d_offsets,
+                                                       dst, dst_cap, aux, streaming);
+    LAUNCHED("k_scatter");
+    return SHRED_OK;
+}
+
+bool bounded(const shred_ctx *ctx) { return ctx->p.min_size > 0 || ctx->p.max_size > 0; }
+
+// Bounded mode needs the whole ordered candidate list: read the count back (the one
+// synchronous point of the bounded path) and size the ctx buffer for it.
+int ensure_cand(shred_ctx *ctx, Aux *aux, cudaStream_t st, uint64_t &total) {
+    CK(cudaMemcpyAsync(ctx->h_pinned, &aux->total, sizeof(uint64_t), cudaMemcpyDeviceToHost, st), "read total");
+    CK(cudaStreamSynchronize(st), "sync total");
+    total = ctx->h_pinned[0];
+    return grow(ctx, ctx->d_cand, ctx->cand_cap, total + 1, "candidate list");
+}
+
+// One piece of a stream (or a whole one-shot stream): window ends [t_begin, t_end).
+// aux->out_pos is the output cursor; results are appended to dst.
+int run_piece(shred_ctx *ctx, Aux *aux, const uint8_t *src, uint64_t p_begin, const uint8_t *prefix,
+              uint32_t prefix_len, uint64_t t_begin, uint64_t t_end, uint64_t c_limit, int final_,
+              uint64_t *dst, uint64_t dst_cap, cudaStream_t st) {
+    Plan pl;
+    int rc = plan_job(ctx, pl, src, p_begin, prefix, prefix_len, t_begin, t_end, c_limit);
+    if (rc) return rc;
+    if ((rc = launch_detect(ctx, pl, aux, nullptr, 0, st))) return rc;
+    if (!bounded(ctx)) {
+        if ((rc = launch_scatter(ctx, pl, dst, dst_cap, aux, 1, st))) return rc;
+        if (final_) {
+            // one-shot: nothing held; out_pos += total
+            k_piece_done<<<1, 1, 0, st>>>(aux, dst, dst_cap, ~0ull);
+        } else {
+            k_piece_done<<<1, 1, 0, st>>>(aux, dst, dst_cap, t_end);
+        }
+        LAUNCHED("k_piece_done");
+        return SHRED_OK;
+    }
+    uint64_t total = 0;
+    if ((rc = ensure_cand(ctx, aux, st, total))) return rc;
+    if ((rc = launch_scatter(ctx, pl, ctx->d_cand, ctx->cand_cap, aux, 0, st))) return rc;
+    k_size_bound<<<1, 32, 0, st>>>(ctx->d_cand, &aux->total, 0, t_end, final_, ctx->p.min_size,
+                                   ctx->p.max_size, dst, dst_cap, aux);
+    LAUNCHED("k_size_bound");
+    return SHRED_OK;
+}
+
+// Kind of a user pointer: 1 = device, 2 = page-locked host, 0 = pageable / unknown.
+int ptr_kind(const void *p) {
+    cudaPointerAttributes a;
+    cudaError_t e = cudaPointerGetAttributes(&a, p);
+    if (e != cudaSuccess) { cudaGetLastError(); return 0; }
+    if (a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged) return 1;
+    if (a.type == cudaMemoryTypeHost) return 2;
+    return 0;
+}
+
+int check_out(shred_ctx *ctx, uint64_t *d_out, uint64_t cap, uint64_t *n_out) {
+    if (!n_out) return fail(ctx, SHRED_EINVAL, "n_out is NULL");
+    if (cap && !d_out) return fail(ctx, SHRED_EINVAL, "d_out is NULL with cap > 0");
+    return SHRED_OK;
+}
+
+struct DevGuard {
+    int prev = -1;
+    explicit DevGuard(int dev) { cudaGetDevice(&prev); if (prev != dev) cudaSetDevice(dev); }
+    ~DevGuard() { if (prev >= 0) cudaSetDevice(prev); }
+};
+
+}  // namespace
+
+// ============================================================================ C ABI
+extern "C" {
+
+void shred_default_params(shred_params *p) {
+    if (!p) return;
+    memset(p, 0, sizeof *p);
+    p->poly = 0xbfe6b8a5bf378d83ull;
+    p->window = 48;
+    p->divisor = 8192;
+    p->magic = 0x78;
+}
+
+const char *shred_strerror(int code) {
+    if (code > 0 || code < -5) return "unknown error";
+    return kErr[-code];
+}
+
+const char *shred_last_error(const shred_ctx *ctx) { return ctx ? ctx->last_error.c_str() : "no ctx"; }
+int shred_path(const shred_ctx *ctx) { return ctx ? ctx->path : 0; }
+uint64_t shred_launch_count(const shred_ctx *ctx) { return ctx ? ctx->launches : 0; }
+
+int shred_get_params(const shred_ctx *ctx, shred_params *out) {
+    if (!ctx || !out) return SHRED_EINVAL;
+    *out = ctx->p;
+    return SHRED_OK;
+}
+
+uint64_t shred_max_cuts(const shred_ctx *ctx, uint64_t len) {
+    if (!ctx || len < 2) return 0;
+    if (ctx->p.min_size == 0) return len - 1;
+    return (len - 1) / ctx->p.min_size + 1;
+}
+
+int shred_init(const shred_params *p, int device, shred_ctx **out) {
+    if (!out) return SHRED_EINVAL;
+    *out = nullptr;
+    int rc = validate(p, nullptr);
+    if (rc) return rc;
+    shred_ctx *ctx = new shred_ctx();
+    ctx->p = *p;
+    ctx->device = device;
+    DevGuard g(device);
+    auto bail = [&](int code) { shred_destroy(ctx); return code; };
+    cudaError_t e = cudaSetDevice(device);
+    if (e != cudaSuccess) return bail(SHRED_ECUDA);
+    int major = 0;
+    cudaDeviceGetAttribute(&major, cudaDevAttrComputeCapabilityMajor, device);
+    cudaDeviceGetAttribute(&ctx->sm_count, cudaDevAttrMultiProcessorCount, device);
+    if (ctx->sm_count <= 0) ctx->sm_count = 148;
+
+    const int k = deg64(p->poly);
+    ctx->k = k;
+    ctx->dp.k = (uint32_t)k;
+    ctx->dp.w = p->window;
+    ctx->dp.kmask = (1ull << k) - 1ull;
+    ctx->dp.dmask = p->divisor - 1ull;
+    ctx->dp.magic = p->magic;
+    const bool fast_w = (p->window == 48);
+    if (k == 63 && fast_w && p->divisor <= (1ull << 32)) ctx->path = SHRED_PATH_K63;
+    else if (k == 32 && fast_w && p->divisor <= (1ull << 32)) ctx->path = SHRED_PATH_K32;
+    else ctx->path = SHRED_PATH_GENERIC;
+    if (major != 10) ctx->path = SHRED_PATH_GENERIC;   // the TMA kernels are built for sm_100a only
+
+    // ---- tables (PAPER.md: shift one byte in, one byte out)
+    uint64_t Tk[256], U[256];
+    byte_times_xpow(p->poly, k, (uint64_t)k, Tk);                 // t x^k mod P
+    byte_times_xpow(p->poly, k, 8ull * p->window, U);             // o x^{8w} mod P
+    GenTables gt;
+    for (int t = 0; t < 256; ++t) { gt.T[t] = Tk[t]; gt.U[t] = U[t]; }
+    std::vector<uint8_t> img(TAB_BYTES, 0);
+    if (ctx->path == SHRED_PATH_K63) {
+        uint64_t T63[256];
+        byte_times_xpow(p->poly, k, 63, T63);                     // t x^63 mod P
+        for (int t = 0; t < 256; ++t) {
+            uint64_t tv = T63[t] ^ ((uint64_t)(t & 1) << 63);     // cancel bit left at 2^63
+            for (int r = 0; r < 16; ++r) {
+                memcpy(&img[t * 256 + r * 8], &tv, 8);
+                memcpy(&img[t * 256 + 128 + r * 8], &U[t], 8);
+            }
+        }
+    } else if (ctx->path == SHRED_PATH_K32) {
+        for (int t = 0; t < 256; ++t) {
+            uint32_t tv = (uint32_t)Tk[t], uv = (uint32_t)U[t];
+            for (int r = 0; r < 32; ++r) {
+                memcpy(&img[t * 256 + r * 4], &tv, 4);
+                memcpy(&img[t * 256 + 128 + r * 4], &uv, 4);
+            }
+        }
+    }
+    if (cudaMalloc(&ctx->d_gen, sizeof(GenTables)) != cudaSuccess ||
+        cudaMalloc(&ctx->d_tab_img, TAB_BYTES) != cudaSuccess ||
+        cudaMalloc(&ctx->d_aux, 2 * sizeof(Aux)) != cudaSuccess ||
+        cudaMalloc(&ctx->d_carry[0], 4096) != cudaSuccess ||
+        cudaMalloc(&ctx->d_carry[1], 4096) != cudaSuccess ||
+        cudaHostAlloc(&ctx->h_pinned, 64, cudaHostAllocDefault) != cudaSuccess ||
+        cudaHostAlloc(&ctx->h_flag, 64, cudaHostAllocMapped) != cudaSuccess ||
+        cudaHostGetDevicePointer((void **)&ctx->d_flag, ctx->h_flag, 0) != cudaSuccess) {
+        cudaGetLastError();
+        return bail(SHRED_ENOMEM);
+    }
+    ctx->h_flag[0] = 0;
+    if (cudaMemcpy(ctx->d_gen, &gt, sizeof gt, cudaMemcpyHostToDevice) != cudaSuccess ||
+        cudaMemcpy(ctx->d_tab_img, img.data(), TAB_BYTES, cudaMemcpyHostToDevice) != cudaSuccess ||
+        cudaMemset(ctx->d_aux, 0, 2 * sizeof(Aux)) != cudaSuccess)
+        return bail(SHRED_ECUDA);
+    if (ctx->path != SHRED_PATH_GENERIC) {
+        void *fn = nullptr;
+        cudaDriverEntryPointQueryResult q;
+        if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fn, cudaEnableDefault, &q) != cudaSuccess || !fn)
+            return bail(SHRED_ECUDA);
+        ctx->encode = (EncodeTiledFn)fn;
+        if (cudaFuncSetAttribute(k1_bulk<MODE_K63>, cudaFuncAttributeMaxDynamicSharedMemorySize, BULK_SMEM) != cudaSuccess ||
+            cudaFuncSetAttribute(k1_bulk<MODE_K32>, cudaFuncAttributeMaxDynamicSharedMemorySize, BULK_SMEM) != cudaSuccess)
+            return bail(SHRED_ECUDA);
+    }
+    if (cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking) != cudaSuccess)
+        return bail(SHRED_ECUDA);
+    if (cudaDeviceSynchronize() != cudaSuccess) return bail(SHRED_ECUDA);
+    *out = ctx;
+    return SHRED_OK;
+}
+
+void shred_destroy(shred_ctx *ctx) {
+    if (!ctx) return;
+    DevGuard g(ctx->device);
+    if (ctx->copy_stream) cudaStreamSynchronize(ctx->copy_stream);
+    cudaDeviceSynchronize();
+    for (auto &e : ctx->ev_free) cudaEventDestroy(e);
+    for (auto &e : ctx->ev_ready) cudaEventDestroy(e);
+    for (auto &e : ctx->prof_ev) cudaEventDestroy(e);
+    for (auto p : ctx->ring) cudaFree(p);
+    if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
+    cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_counts); cudaFree(ctx->d_offsets);
+    cudaFree(ctx->d_scratch); cudaFree(ctx->d_cand); cudaFree(ctx->d_aux);
+    cudaFree(ctx->d_carry[0]); cudaFree(ctx->d_carry[1]);
+    if (ctx->h_pinned) cudaFreeHost(ctx->h_pinned);
+    if (ctx->h_flag) cudaFreeHost(ctx->h_flag);
+    cudaGetLastError();
+    delete ctx;
+}
+
+int shred_chunk(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, uint64_t *d_out, uint64_t cap,
+                uint64_t *n_out, shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    int rc = check_out(ctx, d_out, cap, n_out);
+    if (rc) return rc;
+    if (len && !d_in) return fail(ctx, SHRED_EINVAL, "d_in is NULL");
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    Aux *aux = ctx->d_aux + 0;
+    k_stream_reset<<<1, 1, 0, st>>>(aux);
+    LAUNCHED("k_stream_reset");
+    if (!bounded(ctx)) {
+        Plan pl;
+        if ((rc = plan_job(ctx, pl, d_in, 0, nullptr, 0, 0, len, len))) return rc;
+        if ((rc = launch_detect(ctx, pl, aux, n_out, cap, st))) return rc;
+        return launch_scatter(ctx, pl, d_out, cap, aux, 0, st);
+    }
+    if ((rc = run_piece(ctx, aux, d_in, 0, nullptr, 0, 0, len, len, 1, d_out, cap, st))) return rc;
+    k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, nullptr);
+    LAUNCHED("k_call_end");
+    return SHRED_OK;
+}
+
+int shred_candidates_range(shred_ctx *ctx, const uint8_t *d_in, uint64_t halo, uint64_t start,
+                           uint64_t len, uint64_t total_len, uint64_t *d_out, uint64_t cap,
+                           uint64_t *n_out, shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    int rc = check_out(ctx, d_out, cap, n_out);
+    if (rc) return rc;
+    const uint64_t want = start < (uint64_t)ctx->p.window - 1u ? start : (uint64_t)ctx->p.window - 1u;
+    if (halo != want) return fail(ctx, SHRED_EINVAL, "halo must be min(w-1, start) = %llu", (unsigned long long)want);
+    if (start + len > total_len) return fail(ctx, SHRED_EINVAL, "start + len > total_len");
+    if ((len || halo) && !d_in) return fail(ctx, SHRED_EINVAL, "d_in is NULL");
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    Aux *aux = ctx->d_aux + 0;
+    k_stream_reset<<<1, 1, 0, st>>>(aux);
+    LAUNCHED("k_stream_reset");
+    Plan pl;
+    if ((rc = plan_job(ctx, pl, d_in, start - halo, nullptr, 0, start, start + len, total_len))) return rc;
+    if ((rc = launch_detect(ctx, pl, aux, n_out, cap, st))) return rc;
+    return launch_scatter(ctx, pl, d_out, cap, aux, 0, st);
+}
+
+int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, uint64_t total_len,
+                     uint64_t *d_out, uint64_t cap, uint64_t *n_out, shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    int rc = check_out(ctx, d_out, cap, n_out);
+    if (rc) return rc;
+    if (n_cand && !d_cand) return fail(ctx, SHRED_EINVAL, "d_cand is NULL");
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    Aux *aux = ctx->d_aux + 0;
+    k_stream_reset<<<1, 1, 0, st>>>(aux);
+    LAUNCHED("k_stream_reset");
+    k_size_bound<<<1, 32, 0, st>>>(d_cand, nullptr, n_cand, total_len, 1, ctx->p.min_size,
+                                   ctx->p.max_size, d_out, cap, aux);
+    LAUNCHED("k_size_bound");
+    k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, nullptr);
+    LAUNCHED("k_call_end");
+    return SHRED_OK;
+}
+
+// ---------------------------------------------------------------------------- streaming
+int shred_set_ring(shred_ctx *ctx, int slots, uint64_t slot_bytes) {
+    if (!ctx) return SHRED_EINVAL;
+    if (slots < 1 || slots > 4 || slot_bytes < 4096) return fail(ctx, SHRED_EINVAL, "ring: 1..4 slots of >= 4096 B");
+    if (ctx->pos != 0) return fail(ctx, SHRED_ESTATE, "ring can only change between streams");
+    DevGuard g(ctx->device);
+    if (ctx->copy_stream) cudaStreamSynchronize(ctx->copy_stream);
+    cudaDeviceSynchronize();
+    for (auto p : ctx->ring) cudaFree(p);
+    for (auto &e : ctx->ev_free) cudaEventDestroy(e);
+    for (auto &e : ctx->ev_ready) cudaEventDestroy(e);
+    ctx->ring.clear(); ctx->ev_free.clear(); ctx->ev_ready.clear();
+    ctx->ring_n = slots; ctx->ring_bytes = slot_bytes; ctx->ring_next = 0;
+    return SHRED_OK;
+}
+
+namespace {
+int ensure_ring(shred_ctx *ctx) {
+    if (!ctx->ring.empty()) return SHRED_OK;
+    for (int i = 0; i < ctx->ring_n; ++i) {
+        uint8_t *p = nullptr;
+        if (cudaMalloc(&p, ctx->ring_bytes) != cudaSuccess) { cudaGetLastError(); return fail(ctx, SHRED_ENOMEM, "ring slot alloc"); }
+        ctx->ring.push_back(p);
+        cudaEvent_t a, b;
+        cudaEventCreateWithFlags(&a, cudaEventDisableTiming);
+        cudaEventCreateWithFlags(&b, cudaEventDisableTiming);
+        ctx->ev_free.push_back(a); ctx->ev_ready.push_back(b);
+    }
+    return SHRED_OK;
+}
+
+// Process stream bytes [ctx->pos, ctx->pos + len) that are resident at device pointer `src`.
+int feed_device_piece(shred_ctx *ctx, const uint8_t *src, uint64_t len, uint64_t *d_out, uint64_t cap,
+                      cudaStream_t st) {
+    Aux *aux = ctx->d_aux + 1;
+    const uint8_t *prefix = ctx->d_carry[ctx->carry_idx];
+    int rc = run_piece(ctx, aux, src, ctx->pos, prefix, ctx->carry_len, ctx->pos, ctx->pos + len,
+                       ~0ull, 0, d_out, cap, st);
+    if (rc) return rc;
+    const uint32_t keep = ctx->p.window - 1u;
+    uint8_t *nc = ctx->d_carry[ctx->carry_idx ^ 1];
+    k_carry<<<1, 256, 0, st>>>(prefix, ctx->carry_len, src, len, nc, keep);
+    LAUNCHED("k_carry");
+    ctx->carry_idx ^= 1;
+    const uint64_t tot = (uint64_t)ctx->carry_len + len;
+    ctx->carry_len = (uint32_t)(tot < keep ? tot : keep);
+    ctx->pos += len;
+    return SHRED_OK;
+}
+}  // namespace
+
+int shred_feed(shred_ctx *ctx, const void *in, uint64_t len, uint64_t *d_out, uint64_t cap,
+               uint64_t *n_out, shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    // an earlier streaming call overflowed its output (observed once that call completed)
+    if (*(volatile uint64_t *)ctx->h_flag) ctx->sticky = SHRED_ECAPACITY;
+    if (ctx->sticky) return fail(ctx, ctx->sticky, "sticky error from an earlier call; shred_reset first");
+    int rc = check_out(ctx, d_out, cap, n_out);
+    if (rc) return rc;
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    Aux *aux = ctx->d_aux + 1;
+    k_call_begin<<<1, 1, 0, st>>>(aux);
+    LAUNCHED("k_call_begin");
+    if (len) {
+        if (!in) return fail(ctx, SHRED_EINVAL, "in is NULL");
+        const int kind = ptr_kind(in);
+        if (kind == 0) return fail(ctx, SHRED_EINVAL, "input must be device or page-locked host memory");
+        if (kind == 1) {
+            if ((rc = feed_device_piece(ctx, (const uint8_t *)in, len, d_out, cap, st))) return rc;
+        } else {
+            if ((rc = ensure_ring(ctx))) return rc;
+            const uint8_t *h = (const uint8_t *)in;
+            for (uint64_t off = 0; off < len; off += ctx->ring_bytes) {
+                const uint64_t n = (len - off) < ctx->ring_bytes ? (len - off) : ctx->ring_bytes;
+                const int s = ctx->ring_next;
+                ctx->ring_next = (s + 1) % ctx->ring_n;
+                // slot s is free once the compute stream finished its previous piece
+                CK(cudaStreamWaitEvent(ctx->copy_stream, ctx->ev_free[s], 0), "wait slot free");
+                CK(cudaMemcpyAsync(ctx->ring[s], h + off, n, cudaMemcpyHostToDevice, ctx->copy_stream), "H2D");
+                CK(cudaEventRecord(ctx->ev_ready[s], ctx->copy_stream), "record ready");
+                CK(cudaStreamWaitEvent(st, ctx->ev_ready[s], 0), "wait ready");
+                if ((rc = feed_device_piece(ctx, ctx->ring[s], n, d_out, cap, st))) return rc;
+                CK(cudaEventRecord(ctx->ev_free[s], st), "record free");
+            }
+        }
+    }
+    k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, ctx->d_flag);
+    LAUNCHED("k_call_end");
+    return SHRED_OK;
+}
+
+int shred_flush(shred_ctx *ctx, uint64_t *d_out, uint64_t cap, uint64_t *n_out, shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    int rc = check_out(ctx, d_out, cap, n_out);
+    if (rc) return rc;
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    // Every forced cut strictly inside the stream was emitted by the last feed; a cut held at
+    // exactly the stream end is dropped (c = N is never a cut, reading Q11).
+    k_stream_reset<<<1, 1, 0, st>>>(ctx->d_aux + 1);
+    LAUNCHED("k_stream_reset");
+    k_write_u64<<<1, 1, 0, st>>>(n_out, 0);
+    LAUNCHED("k_write_u64");
+    ctx->pos = 0; ctx->carry_len = 0; ctx->carry_idx = 0;
+    return SHRED_OK;
+}
+
+int shred_reset(shred_ctx *ctx) {
+    if (!ctx) return SHRED_EINVAL;
+    DevGuard g(ctx->device);
+    if (ctx->copy_stream) cudaStreamSynchronize(ctx->copy_stream);
+    cudaDeviceSynchronize();
+    cudaMemset(ctx->d_aux + 1, 0, sizeof(Aux));
+    cudaDeviceSynchronize();
+    ctx->pos = 0; ctx->carry_len = 0; ctx->carry_idx = 0; ctx->sticky = SHRED_OK;
+    ctx->h_flag[0] = 0;
+    return SHRED_OK;
+}
+
+int shred_profile(shred_ctx *ctx, int enable) {
+    if (!ctx) return SHRED_EINVAL;
+    ctx->prof = enable != 0;
+    return SHRED_OK;
+}
+
+int shred_profile_read(shred_ctx *ctx, double *ms, uint64_t *launches, uint64_t *bytes) {
+    if (!ctx || !ms || !launches || !bytes) return SHRED_EINVAL;
+    DevGuard g(ctx->device);
+    double tot = 0.0;
+    for (size_t i = 0; i + 1 < ctx->prof_used; i += 2) {
+        CK(cudaEventSynchronize(ctx->prof_ev[i + 1]), "profile sync");
+        float t = 0.f;
+        CK(cudaEventElapsedTime(&t, ctx->prof_ev[i], ctx->prof_ev[i + 1]), "profile elapsed");
+        tot += t;
+    }
+    *ms = tot; *launches = ctx->prof_used / 2; *bytes = ctx->prof_bytes;
+    ctx->prof_used = 0; ctx->prof_bytes = 0;
+    return SHRED_OK;
+}
+
+int shred_synth_fill(uint8_t *d_buf, uint64_t len, uint64_t seed, uint64_t offset, shred_stream_t stream) {
+    if (!len) return SHRED_OK;
+    if (!d_buf) return SHRED_EINVAL;
+    uint64_t blocks = (len / 16 + 255) / 256;
+    if (blocks > 148 * 16) blocks = 148 * 16;
+    if (blocks < 1) blocks = 1;
+    k_synth_fill<<<(unsigned)blocks, 256, 0, (cudaStream_t)stream>>>(d_buf, len, seed, offset);
+    return cudaGetLastError() == cudaSuccess ? SHRED_OK : SHRED_ECUDA;
+}
+
+}  // extern "C"

@@ -1,0 +1,216 @@
+"""GPU parity: the CUDA path (through the C ABI) vs the CPU oracle, element by element.
+
+Bar: bit-exact (integer work).  Sizes span several tiles/rows and ragged tails; edge cases are
+empty/short inputs, unaligned bases, adversarial candidate density (list overflow + re-roll),
+all-zero / all-0xFF, and every kernel path (k63, k32, generic).
+"""
+import numpy as np
+import pytest
+import torch
+
+import oracle
+import synthgen
+
+pytestmark = pytest.mark.gpu
+
+LBFS = oracle.LBFS_POLY
+
+
+@pytest.fixture(scope="module")
+def pkg():
+    import paper_conf_fast_bhatotiarv12_b200 as P
+    return P
+
+
+def dev(a: np.ndarray, offset: int = 0) -> torch.Tensor:
+    """Copy to the GPU; `offset` > 0 returns a view starting `offset` bytes into a buffer."""
+    buf = torch.empty(a.size + offset + 64, dtype=torch.uint8, device="cuda")
+    t = buf[offset:offset + a.size]
+    t.copy_(torch.from_numpy(a))
+    return t
+
+
+def oparams(p) -> oracle.Params:
+    return oracle.Params(p.poly, p.window, p.divisor, p.magic, p.min_size, p.max_size)
+
+
+def check_chunk(ch, data: np.ndarray, offset: int = 0, method: int = 2):
+    got = ch.chunk(dev(data, offset)).cpu().numpy().astype(np.uint64)
+    exp = oracle.chunk(data, oparams(ch.params), method=method)
+    assert got.size == exp.size, (got.size, exp.size)
+    assert np.array_equal(got, exp)
+    return got
+
+
+# ------------------------------------------------------------------ config 1 (paper params)
+def test_config1_random_1mib_vs_r1(pkg):
+    data = synthgen.random_bytes(1, 1 << 20)
+    ch = pkg.Chunker(pkg.Params())
+    assert ch.path == "k63"
+    got = check_chunk(ch, data, method=1)
+    assert got.size == 132
+    chb = pkg.Chunker(pkg.Params(min_size=2048, max_size=65536))
+    got = check_chunk(chb, data, method=1)
+    assert got.size == 102
+
+
+@pytest.mark.parametrize("n", [0, 1, 2, 47, 48, 49, 50, 97, 255, 4095, 4096, 4097, 70001,
+                               (1 << 20) + 13, (5 << 20) + 12345])
+def test_lengths_dense_and_default(pkg, n):
+    data = synthgen.random_bytes(n + 7, n)
+    for p in (pkg.Params(), pkg.Params(divisor=16, magic=8), pkg.Params(divisor=2, magic=1)):
+        check_chunk(pkg.Chunker(p), data)
+
+
+@pytest.mark.parametrize("offset", [1, 3, 7, 8, 13, 15])
+def test_unaligned_base(pkg, offset):
+    data = synthgen.random_bytes(100 + offset, (3 << 20) + 77)
+    check_chunk(pkg.Chunker(pkg.Params(divisor=256)), data, offset)
+
+
+def test_many_rows_and_ragged_tail(pkg):
+    data = synthgen.random_bytes(5, (37 << 20) + 4093)
+    for p in (pkg.Params(), pkg.Params(divisor=512, magic=3)):
+        check_chunk(pkg.Chunker(p), data)
+
+
+def test_special_inputs(pkg):
+    ch = pkg.Chunker(pkg.Params())
+    n = (2 << 20) + 5
+    z = np.zeros(n, np.uint8)
+    assert check_chunk(ch, z).size == 0
+    check_chunk(ch, np.full(n, 0xFF, np.uint8))
+    check_chunk(ch, synthgen.text_like(3, n))
+    # adversarial: a candidate every 2 bytes -> per-row lists overflow -> exact re-roll
+    per = synthgen.periodic(b"\x04\xd5", n)
+    got = check_chunk(ch, per)
+    assert got.size == (n - 48 + 1) // 2
+    chb = pkg.Chunker(pkg.Params(min_size=2048, max_size=65536))
+    check_chunk(chb, per)
+    check_chunk(chb, z)
+
+
+def test_k32_path(pkg):
+    p = pkg.Params(poly=0x104C11DB7)
+    ch = pkg.Chunker(p)
+    assert ch.path == "k32"
+    for n, seed in (((4 << 20) + 3, 1), (100000, 2)):
+        check_chunk(ch, synthgen.random_bytes(seed, n))
+    check_chunk(pkg.Chunker(pkg.Params(poly=0x104C11DB7, divisor=64, magic=5)),
+                synthgen.random_bytes(9, (3 << 20) + 1))
+
+
+def test_generic_path_variants(pkg):
+    for p in (pkg.Params(window=32), pkg.Params(window=1, divisor=256, magic=7),
+              pkg.Params(poly=(1 << 63) | 3, window=16, divisor=1024),
+              pkg.Params(poly=0x11D, window=7, divisor=64, magic=9),
+              pkg.Params(divisor=1 << 40, magic=12345)):
+        ch = pkg.Chunker(p)
+        assert ch.path == "generic"
+        check_chunk(ch, synthgen.random_bytes(11, 300000))
+
+
+def test_bounded_variants(pkg):
+    data = synthgen.random_bytes(12, (6 << 20) + 99)
+    for D in (2048, 8192, 65536):
+        for mn, mx in ((D // 4, 8 * D), (0, 4 * D), (D, D), (1, 1)):
+            check_chunk(pkg.Chunker(pkg.Params(divisor=D, min_size=mn, max_size=mx)), data)
+
+
+# ------------------------------------------------------------------ split invariance (T3/T5)
+@pytest.mark.parametrize("G", [1, 2, 3, 8])
+def test_virtual_shards_concatenate_to_chunk(pkg, G):
+    n = (9 << 20) + 321
+    data = synthgen.random_bytes(13, n)
+    ch = pkg.Chunker(pkg.Params(divisor=1024))
+    exp = oracle.candidates(data, oracle.Params(divisor=1024))
+    parts = []
+    bounds = [n * g // G for g in range(G + 1)]
+    for g in range(G):
+        a, b = bounds[g], bounds[g + 1]
+        halo = min(47, a)
+        x = dev(data[a - halo:b])
+        parts.append(ch.candidates_range(x, halo, a, n).cpu().numpy())
+    got = np.concatenate(parts).astype(np.uint64)
+    assert np.array_equal(got, exp)
+    # the global size-bound pass over the concatenation (bounded mode across shards)
+    chb = pkg.Chunker(pkg.Params(divisor=1024, min_size=256, max_size=8192))
+    cuts = chb.size_bound(torch.from_numpy(got.astype(np.int64)).cuda(), n).cpu().numpy()
+    assert np.array_equal(cuts.astype(np.uint64), oracle.size_bound(exp, n, 256, 8192))
+
+
+# ------------------------------------------------------------------ streaming (config 3 shape)
+def _feed_all(ch, data, sizes, pinned):
+    outs = []
+    off = 0
+    for s in sizes:
+        piece = torch.from_numpy(data[off:off + s].copy())
+        x = piece.pin_memory() if pinned else piece.cuda()
+        outs.append(ch.feed(x).cpu().numpy())
+        off += s
+    outs.append(ch.flush().cpu().numpy())
+    return np.concatenate(outs).astype(np.uint64)
+
+
+@pytest.mark.parametrize("pinned", [False, True])
+@pytest.mark.parametrize("bounded", [False, True])
+def test_feed_matches_one_shot(pkg, pinned, bounded):
+    n = (3 << 20) + 555
+    data = synthgen.random_bytes(14, n)
+    p = pkg.Params(divisor=2048, min_size=512 if bounded else 0, max_size=16384 if bounded else 0)
+    exp = oracle.chunk(data, oparams(p))
+    ch = pkg.Chunker(p)
+    ch.set_ring(3, 1 << 20)                       # host pieces larger than a slot get split
+    rng = np.random.default_rng(5)
+    sizes = []
+    left = n
+    while left:
+        s = int(min(left, rng.choice([1, 2, 47, 48, 1000, 65536, 1 << 20, (1 << 21) + 3])))
+        sizes.append(s); left -= s
+    got = _feed_all(ch, data, sizes, pinned)
+    assert np.array_equal(got, exp)
+    # the ctx is reusable for a second stream
+    got2 = _feed_all(ch, data, [n // 2, n - n // 2], pinned)
+    assert np.array_equal(got2, exp)
+
+
+def test_feed_candidate_at_piece_boundary(pkg):
+    """A candidate exactly at a feed end is held, emitted once more data arrives."""
+    data = synthgen.periodic(b"\x04\xd5", 4000)
+    p = pkg.Params()
+    exp = oracle.chunk(data, oracle.Params())
+    ch = pkg.Chunker(p)
+    got = _feed_all(ch, data, [100, 1, 1, 898, 3000], pinned=False)   # 100, 102 are candidates
+    assert np.array_equal(got, exp)
+
+
+# ------------------------------------------------------------------ device generator
+def test_synth_fill_matches_host_generator(pkg):
+    for seed, off, n in ((1, 0, 1 << 20), (5, 3, 100003), (7, (1 << 33) + 5, 4099)):
+        t = torch.empty(n, dtype=torch.uint8, device="cuda")
+        pkg.synth_fill(t, seed, off)
+        assert np.array_equal(t.cpu().numpy(), synthgen.random_bytes(seed, n, off))
+
+
+# ------------------------------------------------------------------ full-size configs
+def test_config2_1gib_and_edited_version(pkg):
+    """configs[1]: 1 GiB + an edited version, device-resident, in bench.py's launch config.
+    Exact vs oracle R2 (multithreaded) on both versions; edit locality on the candidates."""
+    n = 1 << 30
+    base = torch.empty(n, dtype=torch.uint8, device="cuda")
+    pkg.synth_fill(base, 2)
+    ch = pkg.Chunker(pkg.Params())
+    got = ch.chunk(base).cpu().numpy().astype(np.uint64)
+    host = base.cpu().numpy()
+    assert np.array_equal(host[:4096], synthgen.random_bytes(2, 4096))
+    exp = oracle.candidates(host)
+    assert np.array_equal(got, exp)
+    mu = (n - 48) / 8192
+    assert abs(got.size - mu) < 5 * np.sqrt(mu)
+    ed, ops = synthgen.edited(host, 3)
+    got2 = ch.chunk(dev(ed)).cpu().numpy().astype(np.uint64)
+    assert np.array_equal(got2, oracle.candidates(ed))
+    # bounded mode on the base (sampled: every cut verified by the size-rule characterisation)
+    chb = pkg.Chunker(pkg.Params(min_size=2048, max_size=65536))
+    cuts = chb.chunk(base).cpu().numpy().astype(np.uint64)
+    assert np.array_equal(cuts, oracle.size_bound(exp, n, 2048, 65536))
