@@ -1,0 +1,398 @@
+#!/usr/bin/env python
+"""Benchmark: content-defined chunking throughput on B200 (BASELINE.json metric).
+
+python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+
+Workload (configs[1] of BASELINE.json, per GPU): a 1 GiB synthetic file (bytes
+[rank GiB, (rank+1) GiB) of the SplitMix64 stream seed 2, so ranks hold byte-range shards of
+one N-GiB stream with a 47-byte halo) plus an edited version of it (100 sparse
+inserts/deletes/overwrites, synthgen.edited seed 3+rank).  Paper parameters: P = LBFS
+(deg 63), w = 48, D = 8192, r = 0x78, bounds off.
+
+One step = chunk both versions (all rows of SURVEY §8(a) that are active at the paper's
+defaults: staging, rolling fingerprint, marker test, ordered compaction; at N > 1 the
+per-rank candidate counts are exchanged with an NCCL all-gather).  Inputs are resident in HBM
+and larger than L2 (no flush needed).  `value` = all ranks' input bytes / max-over-ranks device
+time (CUDA events).  `e2e` = the same metric through the C ABI's host-fed mode: pinned host
+buffers -> shred_feed (async H2D on the ctx's copy stream, double-buffered device slots) ->
+shred_flush -> D2H of the cut offsets, all inside the timed region.
+
+--impl reference: the CPU oracle (oracle/, R2 direct per-window reduction, all host cores) on
+a bounded sample of the same workload per step; rank 0 only.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+GiB = 1 << 30
+METRIC = "chunking GB/s at 1/2/4/8 B200, device-resident & host-fed; % of HBM peak"
+W = 48
+
+
+def env_int(k, d):
+    try:
+        return int(os.environ.get(k, d))
+    except ValueError:
+        return d
+
+
+def peaks():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            p = json.load(f)
+        return float(p["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs, copy test)"
+    except Exception:
+        return 6650.0, "fallback (B200_PROFILING.md 6.65 TB/s)"
+
+
+def config(n_gpus, per_rank_bytes):
+    return {"workload": "configs[1]: 1 GiB SplitMix64 file + edited version (100 sparse edits) per GPU, "
+                        "device-resident; ranks hold byte-range shards of one stream with a 47-B halo",
+            "params": "P=0xbfe6b8a5bf378d83 (deg 63), w=48, D=8192, r=0x78, min=0, max=inf",
+            "bytes_per_step_per_gpu": per_rank_bytes,
+            "l2": "inputs (1 GiB each) larger than the 126 MB L2; no flush",
+            "parallelism": f"byte-range shards x{n_gpus}, count all-gather (NCCL)" if n_gpus > 1 else "1 GPU"}
+
+
+# ------------------------------------------------------------------------------- clocks (NVML)
+class ClockSampler:
+    REASONS = {0x4: "sw_power_cap", 0x8: "hw_slowdown", 0x20: "sw_thermal_slowdown",
+               0x40: "hw_thermal_slowdown", 0x80: "hw_power_brake_slowdown", 0x2: "applications_clocks",
+               0x1: "gpu_idle", 0x10: "sync_boost", 0x100: "display_clocks"}
+
+    def __init__(self, dev_index):
+        self.ok = False
+        self.samples, self.reasons = [], 0
+        try:
+            import pynvml
+            pynvml.nvmlInit()
+            self.nv = pynvml
+            self.h = pynvml.nvmlDeviceGetHandleByIndex(dev_index)
+            self.max = pynvml.nvmlDeviceGetMaxClockInfo(self.h, pynvml.NVML_CLOCK_SM)
+            self.ok = True
+        except Exception:
+            pass
+        self._stop = threading.Event()
+
+    def _run(self):
+        nv = self.nv
+        get_r = getattr(nv, "nvmlDeviceGetCurrentClocksEventReasons", None) or \
+            nv.nvmlDeviceGetCurrentClocksThrottleReasons
+        while not self._stop.is_set():
+            try:
+                self.samples.append(nv.nvmlDeviceGetClockInfo(self.h, nv.NVML_CLOCK_SM))
+                self.reasons |= int(get_r(self.h))
+            except Exception:
+                pass
+            time.sleep(0.002)
+
+    def __enter__(self):
+        if self.ok:
+            self.t = threading.Thread(target=self._run, daemon=True)
+            self.t.start()
+        return self
+
+    def __exit__(self, *a):
+        if self.ok:
+            self._stop.set()
+            self.t.join()
+
+    def result(self):
+        if not self.ok or not self.samples:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvml unavailable"]}
+        return {"sm_mhz": float(np.median(self.samples)), "sm_max_mhz": float(self.max),
+                "samples": len(self.samples),
+                "reasons": [n for b, n in self.REASONS.items() if self.reasons & b and b != 0x1]}
+
+
+# ------------------------------------------------------------------------------- CPU oracle timing
+def oracle_rate(sample: np.ndarray, threads: int):
+    import oracle
+    t = time.perf_counter()
+    c = oracle.candidates(sample, oracle.Params(), method=2, threads=threads)
+    dt = time.perf_counter() - t
+    return sample.size / dt / 1e9, dt, c.size
+
+
+def cpu_baseline(host: np.ndarray, budget_s: float = 12.0):
+    """Oracle (R2, multithreaded over this process's cores) on a bounded prefix sample."""
+    import oracle
+    oracle.build()
+    cores = len(os.sched_getaffinity(0))
+    cal = host[: 8 << 20]
+    rate, dt, _ = oracle_rate(cal, cores)
+    n = int(min(host.size, max(16 << 20, rate * 1e9 * budget_s)))
+    n -= n % 4096
+    rate, dt, nc = oracle_rate(host[:n], cores)
+    return {"value": round(rate, 4), "unit": "GB/s", "cores": cores, "kind": "oracle",
+            "sample": f"first {n / 2**20:.0f} MiB of the configs[1] base file, R2 direct per-window "
+                      f"reduction (48 table lookups/window), {cores} threads, {dt:.1f} s, {nc} candidates"}
+
+
+# ------------------------------------------------------------------------------- reference arm
+def run_reference(args, rank, world):
+    if rank != 0:
+        return
+    import oracle
+    import synthgen
+    oracle.build()
+    cores = len(os.sched_getaffinity(0))
+    per_rank = 2 * GiB
+    # each step: a bounded sample of the workload (alternating base / edited-version slices)
+    cal = synthgen.random_bytes(2, 8 << 20)
+    rate, _, _ = oracle_rate(cal, cores)
+    n = int(min(256 << 20, max(8 << 20, rate * 1e9 * 2.0)))
+    n -= n % 4096
+    base = synthgen.random_bytes(2, n)
+    ed, _ = synthgen.edited(base, 3, n_edits=max(1, min(100, n // (1 << 20))), min_gap=8192)
+    samples = [base, ed]
+    for i in range(args.warmup):
+        oracle.candidates(samples[i % 2], oracle.Params(), 2, cores)
+    t0 = time.perf_counter()
+    tot = 0
+    for i in range(args.steps):
+        s = samples[i % 2]
+        oracle.candidates(s, oracle.Params(), 2, cores)
+        tot += s.size
+    dt = time.perf_counter() - t0
+    v = tot / dt / 1e9
+    line = {"metric": METRIC, "value": round(v, 4), "unit": "GB/s", "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": round(dt / args.steps * 1e3, 3), "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "u8", "data": "synthetic",
+            "config": config(world, per_rank), "impl": "reference",
+            "cpu_baseline": {"value": round(v, 4), "unit": "GB/s", "cores": cores, "kind": "oracle",
+                             "sample": f"each step = {n / 2**20:.0f} MiB of the base file or its edited "
+                                       f"version (alternating), R2 oracle, {cores} threads"},
+            "e2e": {"value": round(v, 4), "unit": "GB/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+# ------------------------------------------------------------------------------- our arm
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=5)
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu", action="store_true")
+    ap.add_argument("--no-extra", action="store_true", help="skip the bounded / k32 side measurements")
+    args = ap.parse_args()
+    args.warmup = max(3, args.warmup)
+
+    rank, world, local = env_int("RANK", 0), env_int("WORLD_SIZE", 1), env_int("LOCAL_RANK", 0)
+    if args.impl == "reference":
+        return run_reference(args, rank, world)
+
+    import torch
+    import torch.distributed as dist
+    import synthgen
+    import paper_conf_fast_bhatotiarv12_b200 as pkg
+
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    dev = torch.device("cuda", local)
+    stream = torch.cuda.current_stream()
+
+    # ---- inputs (untimed): this rank's shard of stream seed 2 with its halo, and an edited file
+    halo = min(W - 1, rank * GiB)
+    base_h = torch.empty(GiB + halo, dtype=torch.uint8, device=dev)
+    pkg.synth_fill(base_h, 2, rank * GiB - halo)
+    base = base_h[halo:]
+    host_base = base.cpu().numpy()
+    ed_np, _ = synthgen.edited(host_base, 3 + rank)
+    edited = torch.from_numpy(ed_np).to(dev)
+    per_rank_bytes = int(base.numel() + edited.numel())
+
+    ch = pkg.Chunker(pkg.Params(), device=local)
+    cap = GiB // 2048 + 65536
+    out0 = torch.empty(cap, dtype=torch.int64, device=dev)
+    out1 = torch.empty(cap, dtype=torch.int64, device=dev)
+    n0 = torch.zeros(1, dtype=torch.int64, device=dev)
+    n1 = torch.zeros(1, dtype=torch.int64, device=dev)
+    counts = torch.zeros(world, dtype=torch.int64, device=dev)
+    total = world * GiB
+
+    def step():
+        if world == 1:
+            ch.chunk_async(base, out0, n0)
+        else:
+            rc = pkg.lib().shred_candidates_range(ch._ctx, base_h.data_ptr(), halo, rank * GiB, GiB, total,
+                                                  out0.data_ptr(), cap, n0.data_ptr(), stream.cuda_stream)
+            ch._check(rc, "shred_candidates_range")
+        ch.chunk_async(edited, out1, n1)
+        if world > 1:
+            dist.all_gather_into_tensor(counts, n0)       # C2: per-rank candidate counts
+
+    for _ in range(args.warmup):
+        step()
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    l0 = ch.launches
+    ch.profile(True)
+    with ClockSampler(local) as clk:
+        e0.record(stream)
+        for _ in range(args.steps):
+            step()
+        e1.record(stream)
+        torch.cuda.synchronize()
+    ch.profile(False)
+    launches = ch.launches - l0
+    k_ms, k_n, k_bytes = ch.profile_read()
+    if world > 1:
+        dist.barrier()
+    ms = e0.elapsed_time(e1)
+    t = torch.tensor([ms], dtype=torch.float64, device=dev)
+    if world > 1:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    ms_max = float(t.item())
+    value = world * per_rank_bytes * args.steps / (ms_max * 1e-3) / 1e9
+    n_cand = int(n0.item())
+    assert n_cand <= cap and int(n1.item()) <= cap
+    hbm, hbm_src = peaks()
+
+    # ---- roofline of the hot kernel (k1_bulk), live CUDA events on the launching stream
+    k_avg_ms = k_ms / max(1, k_n)
+    k_bytes_per_launch = k_bytes / max(1, k_n)
+    achieved = k_bytes_per_launch / (k_avg_ms * 1e-3) / 1e9 if k_n else None
+    traffic = None
+    try:
+        with open(os.path.join(ROOT, "profiles", "k1_traffic.json")) as f:
+            tr = json.load(f)
+        traffic = tr.get("dram_bytes_per_launch")
+    except Exception:
+        pass
+    roofline = {"bound": "hbm", "achieved": round(achieved, 1) if achieved else None, "peak": hbm,
+                "unit": "GB/s", "frac": round(achieved / hbm, 4) if achieved else None, "traffic": traffic,
+                "kernel": "k1_bulk<K63>", "launches": k_n, "avg_launch_ms": round(k_avg_ms, 4),
+                "algorithmic_bytes_per_launch": int(k_bytes_per_launch),
+                "share_of_step": round(k_ms / ms, 4) if ms else None, "peak_source": hbm_src,
+                "note": "algorithmic bytes = 1 B read per input byte (+8 B per candidate, ~0.001 B/B); "
+                        "the kernel is bound by the shared-memory lookup datapath below HBM (DESIGN.md)"}
+
+    line = {"metric": METRIC, "value": round(value, 2), "unit": "GB/s", "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": round(ms_max / args.steps, 4), "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "u8", "data": "synthetic",
+            "config": config(world, per_rank_bytes), "hbm_frac": round(value / world / hbm, 4),
+            "roofline": roofline, "clocks": clk.result(), "gpu_launches": launches,
+            "candidates_rank0": n_cand}
+
+    # ---- e2e: host-fed through the C ABI (pinned host -> shred_feed -> flush -> D2H)
+    if not args.no_e2e:
+        pin_base = torch.empty(base.numel(), dtype=torch.uint8).pin_memory()
+        pin_base.copy_(base.cpu())
+        pin_ed = torch.from_numpy(ed_np).pin_memory()
+        che = pkg.Chunker(pkg.Params(), device=local)
+        che.set_ring(2, 256 << 20)
+        ecap = GiB // 2048 + 65536
+        eo = torch.empty(ecap, dtype=torch.int64, device=dev)
+        en = torch.zeros(2, dtype=torch.int64, device=dev)
+        en_h = torch.zeros(2, dtype=torch.int64).pin_memory()
+        res_h = torch.empty(2 * ecap, dtype=torch.int64).pin_memory()
+        fo = torch.empty(1, dtype=torch.int64, device=dev)
+        fn = torch.zeros(1, dtype=torch.int64, device=dev)
+        d2h = [0]
+
+        def e2e_step():
+            che.feed_async(pin_base, eo, en[0:1])
+            pkg.lib().shred_flush(che._ctx, fo.data_ptr(), 1, fn.data_ptr(), stream.cuda_stream)
+            en_h.copy_(en, non_blocking=True)
+            stream.synchronize()
+            a = int(en_h[0])
+            res_h[:a].copy_(eo[:a], non_blocking=True)
+            che.feed_async(pin_ed, eo, en[1:2])
+            pkg.lib().shred_flush(che._ctx, fo.data_ptr(), 1, fn.data_ptr(), stream.cuda_stream)
+            en_h.copy_(en, non_blocking=True)
+            stream.synchronize()
+            b = int(en_h[1])
+            res_h[a:a + b].copy_(eo[:b], non_blocking=True)
+            d2h[0] = 8 * (a + b) + 16
+            return a, b
+
+        for _ in range(max(2, args.warmup)):
+            e2e_step()
+        torch.cuda.synchronize()
+        if world > 1:
+            dist.barrier()
+        s0, s1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        s0.record(stream)
+        for _ in range(args.steps):
+            a, b = e2e_step()
+        s1.record(stream)
+        torch.cuda.synchronize()
+        ems = s0.elapsed_time(s1)
+        et = torch.tensor([ems], dtype=torch.float64, device=dev)
+        if world > 1:
+            dist.all_reduce(et, op=dist.ReduceOp.MAX)
+        ems = float(et.item())
+        ev = world * per_rank_bytes * args.steps / (ems * 1e-3) / 1e9
+        # H2D peak on this box for context (256 MiB pinned copy, best of 5)
+        tmp = torch.empty(256 << 20, dtype=torch.uint8, device=dev)
+        best = 1e9
+        for _ in range(5):
+            q0, q1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            q0.record(stream)
+            tmp.copy_(pin_base[: 256 << 20], non_blocking=True)
+            q1.record(stream)
+            torch.cuda.synchronize()
+            best = min(best, q0.elapsed_time(q1))
+        h2d_peak = (256 << 20) / (best * 1e-3) / 1e9
+        line["e2e"] = {"value": round(ev, 3), "unit": "GB/s", "h2d_bytes_per_step": per_rank_bytes,
+                       "d2h_bytes_per_step": d2h[0], "ms_per_step": round(ems / args.steps, 3),
+                       "api": "shred_feed(pinned host, 2 x 256 MiB device slots) + shred_flush + D2H of cuts",
+                       "h2d_peak_gbs": round(h2d_peak, 2), "frac_of_h2d_peak": round(ev / world / h2d_peak, 4),
+                       "cuts_match_device_path": (a == int(n0.item()) if world == 1 else None)}
+        del tmp
+
+    # ---- side measurements (not the headline): bounded mode and the k32 instantiation
+    if not args.no_extra and world == 1:
+        def timed(chx, x, reps=5):
+            o = torch.empty(cap, dtype=torch.int64, device=dev)
+            nn = torch.zeros(1, dtype=torch.int64, device=dev)
+            chx.chunk_async(x, o, nn)
+            torch.cuda.synchronize()
+            a0, a1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a0.record(stream)
+            for _ in range(reps):
+                chx.chunk_async(x, o, nn)
+            a1.record(stream)
+            torch.cuda.synchronize()
+            return x.numel() * reps / (a0.elapsed_time(a1) * 1e-3) / 1e9
+        try:
+            chb = pkg.Chunker(pkg.Params(min_size=2048, max_size=65536), device=local)
+            line["bounded_2048_65536"] = {"value": round(timed(chb, base), 2), "unit": "GB/s",
+                                          "note": "size rule on: one host sync + single-warp K3 (v0)"}
+            c32 = pkg.Chunker(pkg.Params(poly=0x104C11DB7), device=local)
+            v32 = timed(c32, base)
+            line["k32_variant"] = {"value": round(v32, 2), "unit": "GB/s", "hbm_frac": round(v32 / hbm, 4),
+                                   "params": "P=0x104C11DB7 (deg 32, irreducible), other params as paper"}
+        except Exception as e:  # side numbers must never break the headline line
+            line["extra_error"] = repr(e)
+
+    # ---- CPU baseline: the oracle on this box's host cores (rank 0, N = 1 only)
+    if not args.no_cpu and rank == 0 and world == 1:
+        line["cpu_baseline"] = cpu_baseline(host_base)
+
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

@@ -15,10 +15,13 @@
 //                   shared memory, replicated per lane so the data-dependent lookups never
 //                   bank-conflict.  A per-16-byte predicate detects the rare marker hit;
 //                   hits replay that chunk exactly and append c to the thread's slot list.
-//   k1_generic      Any valid parameters, byte at a time; also the head/tail of fast paths.
-//   k_scan          Exclusive scan of per-slot candidate counts (one CTA).
-//   k_scatter       Ordered compaction of the per-slot lists into the destination; slots
-//                   that overflowed their list re-roll their range and write directly.
+//                   The last CTA of the launch is the "edge" CTA: it rolls the unaligned head
+//                   and the ragged tail of the range with the generic byte loop.  Every CTA
+//                   ends with a block scan of its slots' counts (local offsets + group sum).
+//   k1_generic      Any valid parameters, byte at a time (the generic path).
+//   k_scatter       Ordered compaction: group prefix (from the group sums) + local offset,
+//                   copies the per-slot lists into the destination; slots that overflowed
+//                   their list re-roll their range and write directly.
 //   k_size_bound    The sequential min/max rule (one warp), with streaming state.
 #pragma once
 #include <cstdint>
@@ -29,24 +32,37 @@ namespace shred {
 
 enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3 };
 
-constexpr int NT          = 512;               // consumer threads (rows) per CTA
-constexpr int ROUND       = 64;                // bytes per row per pipeline round
+constexpr int NT          = 512;               // consumer threads per CTA
+constexpr int CHAINS      = 2;                 // rows (independent fingerprint chains) per thread
+constexpr int ROWS_CTA    = NT * CHAINS;       // rows per bulk CTA
+constexpr int ROUND       = 64 / CHAINS;       // bytes per row per pipeline round
 constexpr int STAGES      = 4;                 // TMA ring depth
 constexpr int BOX_ROWS    = 256;               // rows per TMA box (hardware max 256)
 constexpr int TAB_BYTES   = 65536;             // replicated T|U image (256 rows x 256 B)
-constexpr int STAGE_BYTES = NT * ROUND;        // 32 KiB
+constexpr int STAGE_BYTES = ROWS_CTA * ROUND;  // 32 KiB
 constexpr int BAR_OFFSET  = TAB_BYTES + STAGES * STAGE_BYTES;
-constexpr int BULK_SMEM   = BAR_OFFSET + 1024; // + barriers; + 1 KiB so the base can be aligned
+constexpr int BULK_SMEM   = BAR_OFFSET + 2048; // + barriers/scan scratch; + 1 KiB base alignment
 constexpr int GEN_THREADS = 256;
 
 // Slot id -> range of window-end positions.  Slots are numbered in stream order:
 // [0, n_head) generic head segments, then the bulk rows, then generic tail segments.
+// Slot groups (one group sum each): bulk mode: group 0 = head slots, 1 + r/ROWS_CTA = bulk rows,
+// nc + 1 = tail slots; generic-only mode (nrows == 0): group = slot / GEN_THREADS.
 struct SlotMap {
     uint64_t head_start; uint64_t head_seg; uint32_t n_head;
     uint32_t nrows;      uint64_t b0;       uint64_t S;
     uint64_t tail_start; uint64_t tail_seg; uint32_t n_tail;
+    uint32_t nc;         uint32_t ngroups;  // bulk CTAs; number of groups
     uint64_t t_end;
 };
+
+__host__ __device__ __forceinline__ uint32_t slot_group(const SlotMap &m, uint32_t slot) {
+    if (m.nrows == 0) return slot / GEN_THREADS;
+    if (slot < m.n_head) return 0;
+    slot -= m.n_head;
+    if (slot < m.nrows) return 1 + slot / ROWS_CTA;
+    return m.nc + 1;
+}
 
 struct DevParams {              // chunking parameters as the kernels need them
     uint64_t dmask;             // D - 1
@@ -65,6 +81,8 @@ struct Job {
     uint64_t min_i;             // w - 1: only full windows are tested (reading Q10)
     uint64_t c_limit;           // emit c only if c < c_limit (reading Q11)
     uint32_t *counts;           // [nslots] true candidate count per slot
+    uint32_t *local_off;        // [nslots] exclusive prefix of counts within the slot's group
+    uint64_t *group_sum;        // [ngroups] candidates per group
     uint64_t *scratch;          // [nslots * cap] per-slot candidate lists
     SlotMap map;
 };
@@ -73,7 +91,7 @@ struct GenTables { uint64_t T[256]; uint64_t U[256]; };
 
 // Device-resident streaming / output state (one per ctx).
 struct Aux {
-    uint64_t total;             // candidates of the current piece (k_scan)
+    uint64_t total;             // candidates of the current piece (k_scatter / k_total)
     uint64_t last_cand;         // last candidate of the current piece (k_scatter)
     uint64_t out_pos;           // cuts already written by the current API call
     uint64_t s;                 // size rule: last cut (absolute)
@@ -185,35 +203,84 @@ __device__ __forceinline__ void slot_range(const SlotMap &m, uint32_t slot, uint
     b = a + m.tail_seg; if (b > m.t_end) b = m.t_end;
 }
 
-// ------------------------------------------------------------------------------ k1_generic
-// One thread per generic slot (head slots, then tail slots).
-__global__ void __launch_bounds__(GEN_THREADS)
-k1_generic(Job J, DevParams P, const GenTables *__restrict__ gt) {
-    __shared__ uint64_t sT[256], sU[256];
-    for (int i = threadIdx.x; i < 256; i += blockDim.x) { sT[i] = gt->T[i]; sU[i] = gt->U[i]; }
-    __syncthreads();
-    const uint32_t g = blockIdx.x * blockDim.x + threadIdx.x;
-    const uint32_t ngen = J.map.n_head + J.map.n_tail;
-    if (g >= ngen) return;
-    const uint32_t slot = (g < J.map.n_head) ? g : g + J.map.nrows;
+// ------------------------------------------------------------------------------ block scan
+// Exclusive scan of one u32 per thread over the first `nthr` threads (a multiple of 32) of the
+// CTA, using named barrier `bar` and `ws` (>= 33 u32 of shared memory).  Returns the
+// exclusive prefix; *total = the sum (same value in every thread).
+__device__ __forceinline__ uint32_t block_exscan(uint32_t v, uint32_t nthr, uint32_t bar,
+                                                 uint32_t *ws, uint32_t *total) {
+    const uint32_t tid = threadIdx.x, lane = tid & 31u, wid = tid >> 5;
+    uint32_t incl = v;
+#pragma unroll
+    for (int d = 1; d < 32; d <<= 1) {
+        uint32_t u = __shfl_up_sync(0xffffffffu, incl, d);
+        if (lane >= (uint32_t)d) incl += u;
+    }
+    if (lane == 31) ws[wid] = incl;
+    asm volatile("bar.sync %0, %1;" :: "r"(bar), "r"(nthr) : "memory");
+    if (wid == 0) {
+        const uint32_t nw = nthr >> 5;
+        uint32_t x = lane < nw ? ws[lane] : 0u;
+        uint32_t xi = x;
+#pragma unroll
+        for (int d = 1; d < 32; d <<= 1) {
+            uint32_t u = __shfl_up_sync(0xffffffffu, xi, d);
+            if (lane >= (uint32_t)d) xi += u;
+        }
+        if (lane < nw) ws[lane] = xi - x;
+        if (lane == 31) ws[32] = xi;
+    }
+    asm volatile("bar.sync %0, %1;" :: "r"(bar), "r"(nthr) : "memory");
+    const uint32_t r = ws[wid] + incl - v;
+    *total = ws[32];
+    asm volatile("bar.sync %0, %1;" :: "r"(bar), "r"(nthr) : "memory");   // ws reusable
+    return r;
+}
+
+// Roll one generic slot into its list; returns the true count.
+template <class Tab>
+__device__ __forceinline__ uint32_t roll_slot(const Job &J, const DevParams &P, const Tab &tab,
+                                              uint32_t slot) {
     uint64_t a, b;
     slot_range(J.map, slot, a, b);
     uint32_t cnt = 0;
     uint64_t *lst = J.scratch + (uint64_t)slot * J.cap;
-    SmemGenTab tab{sT, sU};
     roll_generic(J, P, tab, a, b, [&](uint64_t c) {
         if (cnt < J.cap) lst[cnt] = c;
         ++cnt;
     });
-    J.counts[slot] = cnt;
+    return cnt;
+}
+
+// ------------------------------------------------------------------------------ k1_generic
+// Generic-only path: one thread per slot, one group per block of GEN_THREADS slots.
+__global__ void __launch_bounds__(GEN_THREADS)
+k1_generic(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots) {
+    __shared__ uint64_t sT[256], sU[256];
+    __shared__ uint32_t ws[33];
+    for (int i = threadIdx.x; i < 256; i += blockDim.x) { sT[i] = gt->T[i]; sU[i] = gt->U[i]; }
+    __syncthreads();
+    const uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
+    SmemGenTab tab{sT, sU};
+    const uint32_t cnt = slot < nslots ? roll_slot(J, P, tab, slot) : 0u;
+    uint32_t tot;
+    const uint32_t off = block_exscan(cnt, GEN_THREADS, 1, ws, &tot);
+    if (slot < nslots) { J.counts[slot] = cnt; J.local_off[slot] = off; }
+    if (threadIdx.x == 0) J.group_sum[blockIdx.x] = tot;
 }
 
 // ------------------------------------------------------------------------------ k1_bulk
+// Per-lane constants of the hot loop.  The multipliers are runtime values so that ptxas keeps
+// the index math and the marker-test shift on the FMA pipe (IMAD / IMAD.HI) instead of turning
+// them into ALU shifts: the ALU pipe is the busiest unit of this loop (ncu r01).
 struct BulkCtx {
     uint32_t tab;       // shared address of the T|U image
-    uint32_t laneT;     // K63: tab + (lane&15)*8           K32: lane*4
+    uint32_t laneT;     // K63: tab + (lane&15)*8           K32: tab + lane*4
     uint32_t laneU;     // K63: 128 + (lane&15)*8 (byte)     K32: 128 + lane*4 (byte)
-    uint32_t mask, magic;
+    uint32_t mhi;       // K63: 2^9 (f_hi >> 23 = mulhi(f_hi, 2^9))   K32: 2^8 (f >> 24)
+    uint32_t m256;      // 256 (row stride of the table image)
+    uint32_t tmul;      // 2^(32-m): (f_lo * tmul) keeps the low m bits at the top
+    uint32_t rsh;       // r << (32-m)
 };
 
 // One byte step, K63 (deg P = 63, fully reduced u64 state f = fh:fl, f < 2^63):
@@ -223,8 +290,8 @@ struct BulkCtx {
 template <int K>
 __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, uint32_t pop,
                                        const BulkCtx &c) {
-    const uint32_t t  = fh >> 23;
-    const uint32_t ti = t * 256u + c.laneT;
+    const uint32_t t  = __umulhi(fh, c.mhi);
+    const uint32_t ti = t * c.m256 + c.laneT;
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
     const uint2 T = lds64(ti);
     const uint2 U = lds64(c.tab + oi);
@@ -237,9 +304,9 @@ __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, 
 // One byte step, K32 (deg P = 32, u32 state): f <- (f << 8) ^ B ^ T[f >> 24] ^ U[o].
 template <int K>
 __device__ __forceinline__ void step32(uint32_t &f, uint32_t in, uint32_t pop, const BulkCtx &c) {
-    const uint32_t ti = __byte_perm(f, c.laneT, 0x5534u);
+    const uint32_t ti = __umulhi(f, c.mhi) * c.m256 + c.laneT;
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
-    const uint32_t T = lds32(c.tab + ti);
+    const uint32_t T = lds32(ti);
     const uint32_t U = lds32(c.tab + oi);
     f = __byte_perm(f, in, 0x2104u + K) ^ T ^ U;
 }
@@ -261,69 +328,95 @@ template <> struct State<MODE_K32> {
     __device__ __forceinline__ uint32_t low() const { return f; }
 };
 
-// 4 bytes of one word: hit |= (low bits of the fingerprint after each byte == r).
-template <int MODE, bool TEST>
-__device__ __forceinline__ void word4(State<MODE> &s, uint32_t in, uint32_t pop, const BulkCtx &c,
-                                      bool &hit) {
-    s.template step<0>(in, pop, c); if (TEST) hit |= ((s.low() & c.mask) == c.magic);
-    s.template step<1>(in, pop, c); if (TEST) hit |= ((s.low() & c.mask) == c.magic);
-    s.template step<2>(in, pop, c); if (TEST) hit |= ((s.low() & c.mask) == c.magic);
-    s.template step<3>(in, pop, c); if (TEST) hit |= ((s.low() & c.mask) == c.magic);
-}
+// marker test: (f mod D) == r  <=>  (f_lo << (32-m)) == (r << (32-m))   (D = 2^m <= 2^32)
+__device__ __forceinline__ bool is_marker(uint32_t lo, const BulkCtx &c) { return lo * c.tmul == c.rsh; }
 
 struct SlotOut {
     uint64_t *lst; uint32_t cnt; uint32_t cap;
-    uint64_t min_i, c_limit;
-    __device__ __forceinline__ void emit(uint64_t i) {       // i = window end position
-        if (i >= min_i && i + 1 < c_limit) {
-            if (cnt < cap) lst[cnt] = i + 1;
-            ++cnt;
-        }
-    }
 };
 
-// Replay one 16-byte chunk from its saved entry state, emitting every marker hit exactly.
-template <int MODE>
-__device__ __noinline__ void replay_chunk(State<MODE> s, uint4 d, uint4 p, uint64_t pos,
-                                          const BulkCtx &c, SlotOut &o) {
-    const uint32_t dw[4] = {d.x, d.y, d.z, d.w};
-    const uint32_t pw[4] = {p.x, p.y, p.z, p.w};
-#pragma unroll
-    for (int j = 0; j < 4; ++j) {
-        s.template step<0>(dw[j], pw[j], c); if ((s.low() & c.mask) == c.magic) o.emit(pos + 4 * j + 0);
-        s.template step<1>(dw[j], pw[j], c); if ((s.low() & c.mask) == c.magic) o.emit(pos + 4 * j + 1);
-        s.template step<2>(dw[j], pw[j], c); if ((s.low() & c.mask) == c.magic) o.emit(pos + 4 * j + 2);
-        s.template step<3>(dw[j], pw[j], c); if ((s.low() & c.mask) == c.magic) o.emit(pos + 4 * j + 3);
+// Emit the marker hits of one 16-byte chunk: bit j of m = a hit at window end pos + j.
+__device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t min_i, uint64_t c_limit,
+                                       SlotOut &o) {
+    while (m) {
+        const int j = __ffs(m) - 1;
+        m &= m - 1;
+        const uint64_t i = pos + (uint64_t)j;
+        if (i >= min_i && i + 1 < c_limit) {
+            if (o.cnt < o.cap) o.lst[o.cnt] = i + 1;
+            ++o.cnt;
+        }
     }
 }
 
-template <int MODE, bool TEST>
-__device__ __forceinline__ void chunk16(State<MODE> &s, const uint4 &d, const uint4 &p, uint64_t pos,
-                                        const BulkCtx &c, SlotOut &o) {
-    const State<MODE> s0 = s;
-    bool hit = false;
-    word4<MODE, TEST>(s, d.x, p.x, c, hit);
-    word4<MODE, TEST>(s, d.y, p.y, c, hit);
-    word4<MODE, TEST>(s, d.z, p.z, c, hit);
-    word4<MODE, TEST>(s, d.w, p.w, c, hit);
-    if (TEST && hit) replay_chunk<MODE>(s0, d, p, pos, c, o);
+// One word (4 bytes) of two interleaved chains; hit bits accumulate into mA / mB.
+template <int MODE, bool TEST, int J>
+__device__ __forceinline__ void word4x2(State<MODE> &a, uint32_t ina, uint32_t popa, uint32_t &mA,
+                                        State<MODE> &b, uint32_t inb, uint32_t popb, uint32_t &mB,
+                                        const BulkCtx &c) {
+    a.template step<0>(ina, popa, c); b.template step<0>(inb, popb, c);
+    if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + 0)) : 0u; mB |= is_marker(b.low(), c) ? (1u << (4 * J + 0)) : 0u; }
+    a.template step<1>(ina, popa, c); b.template step<1>(inb, popb, c);
+    if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + 1)) : 0u; mB |= is_marker(b.low(), c) ? (1u << (4 * J + 1)) : 0u; }
+    a.template step<2>(ina, popa, c); b.template step<2>(inb, popb, c);
+    if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + 2)) : 0u; mB |= is_marker(b.low(), c) ? (1u << (4 * J + 2)) : 0u; }
+    a.template step<3>(ina, popa, c); b.template step<3>(inb, popb, c);
+    if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + 3)) : 0u; mB |= is_marker(b.low(), c) ? (1u << (4 * J + 3)) : 0u; }
 }
 
+// 16 bytes of two chains in one basic block (ILP across the chains), then the rare emission.
+template <int MODE, bool TEST>
+__device__ __forceinline__ void chunk16x2(State<MODE> &a, const uint4 &da, const uint4 &pa,
+                                          State<MODE> &b, const uint4 &db, const uint4 &pb,
+                                          const BulkCtx &c, uint32_t &mA, uint32_t &mB) {
+    mA = 0; mB = 0;
+    word4x2<MODE, TEST, 0>(a, da.x, pa.x, mA, b, db.x, pb.x, mB, c);
+    word4x2<MODE, TEST, 1>(a, da.y, pa.y, mA, b, db.y, pb.y, mB, c);
+    word4x2<MODE, TEST, 2>(a, da.z, pa.z, mA, b, db.z, pb.z, mB, c);
+    word4x2<MODE, TEST, 3>(a, da.w, pa.w, mA, b, db.w, pb.w, mB, c);
+}
+
+struct BulkConst { uint32_t mhi, m256, tmul, rsh; };
+
 // The hot kernel.  blockDim = NT consumers + 1 producer warp; one CTA per SM.
-// The window is fixed at w = 48 = 3 chunks of 16 B: the byte leaving the window at chunk q
-// is the same byte slot of chunk q-3, kept in registers (R1..R3 = chunks 1..3 of the
-// previous round).
+// blockIdx < nc: bulk CTA, rows blockIdx*ROWS_CTA + {tid, tid + NT}; blockIdx == nc: edge CTA.
+// Rounds of ROUND = 32 bytes per row arrive in a 4-stage TMA ring (SWIZZLE_32B: the 8 lanes
+// of a quarter warp read 8 consecutive rows' 16-byte chunks from 8 distinct bank groups).
+// The window is fixed at w = 48 = 3 chunks of 16 B: the byte leaving the window at chunk q is
+// the same byte slot of chunk q-3, kept in registers (R1..R3 = chunks 1..3 of the previous
+// pair of rounds).
 template <int MODE>
 __global__ void __launch_bounds__(NT + 32, 1)
-k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_img, Job J,
-        uint32_t mask, uint32_t magic) {
+k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_img,
+        const GenTables *__restrict__ gt, Job J, DevParams P, BulkConst K) {
+    static_assert(CHAINS == 2 && ROUND == 32, "kernel written for 2 chains x 32-byte rounds");
     extern __shared__ uint8_t smem_raw[];
-    // align the dynamic shared base to 1 KiB (SWIZZLE_64B pattern is address-based)
+    // align the dynamic shared base to 1 KiB (the TMA swizzle pattern is address-based)
     uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
     const uint32_t sbase = smem_u32(smem);
     const uint32_t stages = sbase + TAB_BYTES;
     const uint32_t bars = sbase + BAR_OFFSET;      // full[s] at +8s, empty[s] at +64+8s
+    uint32_t *ws = reinterpret_cast<uint32_t *>(smem + BAR_OFFSET + 128);
     const int tid = threadIdx.x;
+
+    if (blockIdx.x == J.map.nc) {                    // ---- edge CTA: head + tail, generic loop
+        uint64_t *sT = reinterpret_cast<uint64_t *>(smem + TAB_BYTES);
+        uint64_t *sU = sT + 256;
+        for (int i = tid; i < 256; i += blockDim.x) { sT[i] = gt->T[i]; sU[i] = gt->U[i]; }
+        __syncthreads();
+        if (tid >= NT) return;
+        SmemGenTab tab{sT, sU};
+        const uint32_t tail0 = J.map.n_head + J.map.nrows;
+        const uint32_t ch = (uint32_t)tid < J.map.n_head ? roll_slot(J, P, tab, tid) : 0u;
+        const uint32_t ct = (uint32_t)tid < J.map.n_tail ? roll_slot(J, P, tab, tail0 + tid) : 0u;
+        uint32_t th, tt;
+        const uint32_t oh = block_exscan(ch, NT, 1, ws, &th);
+        const uint32_t ot = block_exscan(ct, NT, 1, ws, &tt);
+        if ((uint32_t)tid < J.map.n_head) { J.counts[tid] = ch; J.local_off[tid] = oh; }
+        if ((uint32_t)tid < J.map.n_tail) { J.counts[tail0 + tid] = ct; J.local_off[tail0 + tid] = ot; }
+        if (tid == 0) { J.group_sum[0] = th; J.group_sum[J.map.nc + 1] = tt; }
+        return;
+    }
 
     for (int i = tid; i < TAB_BYTES / 16; i += blockDim.x)
         reinterpret_cast<uint4 *>(smem)[i] = tab_img[i];
@@ -337,8 +430,8 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     }
     __syncthreads();
 
-    const uint32_t row0 = blockIdx.x * NT;
-    const uint32_t nrounds = (uint32_t)(J.map.S / ROUND);
+    const uint32_t row0 = blockIdx.x * ROWS_CTA;
+    const uint32_t nrounds = (uint32_t)(J.map.S / ROUND);     // even (S is a multiple of 64)
 
     if (tid >= NT) {                                 // ---- producer warp
         if (tid == NT) {
@@ -347,19 +440,21 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                 if (r >= STAGES) mbar_wait(bars + 64 + 8 * s, ((r / STAGES) - 1u) & 1u);
                 mbar_expect_tx(bars + 8 * s, STAGE_BYTES);
                 const uint32_t dst = stages + s * STAGE_BYTES;
-                tma_load_2d(dst, &tmap, (int)(r * ROUND), (int)row0, bars + 8 * s);
-                tma_load_2d(dst + BOX_ROWS * ROUND, &tmap, (int)(r * ROUND), (int)(row0 + BOX_ROWS),
-                            bars + 8 * s);
+#pragma unroll
+                for (int q = 0; q < ROWS_CTA / BOX_ROWS; ++q)
+                    tma_load_2d(dst + q * BOX_ROWS * ROUND, &tmap, (int)(r * ROUND), (int)(row0 + q * BOX_ROWS),
+                                bars + 8 * s);
             }
         }
         return;
     }
 
-    // ---- consumers: thread tid owns row row0 + tid
+    // ---- consumers: thread tid owns rows rA = row0 + tid and rB = row0 + NT + tid
     const int lane = tid & 31;
-    const uint32_t row = row0 + tid;
-    const bool active = row < J.map.nrows;
-    const uint64_t rpos = J.map.b0 + (uint64_t)row * J.map.S;
+    const uint32_t rowA = row0 + tid, rowB = row0 + NT + tid;
+    const bool actA = rowA < J.map.nrows, actB = rowB < J.map.nrows;
+    const uint64_t posA0 = J.map.b0 + (uint64_t)rowA * J.map.S;
+    const uint64_t posB0 = J.map.b0 + (uint64_t)rowB * J.map.S;
 
     BulkCtx c;
     c.tab = sbase;
@@ -367,112 +462,151 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         c.laneT = sbase + (uint32_t)(lane & 15) * 8u;
         c.laneU = 128u + (uint32_t)(lane & 15) * 8u;
     } else {
-        c.laneT = (uint32_t)lane * 4u;
+        c.laneT = sbase + (uint32_t)lane * 4u;
         c.laneU = 128u + (uint32_t)lane * 4u;
     }
-    c.mask = mask; c.magic = magic;
-    SlotOut o;
-    const uint32_t slot = J.map.n_head + row;
-    o.lst = J.scratch + (uint64_t)slot * J.cap;
-    o.cnt = 0; o.cap = J.cap; o.min_i = J.min_i; o.c_limit = J.c_limit;
+    c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh;
+    SlotOut oA, oB;
+    const uint32_t slotA = J.map.n_head + rowA, slotB = J.map.n_head + rowB;
+    oA.lst = J.scratch + (uint64_t)slotA * J.cap; oA.cnt = 0; oA.cap = J.cap;
+    oB.lst = J.scratch + (uint64_t)slotB * J.cap; oB.cnt = 0; oB.cap = J.cap;
 
-    State<MODE> st;
-    uint4 R1 = make_uint4(0, 0, 0, 0), R2 = R1, R3 = R1;
-    if (active) {
-        // warm-up: the 64 bytes before the row (b0 >= p_begin + 64 guarantees they are in src)
-        const uint4 *h = reinterpret_cast<const uint4 *>(J.src + (rpos - 64u - J.p_begin));
-        const uint4 H0 = __ldg(h + 0), H1 = __ldg(h + 1), H2 = __ldg(h + 2), H3 = __ldg(h + 3);
+    State<MODE> sA, sB;
+    uint4 A1 = make_uint4(0, 0, 0, 0), A2 = A1, A3 = A1, B1 = A1, B2 = A1, B3 = A1;
+    {
+        // warm-up: the 64 bytes before each row (b0 >= p_begin + 64 keeps them inside src)
         const uint4 Z = make_uint4(0, 0, 0, 0);
-        chunk16<MODE, false>(st, H0, Z, 0, c, o);
-        chunk16<MODE, false>(st, H1, Z, 0, c, o);
-        chunk16<MODE, false>(st, H2, Z, 0, c, o);
-        chunk16<MODE, false>(st, H3, H0, 0, c, o);
-        R1 = H1; R2 = H2; R3 = H3;
+        uint4 HA0 = Z, HA1 = Z, HA2 = Z, HA3 = Z, HB0 = Z, HB1 = Z, HB2 = Z, HB3 = Z;
+        if (actA) {
+            const uint4 *h = reinterpret_cast<const uint4 *>(J.src + (posA0 - 64u - J.p_begin));
+            HA0 = __ldg(h + 0); HA1 = __ldg(h + 1); HA2 = __ldg(h + 2); HA3 = __ldg(h + 3);
+        }
+        if (actB) {
+            const uint4 *h = reinterpret_cast<const uint4 *>(J.src + (posB0 - 64u - J.p_begin));
+            HB0 = __ldg(h + 0); HB1 = __ldg(h + 1); HB2 = __ldg(h + 2); HB3 = __ldg(h + 3);
+        }
+        uint32_t mA, mB;
+        chunk16x2<MODE, false>(sA, HA0, Z, sB, HB0, Z, c, mA, mB);
+        chunk16x2<MODE, false>(sA, HA1, Z, sB, HB1, Z, c, mA, mB);
+        chunk16x2<MODE, false>(sA, HA2, Z, sB, HB2, Z, c, mA, mB);
+        chunk16x2<MODE, false>(sA, HA3, HA0, sB, HB3, HB0, c, mA, mB);
+        A1 = HA1; A2 = HA2; A3 = HA3; B1 = HB1; B2 = HB2; B3 = HB3;
     }
 
-    const uint32_t sw = ((uint32_t)tid >> 1) & 3u;
-    const uint32_t rowoff = (uint32_t)tid * ROUND;
-    for (uint32_t r = 0; r < nrounds; ++r) {
-        const uint32_t s = r % STAGES;
-        mbar_wait(bars + 8 * s, (r / STAGES) & 1u);
-        const uint32_t rb = stages + s * STAGE_BYTES + rowoff;
-        const uint4 D0 = lds128(rb + ((0u ^ sw) << 4));
-        const uint4 D1 = lds128(rb + ((1u ^ sw) << 4));
-        const uint4 D2 = lds128(rb + ((2u ^ sw) << 4));
-        const uint4 D3 = lds128(rb + ((3u ^ sw) << 4));
+    const uint32_t swz = ((uint32_t)tid >> 2) & 1u;         // SWIZZLE_32B: chunk ^= (row >> 2) & 1
+    const uint32_t offA = (uint32_t)tid * ROUND, offB = (uint32_t)(NT + tid) * ROUND;
+    for (uint32_t r = 0; r < nrounds; r += 2) {
+        const uint32_t s0 = r % STAGES, s1 = (r + 1) % STAGES;
+        mbar_wait(bars + 8 * s0, (r / STAGES) & 1u);
+        const uint32_t b0s = stages + s0 * STAGE_BYTES;
+        const uint4 DA0 = lds128(b0s + offA + ((0u ^ swz) << 4));
+        const uint4 DA1 = lds128(b0s + offA + ((1u ^ swz) << 4));
+        const uint4 DB0 = lds128(b0s + offB + ((0u ^ swz) << 4));
+        const uint4 DB1 = lds128(b0s + offB + ((1u ^ swz) << 4));
         __syncwarp();
-        if (lane == 0) mbar_arrive(bars + 64 + 8 * s);
-        if (active) {
-            const uint64_t pos = rpos + (uint64_t)r * ROUND;
-            chunk16<MODE, true>(st, D0, R1, pos + 0, c, o);
-            chunk16<MODE, true>(st, D1, R2, pos + 16, c, o);
-            chunk16<MODE, true>(st, D2, R3, pos + 32, c, o);
-            chunk16<MODE, true>(st, D3, D0, pos + 48, c, o);
-        }
-        R1 = D1; R2 = D2; R3 = D3;
+        if (lane == 0) mbar_arrive(bars + 64 + 8 * s0);
+        mbar_wait(bars + 8 * s1, ((r + 1) / STAGES) & 1u);
+        const uint32_t b1s = stages + s1 * STAGE_BYTES;
+        const uint4 DA2 = lds128(b1s + offA + ((0u ^ swz) << 4));
+        const uint4 DA3 = lds128(b1s + offA + ((1u ^ swz) << 4));
+        const uint4 DB2 = lds128(b1s + offB + ((0u ^ swz) << 4));
+        const uint4 DB3 = lds128(b1s + offB + ((1u ^ swz) << 4));
+        __syncwarp();
+        if (lane == 0) mbar_arrive(bars + 64 + 8 * s1);
+
+        const uint64_t pA = posA0 + (uint64_t)r * ROUND, pB = posB0 + (uint64_t)r * ROUND;
+        uint32_t mA, mB;
+        chunk16x2<MODE, true>(sA, DA0, A1, sB, DB0, B1, c, mA, mB);
+        if (mA && actA) emit_mask(mA, pA + 0, J.min_i, J.c_limit, oA);
+        if (mB && actB) emit_mask(mB, pB + 0, J.min_i, J.c_limit, oB);
+        chunk16x2<MODE, true>(sA, DA1, A2, sB, DB1, B2, c, mA, mB);
+        if (mA && actA) emit_mask(mA, pA + 16, J.min_i, J.c_limit, oA);
+        if (mB && actB) emit_mask(mB, pB + 16, J.min_i, J.c_limit, oB);
+        chunk16x2<MODE, true>(sA, DA2, A3, sB, DB2, B3, c, mA, mB);
+        if (mA && actA) emit_mask(mA, pA + 32, J.min_i, J.c_limit, oA);
+        if (mB && actB) emit_mask(mB, pB + 32, J.min_i, J.c_limit, oB);
+        chunk16x2<MODE, true>(sA, DA3, DA0, sB, DB3, DB0, c, mA, mB);
+        if (mA && actA) emit_mask(mA, pA + 48, J.min_i, J.c_limit, oA);
+        if (mB && actB) emit_mask(mB, pB + 48, J.min_i, J.c_limit, oB);
+        A1 = DA1; A2 = DA2; A3 = DA3; B1 = DB1; B2 = DB2; B3 = DB3;
     }
-    if (active) J.counts[slot] = o.cnt;
+    uint32_t totA, totB;
+    const uint32_t offsA = block_exscan(actA ? oA.cnt : 0u, NT, 1, ws, &totA);
+    const uint32_t offsB = block_exscan(actB ? oB.cnt : 0u, NT, 1, ws, &totB);
+    if (actA) { J.counts[slotA] = oA.cnt; J.local_off[slotA] = offsA; }
+    if (actB) { J.counts[slotB] = oB.cnt; J.local_off[slotB] = totA + offsB; }
+    if (tid == 0) J.group_sum[1 + blockIdx.x] = totA + totB;
 }
 
-// ------------------------------------------------------------------------------ k_scan
-// Exclusive scan of counts[0..n) -> offsets (u64); total -> aux->total (and *n_direct if set).
-__global__ void __launch_bounds__(1024)
-k_scan(const uint32_t *__restrict__ counts, uint32_t n, uint64_t *__restrict__ offsets, Aux *aux,
-       uint64_t *n_direct, uint64_t direct_cap) {
-    __shared__ uint64_t warp_sums[32];
-    const uint32_t tid = threadIdx.x;
-    const uint32_t per = (n + blockDim.x - 1) / blockDim.x;
-    const uint32_t a = tid * per;
-    const uint32_t b = min(n, a + per);
-    uint64_t sum = 0;
-    for (uint32_t i = a; i < b; ++i) sum += counts[i];
-    // block-wide exclusive scan of `sum`
-    uint64_t incl = sum;
-    for (int d = 1; d < 32; d <<= 1) {
-        uint64_t v = __shfl_up_sync(0xffffffffu, incl, d);
-        if ((tid & 31) >= (uint32_t)d) incl += v;
-    }
-    if ((tid & 31) == 31) warp_sums[tid >> 5] = incl;
+// ------------------------------------------------------------------------------ k_total
+// Sum of the group sums -> aux->total (bounded path: needed on the host before k_scatter).
+__global__ void k_total(const uint64_t *__restrict__ group_sum, uint32_t ngroups, Aux *aux) {
+    uint64_t s = 0;
+    for (uint32_t g = threadIdx.x; g < ngroups; g += blockDim.x) s += group_sum[g];
+    for (int d = 16; d; d >>= 1) s += __shfl_xor_sync(0xffffffffu, s, d);
+    __shared__ uint64_t w[32];
+    if ((threadIdx.x & 31) == 0) w[threadIdx.x >> 5] = s;
     __syncthreads();
-    if (tid < 32) {
-        uint64_t v = warp_sums[tid];
-        uint64_t vi = v;
-        for (int d = 1; d < 32; d <<= 1) {
-            uint64_t u = __shfl_up_sync(0xffffffffu, vi, d);
-            if (tid >= (uint32_t)d) vi += u;
-        }
-        warp_sums[tid] = vi - v;                  // exclusive warp prefix
-    }
-    __syncthreads();
-    uint64_t run = warp_sums[tid >> 5] + incl - sum;
-    for (uint32_t i = a; i < b; ++i) { offsets[i] = run; run += counts[i]; }
-    if (tid == blockDim.x - 1) {
-        aux->total = run;
-        if (n_direct) {
-            *n_direct = run;
-            if (run > direct_cap) aux->overflow = 1;
-        }
+    if (threadIdx.x == 0) {
+        uint64_t t = 0;
+        for (uint32_t i = 0; i < (blockDim.x + 31) / 32; ++i) t += w[i];
+        aux->total = t;
     }
 }
 
 // ------------------------------------------------------------------------------ k_scatter
-// One thread per slot.  dst[base + offsets[slot] + j] for j < count (bounded by dst_cap);
-// base = aux->out_pos + aux->held when `streaming`, else 0.  Overflowed slots re-roll.
-__global__ void __launch_bounds__(256)
+// One thread per slot (blocks of 256).  Every block scans the group sums itself (<= a few
+// hundred) to get its groups' bases; offset(slot) = base(group) + local_off[slot].
+// dst index = (streaming ? aux->out_pos + aux->held : 0) + offset.  Block 0 writes the
+// total (aux->total, and *n_direct with the overflow flag if given).  Overflowed slots re-roll.
+constexpr int SCATTER_THREADS = 256;
+constexpr int MAX_GROUPS = 4096;
+__global__ void __launch_bounds__(SCATTER_THREADS)
 k_scatter(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots,
-          const uint64_t *__restrict__ offsets, uint64_t *__restrict__ dst, uint64_t dst_cap,
-          Aux *aux, int streaming) {
-    const uint32_t slot = blockIdx.x * blockDim.x + threadIdx.x;
+          uint64_t *__restrict__ dst, uint64_t dst_cap, Aux *aux, int streaming,
+          uint64_t *n_direct) {
+    __shared__ uint64_t gbase[MAX_GROUPS];
+    __shared__ uint64_t wsum[SCATTER_THREADS / 32 + 1];
+    const uint32_t ng = J.map.ngroups;
+    const uint32_t tid = threadIdx.x;
+    // exclusive scan of group_sum[0..ng) into gbase (chunks of 256 with a running carry)
+    uint64_t carry = 0;
+    for (uint32_t b = 0; b < ng; b += SCATTER_THREADS) {
+        const uint32_t g = b + tid;
+        const uint64_t v = g < ng ? J.group_sum[g] : 0ull;
+        uint64_t incl = v;
+        for (int d = 1; d < 32; d <<= 1) {
+            uint64_t u = __shfl_up_sync(0xffffffffu, incl, d);
+            if ((tid & 31) >= (uint32_t)d) incl += u;
+        }
+        if ((tid & 31) == 31) wsum[tid >> 5] = incl;
+        __syncthreads();
+        if (tid == 0) {
+            uint64_t r = 0;
+            for (int w = 0; w < SCATTER_THREADS / 32; ++w) { uint64_t x = wsum[w]; wsum[w] = r; r += x; }
+            wsum[SCATTER_THREADS / 32] = r;
+        }
+        __syncthreads();
+        if (g < ng) gbase[g] = carry + wsum[tid >> 5] + incl - v;
+        carry += wsum[SCATTER_THREADS / 32];
+        __syncthreads();
+    }
+    const uint64_t total = carry;
+    if (blockIdx.x == 0 && tid == 0) {
+        aux->total = total;
+        if (n_direct) { *n_direct = total; if (total > dst_cap) aux->overflow = 1; }
+    }
+    const uint32_t slot = blockIdx.x * blockDim.x + tid;
     if (slot >= nslots) return;
     const uint32_t cnt = J.counts[slot];
     if (cnt == 0) return;
-    const uint64_t base = (streaming ? aux->out_pos + aux->held : 0ull) + offsets[slot];
-    const uint64_t total = aux->total;
+    const uint64_t off = gbase[slot_group(J.map, slot)] + J.local_off[slot];
+    const uint64_t base = (streaming ? aux->out_pos + aux->held : 0ull) + off;
     if (cnt <= J.cap) {
         const uint64_t *lst = J.scratch + (uint64_t)slot * J.cap;
         for (uint32_t j = 0; j < cnt; ++j)
             if (base + j < dst_cap) dst[base + j] = lst[j];
-        if (offsets[slot] + cnt == total) aux->last_cand = lst[cnt - 1];
+        if (off + cnt == total) aux->last_cand = lst[cnt - 1];
     } else {
         uint64_t a, b;
         slot_range(J.map, slot, a, b);
@@ -482,7 +616,7 @@ k_scatter(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots,
             if (base + k < dst_cap) dst[base + k] = c;
             ++k; last = c;
         });
-        if (offsets[slot] + cnt == total) aux->last_cand = last;
+        if (off + cnt == total) aux->last_cand = last;
     }
 }
 

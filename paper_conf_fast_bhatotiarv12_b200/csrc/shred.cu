@@ -96,7 +96,8 @@ struct shred_ctx {
 
     // scratch (grown on demand, synchronously)
     uint32_t *d_counts = nullptr; uint64_t counts_cap = 0;
-    uint64_t *d_offsets = nullptr; uint64_t offsets_cap = 0;
+    uint32_t *d_local = nullptr; uint64_t local_cap = 0;
+    uint64_t *d_groups = nullptr; uint64_t groups_cap = 0;
     uint64_t *d_scratch = nullptr; uint64_t scratch_cap = 0;   // in u64 entries
     uint64_t *d_cand = nullptr; uint64_t cand_cap = 0;         // bounded mode ordered list
     Aux *d_aux = nullptr;                // [0] one-shot calls, [1] the stream
@@ -190,7 +191,7 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
     SlotMap &m = J.map;
     m.t_end = t_end;
     const uint64_t len = t_end > t_begin ? t_end - t_begin : 0;
-    const uint64_t GS = 256;                   // generic head/tail segment
+    const uint64_t GS = 64;                    // head/tail segment (edge CTA)
 
     // bulk region: aligned start b0 >= max(t_begin, p_begin + 64), rows of S bytes
     pl.bulk = false;
@@ -199,32 +200,42 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
         uint64_t lo = t_begin > p_begin + 64 ? t_begin : p_begin + 64;
         const uintptr_t a = (uintptr_t)(src + (lo - p_begin));
         b0 = lo + ((16u - (a & 15u)) & 15u);
-        if (b0 < t_end) {
+        if (b0 + 256 < t_end) {
             const uint64_t blen = t_end - b0;
-            const uint64_t target = (uint64_t)ctx->sm_count * NT;
+            // one wave: (SMs - 1) bulk CTAs of ROWS_CTA rows + the edge CTA
+            const uint64_t target = (uint64_t)(ctx->sm_count > 1 ? ctx->sm_count - 1 : 1) * ROWS_CTA;
             S = (blen + target - 1) / target;
-            S = (S + ROUND - 1) / ROUND * ROUND;
+            S = (S + 63) / 64 * 64;                // an even number of ROUND-byte rounds
             if (S < 256) S = 256;
             nrows = blen / S;
-            if (nrows > 0 && nrows < (1ull << 31) && S < (1ull << 39)) pl.bulk = true;
+            if (nrows > 0 && nrows < (1ull << 31) && S < (1ull << 39) && (b0 - t_begin) <= GS * NT)
+                pl.bulk = true;
         }
     }
     if (!pl.bulk) {
-        // everything generic: segments of about len / (sm_count * 4 * 256) bytes, >= GS
-        uint64_t seg = GS;
+        // generic only: segments of about len / (sm_count * 4 * 256) bytes, >= 256
+        uint64_t seg = 256;
         const uint64_t want = (uint64_t)ctx->sm_count * 4 * GEN_THREADS;
         if (len / want > seg) seg = (len / want + 63) / 64 * 64;
         m.head_start = t_begin; m.head_seg = seg;
         m.n_head = (uint32_t)((len + seg - 1) / seg);
         m.nrows = 0; m.b0 = t_end; m.S = 0;
-        m.tail_start = t_end; m.tail_seg = GS; m.n_tail = 0;
+        m.tail_start = t_end; m.tail_seg = seg; m.n_tail = 0;
+        m.nc = 0;
+        m.ngroups = (m.n_head + GEN_THREADS - 1) / GEN_THREADS;
     } else {
         m.head_start = t_begin; m.head_seg = GS;
         m.n_head = (uint32_t)((b0 - t_begin + GS - 1) / GS);
         m.b0 = b0; m.S = S; m.nrows = (uint32_t)nrows;
-        m.tail_start = b0 + nrows * S; m.tail_seg = GS;
-        m.n_tail = (uint32_t)((t_end - m.tail_start + GS - 1) / GS);
-        pl.bulk_ctas = (uint32_t)((nrows + NT - 1) / NT);
+        m.tail_start = b0 + nrows * S;
+        const uint64_t tl = t_end - m.tail_start;
+        uint64_t ts = (tl + NT - 1) / NT;
+        ts = ts < GS ? GS : (ts + 15) / 16 * 16;
+        m.tail_seg = ts;
+        m.n_tail = (uint32_t)((tl + ts - 1) / ts);
+        m.nc = (uint32_t)((nrows + ROWS_CTA - 1) / ROWS_CTA);
+        m.ngroups = m.nc + 2;
+        pl.bulk_ctas = m.nc + 1;               // + the edge CTA (head + tail, group sums 0, nc+1)
         // 2-D tensor map [nrows][S] over the bulk bytes
         cuuint64_t gdim[2] = {(cuuint64_t)S, (cuuint64_t)nrows};
         cuuint64_t gstride[1] = {(cuuint64_t)S};
@@ -232,34 +243,34 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
         cuuint32_t estr[2] = {1, 1};
         CUresult r = ctx->encode(&pl.tmap, CU_TENSOR_MAP_DATA_TYPE_UINT8, 2,
                                  (void *)(src + (b0 - p_begin)), gdim, gstride, box, estr,
-                                 CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_64B,
+                                 CU_TENSOR_MAP_INTERLEAVE_NONE,
+                                 ROUND == 64 ? CU_TENSOR_MAP_SWIZZLE_64B : CU_TENSOR_MAP_SWIZZLE_32B,
                                  CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
         if (r != CUDA_SUCCESS) return fail(ctx, SHRED_ECUDA, "cuTensorMapEncodeTiled failed (%d)", (int)r);
     }
     pl.nslots = m.n_head + m.nrows + m.n_tail;
+    if (m.ngroups > (uint32_t)MAX_GROUPS) return fail(ctx, SHRED_EINVAL, "too many slot groups (%u)", m.ngroups);
     // per-slot list capacity: twice the expected count of the longest segment + slack
-    const uint64_t maxseg = pl.bulk ? (S > GS ? S : GS) : m.head_seg;
+    uint64_t maxseg = pl.bulk ? S : m.head_seg;
+    if (pl.bulk && m.tail_seg > maxseg) maxseg = m.tail_seg;
     uint64_t cap = 2 * maxseg / ctx->p.divisor + 16;
     if (cap > 256) cap = 256;
     J.cap = (uint32_t)cap;
     int rc;
     if ((rc = grow(ctx, ctx->d_counts, ctx->counts_cap, (uint64_t)pl.nslots + 1, "counts"))) return rc;
-    if ((rc = grow(ctx, ctx->d_offsets, ctx->offsets_cap, (uint64_t)pl.nslots + 1, "offsets"))) return rc;
+    if ((rc = grow(ctx, ctx->d_local, ctx->local_cap, (uint64_t)pl.nslots + 1, "local offsets"))) return rc;
+    if ((rc = grow(ctx, ctx->d_groups, ctx->groups_cap, (uint64_t)m.ngroups + 1, "group sums"))) return rc;
     if ((rc = grow(ctx, ctx->d_scratch, ctx->scratch_cap, (uint64_t)pl.nslots * cap + 1, "scratch"))) return rc;
     J.counts = ctx->d_counts;
+    J.local_off = ctx->d_local;
+    J.group_sum = ctx->d_groups;
     J.scratch = ctx->d_scratch;
     return SHRED_OK;
 }
 
-// K1 (bulk + generic) and k_scan.
-int launch_detect(shred_ctx *ctx, Plan &pl, Aux *aux, uint64_t *n_direct, uint64_t direct_cap,
-                  cudaStream_t st) {
-    if (pl.nslots == 0) {
-        // nothing to test: total = 0
-        k_scan<<<1, 1024, 0, st>>>(ctx->d_counts, 0, ctx->d_offsets, aux, n_direct, direct_cap);
-        LAUNCHED("k_scan");
-        return SHRED_OK;
-    }
+// K1: the TMA hot kernel (+ its edge CTA), or the generic kernel.
+int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
+    if (pl.nslots == 0) return SHRED_OK;
     if (pl.bulk) {
         cudaEvent_t e0 = nullptr, e1 = nullptr;
         if (ctx->prof) {
@@ -272,33 +283,42 @@ int launch_detect(shred_ctx *ctx, Plan &pl, Aux *aux, uint64_t *n_direct, uint64
             }
             e0 = ctx->prof_ev[ctx->prof_used]; e1 = ctx->prof_ev[ctx->prof_used + 1];
             ctx->prof_used += 2;
-            ctx->prof_bytes += (uint64_t)pl.J.map.nrows * pl.J.map.S;
+            ctx->prof_bytes += (pl.J.map.t_end - pl.J.map.head_start);
             CK(cudaEventRecord(e0, st), "profile record");
         }
+        const int m = 32 - (int)__builtin_ctzll(ctx->p.divisor);     // D = 2^(32-m')
+        BulkConst K;
+        K.mhi = ctx->path == SHRED_PATH_K63 ? 512u : 256u;
+        K.m256 = 256u;
+        K.tmul = 1u << m;                                           // 2^(32 - log2 D)
+        K.rsh = (uint32_t)(ctx->p.magic << m);
         if (ctx->path == SHRED_PATH_K63)
-            k1_bulk<MODE_K63><<<pl.bulk_ctas, NT + 32, BULK_SMEM, st>>>(pl.tmap, ctx->d_tab_img, pl.J,
-                                                                        (uint32_t)ctx->dp.dmask, (uint32_t)ctx->dp.magic);
+            k1_bulk<MODE_K63><<<pl.bulk_ctas, NT + 32, BULK_SMEM, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen,
+                                                                        pl.J, ctx->dp, K);
         else
-            k1_bulk<MODE_K32><<<pl.bulk_ctas, NT + 32, BULK_SMEM, st>>>(pl.tmap, ctx->d_tab_img, pl.J,
-                                                                        (uint32_t)ctx->dp.dmask, (uint32_t)ctx->dp.magic);
+            k1_bulk<MODE_K32><<<pl.bulk_ctas, NT + 32, BULK_SMEM, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen,
+                                                                        pl.J, ctx->dp, K);
         LAUNCHED("k1_bulk");
         if (e1) CK(cudaEventRecord(e1, st), "profile record");
-    }
-    const uint32_t ngen = pl.J.map.n_head + pl.J.map.n_tail;
-    if (ngen) {
-        k1_generic<<<(ngen + GEN_THREADS - 1) / GEN_THREADS, GEN_THREADS, 0, st>>>(pl.J, ctx->dp, ctx->d_gen);
+    } else {
+        k1_generic<<<(pl.nslots + GEN_THREADS - 1) / GEN_THREADS, GEN_THREADS, 0, st>>>(pl.J, ctx->dp, ctx->d_gen,
+                                                                                       pl.nslots);
         LAUNCHED("k1_generic");
     }
-    k_scan<<<1, 1024, 0, st>>>(ctx->d_counts, pl.nslots, ctx->d_offsets, aux, n_direct, direct_cap);
-    LAUNCHED("k_scan");
     return SHRED_OK;
 }
 
+// Ordered compaction into dst.  With no slots: total = 0 (and *n_direct = 0).
 int launch_scatter(shred_ctx *ctx, Plan &pl, uint64_t *dst, uint64_t dst_cap, Aux *aux, int streaming,
-                   cudaStream_t st) {
-    if (pl.nslots == 0) return SHRED_OK;
-    k_scatter<<<(pl.nslots + 255) / 256, 256, 0, st>>>(pl.J, ctx->dp, ctx->d_gen, pl.nslots, ctx->d_offsets,
-                                                       dst, dst_cap, aux, streaming);
+                   uint64_t *n_direct, cudaStream_t st) {
+    if (pl.nslots == 0) {
+        k_write_u64<<<1, 1, 0, st>>>(&aux->total, 0);
+        LAUNCHED("k_write_u64");
+        if (n_direct) { k_write_u64<<<1, 1, 0, st>>>(n_direct, 0); LAUNCHED("k_write_u64"); }
+        return SHRED_OK;
+    }
+    k_scatter<<<(pl.nslots + SCATTER_THREADS - 1) / SCATTER_THREADS, SCATTER_THREADS, 0, st>>>(
+        pl.J, ctx->dp, ctx->d_gen, pl.nslots, dst, dst_cap, aux, streaming, n_direct);
     LAUNCHED("k_scatter");
     return SHRED_OK;
 }
@@ -307,7 +327,14 @@ bool bounded(const shred_ctx *ctx) { return ctx->p.min_size > 0 || ctx->p.max_si
 
 // Bounded mode needs the whole ordered candidate list: read the count back (the one
 // synchronous point of the bounded path) and size the ctx buffer for it.
-int ensure_cand(shred_ctx *ctx, Aux *aux, cudaStream_t st, uint64_t &total) {
+int ensure_cand(shred_ctx *ctx, Plan &pl, Aux *aux, cudaStream_t st, uint64_t &total) {
+    if (pl.nslots) {
+        k_total<<<1, 256, 0, st>>>(ctx->d_groups, pl.J.map.ngroups, aux);
+        LAUNCHED("k_total");
+    } else {
+        k_write_u64<<<1, 1, 0, st>>>(&aux->total, 0);
+        LAUNCHED("k_write_u64");
+    }
     CK(cudaMemcpyAsync(ctx->h_pinned, &aux->total, sizeof(uint64_t), cudaMemcpyDeviceToHost, st), "read total");
     CK(cudaStreamSynchronize(st), "sync total");
     total = ctx->h_pinned[0];
@@ -322,9 +349,9 @@ int run_piece(shred_ctx *ctx, Aux *aux, const uint8_t *src, uint64_t p_begin, co
     Plan pl;
     int rc = plan_job(ctx, pl, src, p_begin, prefix, prefix_len, t_begin, t_end, c_limit);
     if (rc) return rc;
-    if ((rc = launch_detect(ctx, pl, aux, nullptr, 0, st))) return rc;
+    if ((rc = launch_detect(ctx, pl, st))) return rc;
     if (!bounded(ctx)) {
-        if ((rc = launch_scatter(ctx, pl, dst, dst_cap, aux, 1, st))) return rc;
+        if ((rc = launch_scatter(ctx, pl, dst, dst_cap, aux, 1, nullptr, st))) return rc;
         if (final_) {
             // one-shot: nothing held; out_pos += total
             k_piece_done<<<1, 1, 0, st>>>(aux, dst, dst_cap, ~0ull);
@@ -335,8 +362,8 @@ int run_piece(shred_ctx *ctx, Aux *aux, const uint8_t *src, uint64_t p_begin, co
         return SHRED_OK;
     }
     uint64_t total = 0;
-    if ((rc = ensure_cand(ctx, aux, st, total))) return rc;
-    if ((rc = launch_scatter(ctx, pl, ctx->d_cand, ctx->cand_cap, aux, 0, st))) return rc;
+    if ((rc = ensure_cand(ctx, pl, aux, st, total))) return rc;
+    if ((rc = launch_scatter(ctx, pl, ctx->d_cand, ctx->cand_cap, aux, 0, nullptr, st))) return rc;
     k_size_bound<<<1, 32, 0, st>>>(ctx->d_cand, &aux->total, 0, t_end, final_, ctx->p.min_size,
                                    ctx->p.max_size, dst, dst_cap, aux);
     LAUNCHED("k_size_bound");
@@ -499,7 +526,7 @@ void shred_destroy(shred_ctx *ctx) {
     for (auto &e : ctx->prof_ev) cudaEventDestroy(e);
     for (auto p : ctx->ring) cudaFree(p);
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
-    cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_counts); cudaFree(ctx->d_offsets);
+    cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_counts); cudaFree(ctx->d_local); cudaFree(ctx->d_groups);
     cudaFree(ctx->d_scratch); cudaFree(ctx->d_cand); cudaFree(ctx->d_aux);
     cudaFree(ctx->d_carry[0]); cudaFree(ctx->d_carry[1]);
     if (ctx->h_pinned) cudaFreeHost(ctx->h_pinned);
@@ -517,14 +544,14 @@ int shred_chunk(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, uint64_t *d_o
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
     Aux *aux = ctx->d_aux + 0;
-    k_stream_reset<<<1, 1, 0, st>>>(aux);
-    LAUNCHED("k_stream_reset");
     if (!bounded(ctx)) {
         Plan pl;
         if ((rc = plan_job(ctx, pl, d_in, 0, nullptr, 0, 0, len, len))) return rc;
-        if ((rc = launch_detect(ctx, pl, aux, n_out, cap, st))) return rc;
-        return launch_scatter(ctx, pl, d_out, cap, aux, 0, st);
+        if ((rc = launch_detect(ctx, pl, st))) return rc;
+        return launch_scatter(ctx, pl, d_out, cap, aux, 0, n_out, st);
     }
+    k_stream_reset<<<1, 1, 0, st>>>(aux);
+    LAUNCHED("k_stream_reset");
     if ((rc = run_piece(ctx, aux, d_in, 0, nullptr, 0, 0, len, len, 1, d_out, cap, st))) return rc;
     k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, nullptr);
     LAUNCHED("k_call_end");
@@ -544,12 +571,10 @@ int shred_candidates_range(shred_ctx *ctx, const uint8_t *d_in, uint64_t halo, u
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
     Aux *aux = ctx->d_aux + 0;
-    k_stream_reset<<<1, 1, 0, st>>>(aux);
-    LAUNCHED("k_stream_reset");
     Plan pl;
     if ((rc = plan_job(ctx, pl, d_in, start - halo, nullptr, 0, start, start + len, total_len))) return rc;
-    if ((rc = launch_detect(ctx, pl, aux, n_out, cap, st))) return rc;
-    return launch_scatter(ctx, pl, d_out, cap, aux, 0, st);
+    if ((rc = launch_detect(ctx, pl, st))) return rc;
+    return launch_scatter(ctx, pl, d_out, cap, aux, 0, n_out, st);
 }
 
 int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, uint64_t total_len,

@@ -1,0 +1,16 @@
+#!/bin/bash
+# GPU-box measurement script (run under gpurun): tests, bench line, ncu launch list, ncu full
+# capture of the hot kernel.  Usage: bash tools/gpu_profile.sh <tag> [skip-tests]
+TAG=${1:-rXX}
+mkdir -p gpurun_out
+nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,power.draw --format=csv
+if [ "$2" != "skip-tests" ]; then
+  timeout 900 python -m pytest tests -m gpu -x -q 2>&1 | tail -15
+fi
+python bench.py 2>&1 | tail -3 > gpurun_out/bench_$TAG.json
+cat gpurun_out/bench_$TAG.json
+ncu --metrics gpu__time_duration.sum --clock-control none -c 400 --csv --log-file gpurun_out/launches_$TAG.csv \
+    python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu --no-extra > /dev/null 2>&1
+ncu --set full --clock-control none --import-source on -k regex:k1_bulk -s 3 -c 1 -o gpurun_out/prof_k1_$TAG \
+    python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu --no-extra > gpurun_out/ncu_full_$TAG.log 2>&1
+tail -2 gpurun_out/ncu_full_$TAG.log
