@@ -1,0 +1,93 @@
+"""Multi-GPU byte-range sharding.
+
+Rank g of G owns the window ends [start_g, end_g) of one stream of `total_len` bytes and holds
+its bytes plus the w-1 = 47 bytes before them (the halo: "a small overlap of the size of the
+sliding window (w bytes) near partition boundaries", L282-L287).  Candidates are independent
+per shard; the only exchange is:
+
+* C2 - an all-gather of the per-rank candidate counts (8 B per rank) -> each rank's exclusive
+  prefix = the index of its first candidate in the global list (unbounded mode, the paper's
+  default: nothing else is exchanged);
+* C3 - bounded mode only: an all-gather of the candidate lists (padded to the largest count),
+  then the sequential size rule over the concatenation on every rank (replicated).
+
+The collectives go through ``torch.distributed`` (NCCL on GPUs; gloo in the CPU tests).  The
+per-shard compute is an *engine*: the product uses :class:`paper_conf_fast_bhatotiarv12_b200.Chunker`
+(CUDA, via the C ABI); the CPU tests plug in an oracle-backed engine instead.
+"""
+from __future__ import annotations
+
+from dataclasses import dataclass
+
+import torch
+import torch.distributed as dist
+
+
+def shard_bounds(total_len: int, world: int, rank: int, align: int = 4096) -> tuple[int, int]:
+    """[start, end) of rank's window ends: contiguous ranges, starts rounded down to `align`."""
+    def cut(g):
+        if g <= 0:
+            return 0
+        if g >= world:
+            return total_len
+        return (total_len * g // world) // align * align
+    return cut(rank), cut(rank + 1)
+
+
+def halo_of(start: int, window: int = 48) -> int:
+    return min(window - 1, start)
+
+
+@dataclass
+class ShardResult:
+    local: torch.Tensor          # this rank's candidates (absolute offsets, ascending)
+    base: int                    # index of local[0] in the global candidate list
+    total: int                   # global number of candidates
+    counts: torch.Tensor         # per-rank counts (int64, on the collective's device)
+    cuts: torch.Tensor | None = None   # bounded mode: the global cut list (replicated)
+
+
+def chunk_sharded(x: torch.Tensor, halo: int, start: int, total_len: int, engine,
+                  group=None, bounded: bool | None = None) -> ShardResult:
+    """Chunk this rank's shard `x` (= stream bytes [start - halo, start + len(x) - halo)).
+
+    engine: has ``candidates_range(x, halo, start, total_len) -> int64 tensor`` and
+    ``size_bound(cands, total_len) -> int64 tensor`` and ``params`` (min_size, max_size)."""
+    world = dist.get_world_size(group)
+    rank = dist.get_rank(group)
+    if bounded is None:
+        bounded = bool(engine.params.min_size or engine.params.max_size)
+    local = engine.candidates_range(x, halo, start, total_len)
+    dev = local.device
+    n = torch.tensor([local.numel()], dtype=torch.int64, device=dev)
+    counts = torch.zeros(world, dtype=torch.int64, device=dev)
+    dist.all_gather_into_tensor(counts, n, group=group)            # C2
+    cs = counts.cpu().tolist()
+    base = int(sum(cs[:rank]))
+    total = int(sum(cs))
+    res = ShardResult(local=local, base=base, total=total, counts=counts)
+    if not bounded:
+        return res
+    # C3: all-gather the (padded) candidate lists, then the global size rule (replicated)
+    mx = max(cs) if cs else 0
+    pad = torch.zeros(max(1, mx), dtype=torch.int64, device=dev)
+    pad[:local.numel()] = local
+    allp = torch.zeros(world * max(1, mx), dtype=torch.int64, device=dev)
+    dist.all_gather_into_tensor(allp, pad, group=group)
+    allp = allp.view(world, max(1, mx))
+    cat = torch.cat([allp[g, :cs[g]] for g in range(world)]) if total else allp.new_zeros(0)
+    res.cuts = engine.size_bound(cat.contiguous(), total_len)
+    return res
+
+
+def gather_all(res: ShardResult, group=None) -> torch.Tensor:
+    """Concatenate every rank's local candidates (rank order) on every rank."""
+    world = dist.get_world_size(group)
+    cs = res.counts.cpu().tolist()
+    mx = max(1, max(cs) if cs else 0)
+    pad = torch.zeros(mx, dtype=torch.int64, device=res.local.device)
+    pad[:res.local.numel()] = res.local
+    allp = torch.zeros(world * mx, dtype=torch.int64, device=res.local.device)
+    dist.all_gather_into_tensor(allp, pad, group=group)
+    allp = allp.view(world, mx)
+    return torch.cat([allp[g, :cs[g]] for g in range(world)])

@@ -1,0 +1,120 @@
+"""Multi-process (gloo, world size 2 and 3, CPU) tests of the sharding orchestration (dist.py).
+
+The per-shard engine here is the CPU oracle (test infrastructure), so these tests pin the
+host logic: shard bounds, halos, the count all-gather and global offsets (C2), and the bounded
+mode's candidate all-gather + global size rule (C3).  The CUDA engine is the same interface
+(Chunker.candidates_range / size_bound) and is covered by tests/test_gpu_parity.py (virtual
+shards) on one GPU.
+"""
+import os
+import socket
+
+import numpy as np
+import pytest
+import torch
+import torch.distributed as dist
+import torch.multiprocessing as mp
+
+import oracle
+import synthgen
+
+
+class OracleEngine:
+    """Per-shard engine backed by the oracle (tests only)."""
+
+    def __init__(self, params: oracle.Params, data: np.ndarray):
+        self.params = params
+        self.data = data
+
+    def candidates_range(self, x, halo, start, total_len):
+        xs = x.numpy()
+        w = self.params.window
+        fps = oracle.window_fps(xs, self.params)                  # fp_i for local i >= w-1
+        i_loc = np.nonzero(fps % np.uint64(self.params.divisor) == np.uint64(self.params.magic))[0] + (w - 1)
+        c = i_loc.astype(np.int64) + (start - halo) + 1           # absolute cut c = i + 1
+        c = c[(c >= start + 1) & (c < total_len)]                 # window ends i >= start
+        return torch.from_numpy(c)
+
+    def size_bound(self, cands, total_len):
+        return torch.from_numpy(oracle.size_bound(cands.numpy().astype(np.uint64), total_len,
+                                                  self.params.min_size, self.params.max_size).astype(np.int64))
+
+
+def _free_port():
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    p = s.getsockname()[1]
+    s.close()
+    return p
+
+
+def _worker(rank, world, port, n, seed, params, q):
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        from paper_conf_fast_bhatotiarv12_b200 import dist as sd
+        data = synthgen.random_bytes(seed, n)
+        start, end = sd.shard_bounds(n, world, rank, align=4096)
+        halo = sd.halo_of(start, params.window)
+        x = torch.from_numpy(synthgen.random_bytes(seed, end - start + halo, start - halo))
+        assert np.array_equal(x.numpy(), data[start - halo:end])   # halo regenerated locally
+        eng = OracleEngine(params, data)
+        res = sd.chunk_sharded(x, halo, start, n, eng)
+        allc = sd.gather_all(res).numpy()
+        q.put((rank, res.base, res.total, res.local.numpy().tolist(), allc.tolist(),
+               None if res.cuts is None else res.cuts.numpy().tolist()))
+    finally:
+        dist.destroy_process_group()
+
+
+def _run(world, n, seed, params):
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_worker, args=(r, world, port, n, seed, params, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    out = [q.get(timeout=300) for _ in range(world)]
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    return sorted(out)
+
+
+@pytest.mark.parametrize("world", [2, 3])
+def test_sharded_unbounded_matches_whole_stream(world):
+    n = (1 << 20) + 12345
+    params = oracle.Params(divisor=1024)
+    exp = oracle.candidates(synthgen.random_bytes(7, n), params).astype(np.int64).tolist()
+    out = _run(world, n, 7, params)
+    cat = []
+    for rank, base, total, local, allc, cuts in out:
+        assert base == len(cat)
+        assert total == len(exp)
+        cat += local
+        assert allc == exp
+        assert cuts is None
+    assert cat == exp
+
+
+def test_sharded_bounded_global_size_rule():
+    n = (1 << 20) + 999
+    params = oracle.Params(divisor=512, min_size=128, max_size=4096)
+    data = synthgen.random_bytes(9, n)
+    exp = oracle.chunk(data, params).astype(np.int64).tolist()
+    out = _run(2, n, 9, params)
+    for rank, base, total, local, allc, cuts in out:
+        assert cuts == exp
+
+
+def test_shard_bounds_cover_the_stream():
+    from paper_conf_fast_bhatotiarv12_b200 import dist as sd
+    for n in (0, 1, 4095, 4096, 10 ** 6, 64 << 30):
+        for world in (1, 2, 3, 8):
+            spans = [sd.shard_bounds(n, world, r) for r in range(world)]
+            assert spans[0][0] == 0 and spans[-1][1] == n
+            for (a, b), (c, d) in zip(spans, spans[1:]):
+                assert b == c and a <= b
+            for a, _ in spans:
+                assert sd.halo_of(a) == min(47, a)
