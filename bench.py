@@ -375,7 +375,7 @@ def main():
         try:
             chb = pkg.Chunker(pkg.Params(min_size=2048, max_size=65536), device=local)
             line["bounded_2048_65536"] = {"value": round(timed(chb, base), 2), "unit": "GB/s",
-                                          "note": "size rule on: one host sync + single-warp K3 (v0)"}
+                                          "note": "size rule on: one host sync (count) + parallel speculative size-rule kernels"}
             c32 = pkg.Chunker(pkg.Params(poly=0x104C11DB7), device=local)
             v32 = timed(c32, base)
             line["k32_variant"] = {"value": round(v32, 2), "unit": "GB/s", "hbm_frac": round(v32 / hbm, 4),

@@ -22,7 +22,7 @@
 //   k_scatter       Ordered compaction: group prefix (from the group sums) + local offset,
 //                   copies the per-slot lists into the destination; slots that overflowed
 //                   their list re-roll their range and write directly.
-//   k_size_bound    The sequential min/max rule (one warp), with streaming state.
+//   (size_bound.cuh) the min/max rule: speculative blocks + convergence check + emit.
 #pragma once
 #include <cstdint>
 #include <cuda.h>
@@ -659,47 +659,6 @@ __global__ void k_carry(const uint8_t *old_c, uint32_t old_len, const uint8_t *s
     for (uint32_t j = threadIdx.x; j < nl; j += blockDim.x) {
         const uint64_t v = tot - nl + j;        // index into (old || src)
         new_c[j] = (v < old_len) ? old_c[v] : src[v - old_len];
-    }
-}
-
-// ------------------------------------------------------------------------------ k_size_bound
-// The min/max rule (readings Q12-Q15), one warp, sequential over the
-// ascending candidates; lanes load 32 candidates at a time.  State (s, held) lives in `aux`.
-//   final = 1 (one-shot): stream end N = end; cuts must be < N.
-//   final = 0 (streaming piece): a cut exactly at `end` is held (emitted by the next piece).
-// ncand is read from *ncand_dev if non-null, else ncand_host.
-__global__ void __launch_bounds__(32)
-k_size_bound(const uint64_t *__restrict__ cand, const uint64_t *ncand_dev, uint64_t ncand_host,
-             uint64_t end, int final_, uint64_t minsz, uint64_t maxsz,
-             uint64_t *__restrict__ dst, uint64_t dst_cap, Aux *aux) {
-    const int lane = threadIdx.x;
-    const uint64_t n = ncand_dev ? *ncand_dev : ncand_host;
-    uint64_t s = aux->s;
-    uint64_t k = aux->out_pos;
-    uint64_t held = aux->held, held_val = aux->held_val;
-    if (held) { if (lane == 0 && k < dst_cap) dst[k] = held_val; ++k; held = 0; }
-    const uint64_t INF = ~0ull;
-    const uint64_t mx = maxsz ? maxsz : INF;
-    for (uint64_t b = 0; b < n; b += 32) {
-        const uint64_t v = (b + lane < n) ? cand[b + lane] : 0ull;
-        const int m = (int)((n - b) < 32 ? (n - b) : 32);
-        for (int j = 0; j < m; ++j) {
-            const uint64_t c = __shfl_sync(0xffffffffu, v, j);
-            if (maxsz) {
-                while (c - s > mx) { s += mx; if (lane == 0 && k < dst_cap) dst[k] = s; ++k; }
-            }
-            if (c - s >= minsz) {
-                s = c;
-                if (!final_ && c == end) { held = 1; held_val = c; }
-                else { if (lane == 0 && k < dst_cap) dst[k] = c; ++k; }
-            }
-        }
-    }
-    if (maxsz) {
-        while (end - s > mx) { s += mx; if (lane == 0 && k < dst_cap) dst[k] = s; ++k; }
-    }
-    if (lane == 0) {
-        aux->s = s; aux->out_pos = k; aux->held = held; aux->held_val = held_val;
     }
 }
 

@@ -2,11 +2,12 @@
 //
 // Owns: parameter validation (incl. an irreducibility test of div(x)),
 // host construction of the push/pop tables, the per-ctx device buffers, the launch sequence
-//   K1 (k1_bulk TMA hot loop + k1_generic head/tail) -> k_scan -> k_scatter [-> k_size_bound]
+//   K1 (k1_bulk TMA hot loop + its edge CTA | k1_generic) -> k_scatter [-> sb_* size rule]
 // and the host-fed streaming ring (§4.1-§4.2: pinned buffers, async H2D on a copy
 // stream, double/triple buffering of device slots).  No CPU fallback: every step of the path
 // runs in the kernels of kernels.cuh.
 #include "kernels.cuh"
+#include "size_bound.cuh"
 #include "../../include/shred.h"
 
 #include <cstdarg>
@@ -100,6 +101,7 @@ struct shred_ctx {
     uint64_t *d_groups = nullptr; uint64_t groups_cap = 0;
     uint64_t *d_scratch = nullptr; uint64_t scratch_cap = 0;   // in u64 entries
     uint64_t *d_cand = nullptr; uint64_t cand_cap = 0;         // bounded mode ordered list
+    uint64_t *d_sb = nullptr; uint64_t sb_cap = 0;             // size-rule block scratch
     Aux *d_aux = nullptr;                // [0] one-shot calls, [1] the stream
     uint64_t *h_pinned = nullptr;        // small pinned readback area
     uint64_t *h_flag = nullptr;          // mapped pinned word: a streaming call overflowed
@@ -325,6 +327,34 @@ int launch_scatter(shred_ctx *ctx, Plan &pl, uint64_t *dst, uint64_t dst_cap, Au
 
 bool bounded(const shred_ctx *ctx) { return ctx->p.min_size > 0 || ctx->p.max_size > 0; }
 
+// The size rule over n ascending candidates (n known on the host for the grid sizes; the
+// kernels read the count from n_dev if given).  Appends to dst at aux->out_pos; updates aux.
+int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_dev, uint64_t n,
+                      uint64_t end, int fin, uint64_t *dst, uint64_t cap, Aux *aux, cudaStream_t st) {
+    const uint64_t nb = (n + SB_B - 1) / SB_B;
+    int rc = grow(ctx, ctx->d_sb, ctx->sb_cap, 6 * (nb + 2), "size-rule scratch");
+    if (rc) return rc;
+    SBArgs A;
+    A.cand = cand; A.n_dev = n_dev; A.n_host = n;
+    A.minsz = ctx->p.min_size; A.maxsz = ctx->p.max_size; A.end = end; A.fin = fin;
+    uint64_t *b = ctx->d_sb;
+    A.spec_exit = b; A.spec_cnt = b + (nb + 2); A.entry = b + 2 * (nb + 2); A.offs = b + 3 * (nb + 2);
+    A.delta = (int64_t *)(b + 4 * (nb + 2)); A.ok = (uint32_t *)(b + 5 * (nb + 2));
+    A.dst = dst; A.dst_cap = cap; A.aux = aux;
+    const unsigned g = (unsigned)((nb + SB_THREADS - 1) / SB_THREADS);
+    if (nb) {
+        sb_spec<<<g, SB_THREADS, 0, st>>>(A);
+        LAUNCHED("sb_spec");
+        sb_check<<<g, SB_THREADS, 0, st>>>(A);
+        LAUNCHED("sb_check");
+    }
+    sb_plan<<<1, 1024, 0, st>>>(A);
+    LAUNCHED("sb_plan");
+    sb_emit<<<(unsigned)((nb + 1 + SB_THREADS - 1) / SB_THREADS), SB_THREADS, 0, st>>>(A);
+    LAUNCHED("sb_emit");
+    return SHRED_OK;
+}
+
 // Bounded mode needs the whole ordered candidate list: read the count back (the one
 // synchronous point of the bounded path) and size the ctx buffer for it.
 int ensure_cand(shred_ctx *ctx, Plan &pl, Aux *aux, cudaStream_t st, uint64_t &total) {
@@ -364,10 +394,7 @@ int run_piece(shred_ctx *ctx, Aux *aux, const uint8_t *src, uint64_t p_begin, co
     uint64_t total = 0;
     if ((rc = ensure_cand(ctx, pl, aux, st, total))) return rc;
     if ((rc = launch_scatter(ctx, pl, ctx->d_cand, ctx->cand_cap, aux, 0, nullptr, st))) return rc;
-    k_size_bound<<<1, 32, 0, st>>>(ctx->d_cand, &aux->total, 0, t_end, final_, ctx->p.min_size,
-                                   ctx->p.max_size, dst, dst_cap, aux);
-    LAUNCHED("k_size_bound");
-    return SHRED_OK;
+    return launch_size_bound(ctx, ctx->d_cand, nullptr, total, t_end, final_, dst, dst_cap, aux, st);
 }
 
 // Kind of a user pointer: 1 = device, 2 = page-locked host, 0 = pageable / unknown.
@@ -527,7 +554,7 @@ void shred_destroy(shred_ctx *ctx) {
     for (auto p : ctx->ring) cudaFree(p);
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
     cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_counts); cudaFree(ctx->d_local); cudaFree(ctx->d_groups);
-    cudaFree(ctx->d_scratch); cudaFree(ctx->d_cand); cudaFree(ctx->d_aux);
+    cudaFree(ctx->d_scratch); cudaFree(ctx->d_cand); cudaFree(ctx->d_sb); cudaFree(ctx->d_aux);
     cudaFree(ctx->d_carry[0]); cudaFree(ctx->d_carry[1]);
     if (ctx->h_pinned) cudaFreeHost(ctx->h_pinned);
     if (ctx->h_flag) cudaFreeHost(ctx->h_flag);
@@ -588,9 +615,7 @@ int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, ui
     Aux *aux = ctx->d_aux + 0;
     k_stream_reset<<<1, 1, 0, st>>>(aux);
     LAUNCHED("k_stream_reset");
-    k_size_bound<<<1, 32, 0, st>>>(d_cand, nullptr, n_cand, total_len, 1, ctx->p.min_size,
-                                   ctx->p.max_size, d_out, cap, aux);
-    LAUNCHED("k_size_bound");
+    if ((rc = launch_size_bound(ctx, d_cand, nullptr, n_cand, total_len, 1, d_out, cap, aux, st))) return rc;
     k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, nullptr);
     LAUNCHED("k_call_end");
     return SHRED_OK;

@@ -1,0 +1,214 @@
+// size_bound.cuh — the min/max chunk-size rule on the device.
+//
+// The rule (readings Q12-Q15), over ascending candidates c with state
+// s = the last cut (0 at the stream start):
+//     while c - s > max: s += max, emit s          (forced cut: no acceptable marker in max bytes)
+//     if c - s >= min:   emit c, s = c             (markers closer than min are dropped)
+//   and at the end of the stream N: while N - s > max: s += max, emit s (s < N).
+// It is sequential in s, but the state is a single number and two runs over the same
+// candidates that ever reach the same s stay identical afterwards.  The parallel form
+// (exact for any input):
+//   sb_spec   block b of SB_B candidates runs speculatively from g_b = c[first-1] (i.e. "the
+//             previous candidate was accepted"); block 0 runs from the true initial state.
+//             -> spec exit state, spec count.
+//   sb_check  block b runs from e_b = spec exit of block b-1 in lockstep with its speculation
+//             until the two states coincide (sync) -> count delta; no sync -> not ok.
+//   sb_plan   one CTA: if every block synced, entries = spec exits and the offsets are a scan
+//             of the counts; otherwise thread 0 walks the unsynced blocks sequentially (exact).
+//   sb_emit   every block re-runs from its true entry and writes its cuts at its offset; one
+//             extra thread writes the forced cuts after the last candidate.
+// Streaming: `fin` = 1 for a whole stream (cuts < end = N); fin = 0 for a fed piece: an accepted
+// candidate exactly at `end` is held (emitted first by the next piece or dropped by the flush),
+// forced cuts strictly before `end` are emitted.
+#pragma once
+#include "kernels.cuh"
+
+namespace shred {
+
+constexpr int SB_B = 256;           // candidates per block
+constexpr int SB_THREADS = 128;
+
+struct SBArgs {
+    const uint64_t *cand;           // ascending candidates
+    const uint64_t *n_dev;          // candidate count (device), or null -> n_host
+    uint64_t n_host;
+    uint64_t minsz, maxsz;          // maxsz 0 = inf
+    uint64_t end;                   // stream end (fin = 1) or current fed end (fin = 0)
+    int fin;
+    uint64_t *spec_exit, *spec_cnt, *entry, *offs;   // [nb] each
+    int64_t *delta;
+    uint32_t *ok;
+    uint64_t *dst; uint64_t dst_cap;
+    Aux *aux;                       // s, held, held_val, out_pos (streaming state)
+};
+
+__device__ __forceinline__ uint64_t sb_n(const SBArgs &A) { return A.n_dev ? *A.n_dev : A.n_host; }
+
+// One candidate: returns the number of cuts emitted (forced + accepted, held excluded).
+template <class Emit>
+__device__ __forceinline__ uint64_t sb_step(uint64_t &s, uint64_t c, const SBArgs &A, int &held, Emit emit) {
+    uint64_t k = 0;
+    if (A.maxsz && c - s > A.maxsz) {
+        const uint64_t m = (c - s - 1) / A.maxsz;     // forced cuts s+max, ..., s+m*max (all < c)
+        for (uint64_t j = 1; j <= m; ++j) emit(s + j * A.maxsz);
+        s += m * A.maxsz;
+        k += m;
+    }
+    if (c - s >= A.minsz) {
+        s = c;
+        if (!A.fin && c == A.end) held = 1;
+        else { emit(c); ++k; }
+    }
+    return k;
+}
+struct NoEmit { __device__ void operator()(uint64_t) const {} };
+
+// Forced cuts after the last candidate, strictly before `end`.
+__device__ __forceinline__ uint64_t sb_tail_count(uint64_t s, const SBArgs &A) {
+    if (!A.maxsz || A.end <= s) return 0;
+    return (A.end - s - 1) / A.maxsz;
+}
+
+__global__ void __launch_bounds__(SB_THREADS) sb_spec(SBArgs A) {
+    const uint64_t n = sb_n(A);
+    const uint64_t nb = (n + SB_B - 1) / SB_B;
+    const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    if (b >= nb) return;
+    const uint64_t first = b * SB_B, last = min(n, first + SB_B);
+    uint64_t s = b ? A.cand[first - 1] : A.aux->s;
+    uint64_t cnt = 0;
+    int held = 0;
+    for (uint64_t k = first; k < last; ++k) cnt += sb_step(s, A.cand[k], A, held, NoEmit{});
+    A.spec_exit[b] = s;
+    A.spec_cnt[b] = cnt;
+}
+
+__global__ void __launch_bounds__(SB_THREADS) sb_check(SBArgs A) {
+    const uint64_t n = sb_n(A);
+    const uint64_t nb = (n + SB_B - 1) / SB_B;
+    const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    if (b >= nb) return;
+    if (b == 0) { A.ok[0] = 1; A.delta[0] = 0; return; }
+    const uint64_t first = b * SB_B, last = min(n, first + SB_B);
+    uint64_t s1 = A.spec_exit[b - 1], s2 = A.cand[first - 1];
+    int64_t c1 = 0, c2 = 0;
+    int h1 = 0, h2 = 0;
+    uint32_t ok = (s1 == s2);
+    for (uint64_t k = first; k < last && !ok; ++k) {
+        const uint64_t c = A.cand[k];
+        c1 += (int64_t)sb_step(s1, c, A, h1, NoEmit{});
+        c2 += (int64_t)sb_step(s2, c, A, h2, NoEmit{});
+        ok = (s1 == s2) && (h1 == h2);
+    }
+    A.ok[b] = ok;
+    A.delta[b] = c1 - c2;
+}
+
+// One CTA: entries, offsets, totals and the streaming state.
+__global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
+    __shared__ uint64_t wsum[33];
+    __shared__ int all_ok;
+    const uint64_t n = sb_n(A);
+    const uint32_t nb = (uint32_t)((n + SB_B - 1) / SB_B);
+    const uint32_t tid = threadIdx.x;
+    if (tid == 0) all_ok = 1;
+    __syncthreads();
+    for (uint32_t b = tid; b < nb; b += blockDim.x)
+        if (!A.ok[b]) all_ok = 0;
+    __syncthreads();
+    Aux *aux = A.aux;
+    const uint64_t held_prev = aux->held;
+    const uint64_t base0 = aux->out_pos + held_prev;
+    if (all_ok) {
+        // exclusive scan of true counts, in chunks of 1024 with a carry
+        uint64_t carry = 0;
+        for (uint32_t b0 = 0; b0 < nb; b0 += blockDim.x) {
+            const uint32_t b = b0 + tid;
+            const uint64_t v = b < nb ? (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]) : 0ull;
+            uint64_t incl = v;
+            for (int d = 1; d < 32; d <<= 1) {
+                uint64_t u = __shfl_up_sync(0xffffffffu, incl, d);
+                if ((tid & 31) >= (uint32_t)d) incl += u;
+            }
+            if ((tid & 31) == 31) wsum[tid >> 5] = incl;
+            __syncthreads();
+            if (tid == 0) {
+                uint64_t r = 0;
+                for (int w = 0; w < 32; ++w) { uint64_t x = wsum[w]; wsum[w] = r; r += x; }
+                wsum[32] = r;
+            }
+            __syncthreads();
+            if (b < nb) {
+                A.offs[b] = base0 + carry + wsum[tid >> 5] + incl - v;
+                A.entry[b] = b ? A.spec_exit[b - 1] : aux->s;
+            }
+            carry += wsum[32];
+            __syncthreads();
+        }
+        if (tid == 0) {
+            const uint64_t s_last = nb ? A.spec_exit[nb - 1] : aux->s;
+            // the held flag of the piece: the last candidate accepted exactly at `end`
+            int held_new = 0;
+            if (!A.fin && n > 0 && A.cand[n - 1] == A.end && s_last == A.end) held_new = 1;
+            const uint64_t mt = sb_tail_count(s_last, A);
+            if (held_prev && aux->out_pos < A.dst_cap) A.dst[aux->out_pos] = aux->held_val;
+            aux->out_pos = base0 + carry + mt;
+            aux->s = s_last + mt * A.maxsz;
+            aux->held = (uint64_t)held_new;
+            aux->held_val = held_new ? A.end : 0;
+            aux->total = carry + mt;
+            A.offs[nb] = base0 + carry;           // the tail's forced cuts start here
+            A.entry[nb] = s_last;
+        }
+        return;
+    }
+    if (tid != 0) return;
+    // ---- sequential fallback (blocks that never synced with their speculation): exact
+    uint64_t s = aux->s, off = base0;
+    int held = 0;
+    for (uint32_t b = 0; b < nb; ++b) {
+        const uint64_t first = (uint64_t)b * SB_B, last = min(n, first + SB_B);
+        A.entry[b] = s;
+        A.offs[b] = off;
+        if (b == 0 || (A.ok[b] && s == A.spec_exit[b - 1])) {
+            off += (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]);
+            s = A.spec_exit[b];
+            held = (!A.fin && last == n && A.cand[n - 1] == A.end && s == A.end) ? 1 : 0;
+        } else {
+            held = 0;
+            for (uint64_t k = first; k < last; ++k) off += sb_step(s, A.cand[k], A, held, NoEmit{});
+        }
+    }
+    const uint64_t mt = sb_tail_count(s, A);
+    if (held_prev && aux->out_pos < A.dst_cap) A.dst[aux->out_pos] = aux->held_val;
+    A.offs[nb] = off;
+    A.entry[nb] = s;
+    aux->total = off - base0 + mt;
+    aux->out_pos = off + mt;
+    aux->s = s + mt * A.maxsz;
+    aux->held = (uint64_t)held;
+    aux->held_val = held ? A.end : 0;
+}
+
+// Every block writes its cuts; thread nb writes the forced cuts after the last candidate.
+__global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
+    const uint64_t n = sb_n(A);
+    const uint64_t nb = (n + SB_B - 1) / SB_B;
+    const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
+    if (b > nb) return;
+    uint64_t s = A.entry[b];
+    uint64_t o = A.offs[b];
+    uint64_t *dst = A.dst;
+    const uint64_t cap = A.dst_cap;
+    auto emit = [&](uint64_t v) { if (o < cap) dst[o] = v; ++o; };
+    if (b == nb) {
+        const uint64_t mt = sb_tail_count(s, A);
+        for (uint64_t j = 1; j <= mt; ++j) emit(s + j * A.maxsz);
+        return;
+    }
+    const uint64_t first = b * SB_B, last = min(n, first + SB_B);
+    int held = 0;
+    for (uint64_t k = first; k < last; ++k) sb_step(s, A.cand[k], A, held, emit);
+}
+
+}  // namespace shred

@@ -214,3 +214,36 @@ def test_config2_1gib_and_edited_version(pkg):
     chb = pkg.Chunker(pkg.Params(min_size=2048, max_size=65536))
     cuts = chb.chunk(base).cpu().numpy().astype(np.uint64)
     assert np.array_equal(cuts, oracle.size_bound(exp, n, 2048, 65536))
+
+
+# ------------------------------------------------------------------ size rule (a5) in isolation
+def _sb_cases():
+    rng = np.random.default_rng(17)
+    yield np.arange(48, 200000, 2, dtype=np.uint64), 200001, 3, 0          # phases never sync
+    yield np.arange(48, 200000, 2, dtype=np.uint64), 200001, 5, 9
+    yield np.arange(48, 300000, 3, dtype=np.uint64), 300000, 4, 0
+    yield np.zeros(0, np.uint64), 1 << 20, 2048, 65536                    # forced cuts only
+    yield np.array([5], np.uint64), 10, 0, 3
+    yield np.unique(rng.integers(1, 1 << 26, 200000)).astype(np.uint64), 1 << 26, 256, 1024
+    yield np.unique(rng.integers(1, 1 << 30, 5000)).astype(np.uint64), 1 << 30, 2048, 65536  # long gaps
+    c = np.unique(rng.integers(1, 1 << 22, 100000)).astype(np.uint64)
+    yield c, 1 << 22, 0, 64
+    yield c, 1 << 22, 64, 64
+    yield c, 1 << 22, 1, 1
+
+
+def test_size_bound_api_vs_oracle(pkg):
+    for cand, n, mn, mx in _sb_cases():
+        ch = pkg.Chunker(pkg.Params(divisor=2, magic=0, min_size=mn, max_size=mx))
+        got = ch.size_bound(torch.from_numpy(cand.astype(np.int64)).cuda(), n).cpu().numpy()
+        exp = oracle.size_bound(cand, n, mn, mx)
+        assert np.array_equal(got.astype(np.uint64), exp), (len(cand), n, mn, mx)
+
+
+def test_bounded_adversarial_stream(pkg):
+    """(04 D5)* gives a candidate every 2 bytes: with min = 3 the blocks' speculative runs are
+    out of phase half the time, so the exact sequential fallback of sb_plan is exercised."""
+    n = (4 << 20) + 11
+    per = synthgen.periodic(b"\x04\xd5", n)
+    for mn, mx in ((3, 0), (3, 1000), (4097, 65536)):
+        check_chunk(pkg.Chunker(pkg.Params(min_size=mn, max_size=mx)), per)
