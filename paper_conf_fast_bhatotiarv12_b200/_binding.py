@@ -14,7 +14,7 @@ import torch
 
 from . import _build
 
-LIB_PATH = _build.LIB
+LIB_PATH = os.environ.get("SHRED_LIB", _build.LIB)   # override: A/B variant builds
 
 SHRED_PATH_K63, SHRED_PATH_K32, SHRED_PATH_GENERIC = 1, 2, 3
 PATH_NAMES = {1: "k63", 2: "k32", 3: "generic"}
@@ -51,7 +51,7 @@ def lib() -> ctypes.CDLL:
     """Load libshred.so (building it in-tree if the sources are newer). Raises if unavailable."""
     global _lib
     if _lib is None:
-        if _build.stale():
+        if LIB_PATH == _build.LIB and _build.stale():
             _build.build()
         if not os.path.exists(LIB_PATH):
             raise ShredError(f"{LIB_PATH} missing: run __graft_entry__.build()")

@@ -23,20 +23,24 @@ def stale() -> bool:
     return any(os.path.getmtime(d) > t for d in DEPS)
 
 
-def build(force: bool = False, verbose: bool = False) -> str:
-    if not force and not stale():
+def build(force: bool = False, verbose: bool = False, out: str | None = None,
+          defines: tuple[str, ...] = ()) -> str:
+    """Build libshred.so (or a variant `out` with extra -D defines, for A/B measurements)."""
+    target = out or LIB
+    if out is None and not force and not stale():
         return LIB
-    tmp = LIB + f".tmp{os.getpid()}"
-    cmd = [NVCC, *FLAGS, "-o", tmp, *SOURCES]
+    tmp = target + f".tmp{os.getpid()}"
+    cmd = [NVCC, *FLAGS, *[f"-D{d}" for d in defines], "-o", tmp, *SOURCES]
     r = subprocess.run(cmd, capture_output=True, text=True)
     if r.returncode != 0:
         raise RuntimeError("nvcc failed:\n" + r.stdout + r.stderr)
     if verbose:
         print(r.stderr)
-    with open(os.path.join(PKG, "ptxas_info.txt"), "w") as f:
-        f.write(r.stderr)
-    os.replace(tmp, LIB)
-    return LIB
+    if out is None:
+        with open(os.path.join(PKG, "ptxas_info.txt"), "w") as f:
+            f.write(r.stderr)
+    os.replace(tmp, target)
+    return target
 
 
 if __name__ == "__main__":

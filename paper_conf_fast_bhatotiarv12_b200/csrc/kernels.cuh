@@ -28,6 +28,13 @@
 #include <cuda.h>
 #include <cuda_runtime.h>
 
+#ifndef SHRED_PUSHHI_FMA
+#define SHRED_PUSHHI_FMA 0      // 1: f_hi shift-in as IMAD.HI + IMAD (FMA pipe) instead of PRMT
+#endif
+#ifndef SHRED_HITMODE
+#define SHRED_HITMODE 0         // 0: per-byte hit bitmask; 1: chunk predicate + exact replay on hit
+#endif
+
 namespace shred {
 
 enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3 };
@@ -295,7 +302,11 @@ __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, 
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
     const uint2 T = lds64(ti);
     const uint2 U = lds64(c.tab + oi);
+#if SHRED_PUSHHI_FMA
+    const uint32_t nh = fh * c.m256 + __umulhi(fl, c.m256);       // (fh << 8) | (fl >> 24)
+#else
     const uint32_t nh = __byte_perm(fh, fl, 0x2107u);
+#endif
     const uint32_t nl = __byte_perm(fl, in, 0x2104u + K);
     fl = nl ^ T.x ^ U.x;
     fh = nh ^ T.y ^ U.y;
@@ -354,14 +365,21 @@ template <int MODE, bool TEST, int J>
 __device__ __forceinline__ void word4x2(State<MODE> &a, uint32_t ina, uint32_t popa, uint32_t &mA,
                                         State<MODE> &b, uint32_t inb, uint32_t popb, uint32_t &mB,
                                         const BulkCtx &c) {
+#if SHRED_HITMODE == 0
+#define SHRED_MARK(q) if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + q)) : 0u; \
+                                  mB |= is_marker(b.low(), c) ? (1u << (4 * J + q)) : 0u; }
+#else
+#define SHRED_MARK(q) if (TEST) { mA |= (uint32_t)is_marker(a.low(), c); mB |= (uint32_t)is_marker(b.low(), c); }
+#endif
     a.template step<0>(ina, popa, c); b.template step<0>(inb, popb, c);
-    if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + 0)) : 0u; mB |= is_marker(b.low(), c) ? (1u << (4 * J + 0)) : 0u; }
+    SHRED_MARK(0)
     a.template step<1>(ina, popa, c); b.template step<1>(inb, popb, c);
-    if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + 1)) : 0u; mB |= is_marker(b.low(), c) ? (1u << (4 * J + 1)) : 0u; }
+    SHRED_MARK(1)
     a.template step<2>(ina, popa, c); b.template step<2>(inb, popb, c);
-    if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + 2)) : 0u; mB |= is_marker(b.low(), c) ? (1u << (4 * J + 2)) : 0u; }
+    SHRED_MARK(2)
     a.template step<3>(ina, popa, c); b.template step<3>(inb, popb, c);
-    if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + 3)) : 0u; mB |= is_marker(b.low(), c) ? (1u << (4 * J + 3)) : 0u; }
+    SHRED_MARK(3)
+#undef SHRED_MARK
 }
 
 // 16 bytes of two chains in one basic block (ILP across the chains), then the rare emission.
@@ -374,6 +392,23 @@ __device__ __forceinline__ void chunk16x2(State<MODE> &a, const uint4 &da, const
     word4x2<MODE, TEST, 1>(a, da.y, pa.y, mA, b, db.y, pb.y, mB, c);
     word4x2<MODE, TEST, 2>(a, da.z, pa.z, mA, b, db.z, pb.z, mB, c);
     word4x2<MODE, TEST, 3>(a, da.w, pa.w, mA, b, db.w, pb.w, mB, c);
+}
+
+// Exact hit mask of one 16-byte chunk of one chain, recomputed from its entry state (the rare
+// path of SHRED_HITMODE 1).
+template <int MODE>
+__device__ __noinline__ uint32_t replay_mask(State<MODE> s, uint4 d, uint4 p, const BulkCtx &c) {
+    const uint32_t dw[4] = {d.x, d.y, d.z, d.w};
+    const uint32_t pw[4] = {p.x, p.y, p.z, p.w};
+    uint32_t m = 0;
+#pragma unroll
+    for (int j = 0; j < 4; ++j) {
+        s.template step<0>(dw[j], pw[j], c); m |= is_marker(s.low(), c) ? (1u << (4 * j + 0)) : 0u;
+        s.template step<1>(dw[j], pw[j], c); m |= is_marker(s.low(), c) ? (1u << (4 * j + 1)) : 0u;
+        s.template step<2>(dw[j], pw[j], c); m |= is_marker(s.low(), c) ? (1u << (4 * j + 2)) : 0u;
+        s.template step<3>(dw[j], pw[j], c); m |= is_marker(s.low(), c) ? (1u << (4 * j + 3)) : 0u;
+    }
+    return m;
 }
 
 struct BulkConst { uint32_t mhi, m256, tmul, rsh; };
@@ -516,18 +551,25 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
 
         const uint64_t pA = posA0 + (uint64_t)r * ROUND, pB = posB0 + (uint64_t)r * ROUND;
         uint32_t mA, mB;
-        chunk16x2<MODE, true>(sA, DA0, A1, sB, DB0, B1, c, mA, mB);
-        if (mA && actA) emit_mask(mA, pA + 0, J.min_i, J.c_limit, oA);
-        if (mB && actB) emit_mask(mB, pB + 0, J.min_i, J.c_limit, oB);
-        chunk16x2<MODE, true>(sA, DA1, A2, sB, DB1, B2, c, mA, mB);
-        if (mA && actA) emit_mask(mA, pA + 16, J.min_i, J.c_limit, oA);
-        if (mB && actB) emit_mask(mB, pB + 16, J.min_i, J.c_limit, oB);
-        chunk16x2<MODE, true>(sA, DA2, A3, sB, DB2, B3, c, mA, mB);
-        if (mA && actA) emit_mask(mA, pA + 32, J.min_i, J.c_limit, oA);
-        if (mB && actB) emit_mask(mB, pB + 32, J.min_i, J.c_limit, oB);
-        chunk16x2<MODE, true>(sA, DA3, DA0, sB, DB3, DB0, c, mA, mB);
-        if (mA && actA) emit_mask(mA, pA + 48, J.min_i, J.c_limit, oA);
-        if (mB && actB) emit_mask(mB, pB + 48, J.min_i, J.c_limit, oB);
+#if SHRED_HITMODE == 0
+#define SHRED_CHUNK(DA, PA, DB, PB, OFF)                                                   \
+        chunk16x2<MODE, true>(sA, DA, PA, sB, DB, PB, c, mA, mB);                         \
+        if (mA && actA) emit_mask(mA, pA + OFF, J.min_i, J.c_limit, oA);                  \
+        if (mB && actB) emit_mask(mB, pB + OFF, J.min_i, J.c_limit, oB);
+#else
+#define SHRED_CHUNK(DA, PA, DB, PB, OFF)                                                   \
+        {                                                                                  \
+            const State<MODE> a0 = sA, b0 = sB;                                            \
+            chunk16x2<MODE, true>(sA, DA, PA, sB, DB, PB, c, mA, mB);                     \
+            if (mA && actA) emit_mask(replay_mask<MODE>(a0, DA, PA, c), pA + OFF, J.min_i, J.c_limit, oA); \
+            if (mB && actB) emit_mask(replay_mask<MODE>(b0, DB, PB, c), pB + OFF, J.min_i, J.c_limit, oB); \
+        }
+#endif
+        SHRED_CHUNK(DA0, A1, DB0, B1, 0)
+        SHRED_CHUNK(DA1, A2, DB1, B2, 16)
+        SHRED_CHUNK(DA2, A3, DB2, B3, 32)
+        SHRED_CHUNK(DA3, DA0, DB3, DB0, 48)
+#undef SHRED_CHUNK
         A1 = DA1; A2 = DA2; A3 = DA3; B1 = DB1; B2 = DB2; B3 = DB3;
     }
     uint32_t totA, totB;

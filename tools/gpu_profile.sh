@@ -14,3 +14,7 @@ ncu --metrics gpu__time_duration.sum --clock-control none -c 400 --csv --log-fil
 ncu --set full --clock-control none --import-source on -k regex:k1_bulk -s 3 -c 1 -o gpurun_out/prof_k1_$TAG \
     python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu --no-extra > gpurun_out/ncu_full_$TAG.log 2>&1
 tail -2 gpurun_out/ncu_full_$TAG.log
+if [ "$3" == "k32" ]; then
+  ncu --set full --clock-control none --import-source on -k regex:k1_bulk -s 3 -c 1 -o gpurun_out/prof_k1k32_$TAG \
+      python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu --no-extra --variant k32 > /dev/null 2>&1
+fi
