@@ -693,19 +693,39 @@ int shred_feed(shred_ctx *ctx, const void *in, uint64_t len, uint64_t *d_out, ui
             if ((rc = feed_device_piece(ctx, (const uint8_t *)in, len, d_out, cap, st))) return rc;
         } else {
             if ((rc = ensure_ring(ctx))) return rc;
+            // Pieces of <= one slot.  The H2D copy of piece p+ring-1 is enqueued on the copy
+            // stream before piece p is processed, so transfers overlap the chunking (also in
+            // bounded mode, whose piece processing synchronises once on the candidate count).
             const uint8_t *h = (const uint8_t *)in;
-            for (uint64_t off = 0; off < len; off += ctx->ring_bytes) {
+            const uint64_t npieces = (len + ctx->ring_bytes - 1) / ctx->ring_bytes;
+            const int R = ctx->ring_n;
+            auto slot_of = [&](uint64_t q) { return (int)((ctx->ring_next + q) % (uint64_t)R); };
+            auto issue_copy = [&](uint64_t q) -> int {
+                const uint64_t off = q * ctx->ring_bytes;
                 const uint64_t n = (len - off) < ctx->ring_bytes ? (len - off) : ctx->ring_bytes;
-                const int s = ctx->ring_next;
-                ctx->ring_next = (s + 1) % ctx->ring_n;
-                // slot s is free once the compute stream finished its previous piece
-                CK(cudaStreamWaitEvent(ctx->copy_stream, ctx->ev_free[s], 0), "wait slot free");
-                CK(cudaMemcpyAsync(ctx->ring[s], h + off, n, cudaMemcpyHostToDevice, ctx->copy_stream), "H2D");
-                CK(cudaEventRecord(ctx->ev_ready[s], ctx->copy_stream), "record ready");
-                CK(cudaStreamWaitEvent(st, ctx->ev_ready[s], 0), "wait ready");
-                if ((rc = feed_device_piece(ctx, ctx->ring[s], n, d_out, cap, st))) return rc;
-                CK(cudaEventRecord(ctx->ev_free[s], st), "record free");
+                const int sl = slot_of(q);
+                CK(cudaStreamWaitEvent(ctx->copy_stream, ctx->ev_free[sl], 0), "wait slot free");
+                CK(cudaMemcpyAsync(ctx->ring[sl], h + off, n, cudaMemcpyHostToDevice, ctx->copy_stream), "H2D");
+                CK(cudaEventRecord(ctx->ev_ready[sl], ctx->copy_stream), "record ready");
+                return SHRED_OK;
+            };
+            uint64_t issued = 0;
+            for (; issued < npieces && issued < (uint64_t)(R > 1 ? R - 1 : 1); ++issued)
+                if ((rc = issue_copy(issued))) return rc;
+            for (uint64_t q = 0; q < npieces; ++q) {
+                if (R > 1 && issued < npieces && issued <= q + (uint64_t)(R - 1)) {
+                    if ((rc = issue_copy(issued))) return rc;
+                    ++issued;
+                }
+                const uint64_t off = q * ctx->ring_bytes;
+                const uint64_t n = (len - off) < ctx->ring_bytes ? (len - off) : ctx->ring_bytes;
+                const int sl = slot_of(q);
+                CK(cudaStreamWaitEvent(st, ctx->ev_ready[sl], 0), "wait ready");
+                if ((rc = feed_device_piece(ctx, ctx->ring[sl], n, d_out, cap, st))) return rc;
+                CK(cudaEventRecord(ctx->ev_free[sl], st), "record free");
+                if (R == 1 && issued < npieces) { if ((rc = issue_copy(issued))) return rc; ++issued; }
             }
+            ctx->ring_next = slot_of(npieces);
         }
     }
     k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, ctx->d_flag);

@@ -14,7 +14,8 @@
 //   sb_check  block b runs from e_b = spec exit of block b-1 in lockstep with its speculation
 //             until the two states coincide (sync) -> count delta; no sync -> not ok.
 //   sb_plan   one CTA: if every block synced, entries = spec exits and the offsets are a scan
-//             of the counts; otherwise thread 0 walks the unsynced blocks sequentially (exact).
+//             of the counts; otherwise warp 0 walks the blocks in order, re-walking the ones
+//             whose assumed entry does not hold (exact; serial only through those blocks).
 //   sb_emit   every block re-runs from its true entry and writes its cuts at its offset; one
 //             extra thread writes the forced cuts after the last candidate.
 // Streaming: `fin` = 1 for a whole stream (cuts < end = N); fin = 0 for a fed piece: an accepted
@@ -25,7 +26,7 @@
 
 namespace shred {
 
-constexpr int SB_B = 256;           // candidates per block
+constexpr int SB_B = 32;            // candidates per block (one thread; prefetched into registers)
 constexpr int SB_THREADS = 128;
 
 struct SBArgs {
@@ -75,10 +76,15 @@ __global__ void __launch_bounds__(SB_THREADS) sb_spec(SBArgs A) {
     const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
     if (b >= nb) return;
     const uint64_t first = b * SB_B, last = min(n, first + SB_B);
+    uint64_t v[SB_B];
+#pragma unroll
+    for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
     uint64_t s = b ? A.cand[first - 1] : A.aux->s;
     uint64_t cnt = 0;
     int held = 0;
-    for (uint64_t k = first; k < last; ++k) cnt += sb_step(s, A.cand[k], A, held, NoEmit{});
+#pragma unroll
+    for (int j = 0; j < SB_B; ++j)
+        if (first + j < last) cnt += sb_step(s, v[j], A, held, NoEmit{});
     A.spec_exit[b] = s;
     A.spec_cnt[b] = cnt;
 }
@@ -94,11 +100,16 @@ __global__ void __launch_bounds__(SB_THREADS) sb_check(SBArgs A) {
     int64_t c1 = 0, c2 = 0;
     int h1 = 0, h2 = 0;
     uint32_t ok = (s1 == s2);
-    for (uint64_t k = first; k < last && !ok; ++k) {
-        const uint64_t c = A.cand[k];
-        c1 += (int64_t)sb_step(s1, c, A, h1, NoEmit{});
-        c2 += (int64_t)sb_step(s2, c, A, h2, NoEmit{});
-        ok = (s1 == s2) && (h1 == h2);
+    uint64_t v[SB_B];
+#pragma unroll
+    for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
+#pragma unroll
+    for (int j = 0; j < SB_B; ++j) {
+        if (first + j < last && !ok) {
+            c1 += (int64_t)sb_step(s1, v[j], A, h1, NoEmit{});
+            c2 += (int64_t)sb_step(s2, v[j], A, h2, NoEmit{});
+            ok = (s1 == s2) && (h1 == h2);
+        }
     }
     A.ok[b] = ok;
     A.delta[b] = c1 - c2;
@@ -162,23 +173,31 @@ __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
         }
         return;
     }
-    if (tid != 0) return;
-    // ---- sequential fallback (blocks that never synced with their speculation): exact
+    if (tid >= 32) return;
+    // ---- sequential fallback (some block never synced with its speculation): exact.  Warp 0
+    // walks the blocks in order; a block whose assumed entry holds uses its (spec + delta)
+    // count, any other block is re-walked with its 32 candidates loaded one per lane.
+    const uint32_t lane = tid;
     uint64_t s = aux->s, off = base0;
     int held = 0;
     for (uint32_t b = 0; b < nb; ++b) {
         const uint64_t first = (uint64_t)b * SB_B, last = min(n, first + SB_B);
-        A.entry[b] = s;
-        A.offs[b] = off;
+        if (lane == 0) { A.entry[b] = s; A.offs[b] = off; }
         if (b == 0 || (A.ok[b] && s == A.spec_exit[b - 1])) {
             off += (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]);
             s = A.spec_exit[b];
             held = (!A.fin && last == n && A.cand[n - 1] == A.end && s == A.end) ? 1 : 0;
         } else {
             held = 0;
-            for (uint64_t k = first; k < last; ++k) off += sb_step(s, A.cand[k], A, held, NoEmit{});
+            const uint64_t mine = (first + lane < last) ? A.cand[first + lane] : 0ull;
+            const int m = (int)(last - first);
+            for (int j = 0; j < m; ++j) {
+                const uint64_t c = __shfl_sync(0xffffffffu, mine, j);
+                off += sb_step(s, c, A, held, NoEmit{});
+            }
         }
     }
+    if (lane != 0) return;
     const uint64_t mt = sb_tail_count(s, A);
     if (held_prev && aux->out_pos < A.dst_cap) A.dst[aux->out_pos] = aux->held_val;
     A.offs[nb] = off;
@@ -207,8 +226,13 @@ __global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
         return;
     }
     const uint64_t first = b * SB_B, last = min(n, first + SB_B);
+    uint64_t v[SB_B];
+#pragma unroll
+    for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
     int held = 0;
-    for (uint64_t k = first; k < last; ++k) sb_step(s, A.cand[k], A, held, emit);
+#pragma unroll
+    for (int j = 0; j < SB_B; ++j)
+        if (first + j < last) sb_step(s, v[j], A, held, emit);
 }
 
 }  // namespace shred
