@@ -31,6 +31,9 @@
 #ifndef SHRED_PUSHHI_FMA
 #define SHRED_PUSHHI_FMA 0      // 1: f_hi shift-in as IMAD.HI + IMAD (FMA pipe) instead of PRMT
 #endif
+#ifndef SHRED_PRODUCER_SLEEP_NS
+#define SHRED_PRODUCER_SLEEP_NS 512
+#endif
 #ifndef SHRED_HITMODE
 #define SHRED_HITMODE 0         // 0: per-byte hit bitmask; 1: chunk predicate + exact replay on hit
 #endif
@@ -147,6 +150,21 @@ __device__ __forceinline__ void mbar_wait(uint32_t bar, uint32_t parity) {
                  "bra LAB_WAIT;\n"
                  "DONE:\n"
                  "}\n" :: "r"(bar), "r"(parity) : "memory");
+}
+__device__ __forceinline__ bool mbar_try_wait(uint32_t bar, uint32_t parity) {
+    uint32_t ok;
+    asm volatile("{\n"
+                 ".reg .pred P1;\n"
+                 "mbarrier.try_wait.parity.shared::cta.b64 P1, [%1], %2;\n"
+                 "selp.u32 %0, 1, 0, P1;\n"
+                 "}\n" : "=r"(ok) : "r"(bar), "r"(parity) : "memory");
+    return ok != 0;
+}
+// Producer-side wait: back off with nanosleep so the spinning warp does not steal issue slots
+// from the consumer warps of its SM sub-partition (ncu r01: the spin was ~12% of all issued
+// instructions).
+__device__ __forceinline__ void mbar_wait_sleep(uint32_t bar, uint32_t parity) {
+    while (!mbar_try_wait(bar, parity)) __nanosleep(SHRED_PRODUCER_SLEEP_NS);
 }
 __device__ __forceinline__ void tma_load_2d(uint32_t dst, const CUtensorMap *map, int x, int y,
                                             uint32_t bar) {
@@ -288,6 +306,8 @@ struct BulkCtx {
     uint32_t m256;      // 256 (row stride of the table image)
     uint32_t tmul;      // 2^(32-m): (f_lo * tmul) keeps the low m bits at the top
     uint32_t rsh;       // r << (32-m)
+    uint32_t one;       // 1 (runtime, keeps IMAD.WIDE on the FMA pipe in SHRED_HITMODE 2)
+    uint32_t two;       // 2 (runtime, shift-accumulate of the hit bits by IMAD)
 };
 
 // One byte step, K63 (deg P = 63, fully reduced u64 state f = fh:fl, f < 2^63):
@@ -341,6 +361,13 @@ template <> struct State<MODE_K32> {
 
 // marker test: (f mod D) == r  <=>  (f_lo << (32-m)) == (r << (32-m))   (D = 2^m <= 2^32)
 __device__ __forceinline__ bool is_marker(uint32_t lo, const BulkCtx &c) { return lo * c.tmul == c.rsh; }
+// FMA-pipe form: 1 if NOT a marker.  y = (f_lo << (32-m)) - (r << (32-m)) is 0 iff marker;
+// hi32(y * 1 + 0xFFFFFFFF) = (y != 0).
+__device__ __forceinline__ uint32_t not_marker(uint32_t lo, const BulkCtx &c) {
+    const uint32_t y = lo * c.tmul - c.rsh;
+    const uint64_t w = (uint64_t)y * (uint64_t)c.one + 0xFFFFFFFFull;
+    return (uint32_t)(w >> 32);
+}
 
 struct SlotOut {
     uint64_t *lst; uint32_t cnt; uint32_t cap;
@@ -368,6 +395,9 @@ __device__ __forceinline__ void word4x2(State<MODE> &a, uint32_t ina, uint32_t p
 #if SHRED_HITMODE == 0
 #define SHRED_MARK(q) if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + q)) : 0u; \
                                   mB |= is_marker(b.low(), c) ? (1u << (4 * J + q)) : 0u; }
+#elif SHRED_HITMODE == 2
+#define SHRED_MARK(q) if (TEST) { mA = mA * c.two + not_marker(a.low(), c); \
+                                  mB = mB * c.two + not_marker(b.low(), c); }
 #else
 #define SHRED_MARK(q) if (TEST) { mA |= (uint32_t)is_marker(a.low(), c); mB |= (uint32_t)is_marker(b.low(), c); }
 #endif
@@ -392,6 +422,10 @@ __device__ __forceinline__ void chunk16x2(State<MODE> &a, const uint4 &da, const
     word4x2<MODE, TEST, 1>(a, da.y, pa.y, mA, b, db.y, pb.y, mB, c);
     word4x2<MODE, TEST, 2>(a, da.z, pa.z, mA, b, db.z, pb.z, mB, c);
     word4x2<MODE, TEST, 3>(a, da.w, pa.w, mA, b, db.w, pb.w, mB, c);
+#if SHRED_HITMODE == 2
+    // bit 15-j of mA = "position j is not a marker" -> bit j = "position j is a marker"
+    if (TEST) { mA = __brev(~mA) >> 16; mB = __brev(~mB) >> 16; }
+#endif
 }
 
 // Exact hit mask of one 16-byte chunk of one chain, recomputed from its entry state (the rare
@@ -411,7 +445,7 @@ __device__ __noinline__ uint32_t replay_mask(State<MODE> s, uint4 d, uint4 p, co
     return m;
 }
 
-struct BulkConst { uint32_t mhi, m256, tmul, rsh; };
+struct BulkConst { uint32_t mhi, m256, tmul, rsh, one; };
 
 // The hot kernel.  blockDim = NT consumers + 1 producer warp; one CTA per SM.
 // blockIdx < nc: bulk CTA, rows blockIdx*ROWS_CTA + {tid, tid + NT}; blockIdx == nc: edge CTA.
@@ -472,7 +506,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         if (tid == NT) {
             for (uint32_t r = 0; r < nrounds; ++r) {
                 const uint32_t s = r % STAGES;
-                if (r >= STAGES) mbar_wait(bars + 64 + 8 * s, ((r / STAGES) - 1u) & 1u);
+                if (r >= STAGES) mbar_wait_sleep(bars + 64 + 8 * s, ((r / STAGES) - 1u) & 1u);
                 mbar_expect_tx(bars + 8 * s, STAGE_BYTES);
                 const uint32_t dst = stages + s * STAGE_BYTES;
 #pragma unroll
@@ -500,7 +534,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         c.laneT = sbase + (uint32_t)lane * 4u;
         c.laneU = 128u + (uint32_t)lane * 4u;
     }
-    c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh;
+    c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh; c.one = K.one; c.two = 2u * K.one;
     SlotOut oA, oB;
     const uint32_t slotA = J.map.n_head + rowA, slotB = J.map.n_head + rowB;
     oA.lst = J.scratch + (uint64_t)slotA * J.cap; oA.cnt = 0; oA.cap = J.cap;

@@ -294,6 +294,7 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         K.m256 = 256u;
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
+        K.one = 1u;
         if (ctx->path == SHRED_PATH_K63)
             k1_bulk<MODE_K63><<<pl.bulk_ctas, NT + 32, BULK_SMEM, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen,
                                                                         pl.J, ctx->dp, K);
