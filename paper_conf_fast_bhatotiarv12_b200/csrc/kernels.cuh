@@ -42,27 +42,51 @@ namespace shred {
 
 enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3 };
 
-constexpr int NT          = 512;               // consumer threads per CTA
-constexpr int CHAINS      = 2;                 // rows (independent fingerprint chains) per thread
-constexpr int ROWS_CTA    = NT * CHAINS;       // rows per bulk CTA
-constexpr int ROUND       = 64 / CHAINS;       // bytes per row per pipeline round
 constexpr int STAGES      = 4;                 // TMA ring depth
 constexpr int BOX_ROWS    = 256;               // rows per TMA box (hardware max 256)
 constexpr int TAB_BYTES   = 65536;             // replicated T|U image (256 rows x 256 B)
-constexpr int STAGE_BYTES = ROWS_CTA * ROUND;  // 32 KiB
-constexpr int BAR_OFFSET  = TAB_BYTES + STAGES * STAGE_BYTES;
-constexpr int BULK_SMEM   = BAR_OFFSET + 2048; // + barriers/scan scratch; + 1 KiB base alignment
 constexpr int GEN_THREADS = 256;
+
+// Launch shape of the hot kernel: CH rows (independent fingerprint chains) per consumer
+// thread, NTC consumer threads (+ 1 producer warp) per CTA, one CTA per SM.  A pipeline round
+// brings ROUND = 64/CH bytes of every row; 4 chunks of 16 B per row per loop iteration.
+template <int CH_, int NTC_>
+struct BulkCfg {
+    static constexpr int CH = CH_, NTC = NTC_;
+    static constexpr int ROWS = NTC * CH;                 // rows per bulk CTA
+    static constexpr int ROUND = 64 / CH;                 // bytes per row per round
+    static constexpr int CPR = ROUND / 16;                // 16-byte chunks per row per round
+    static constexpr int STAGE = ROWS * ROUND;            // bytes per TMA stage
+    static constexpr int BAR_OFF = TAB_BYTES + STAGES * STAGE;
+    static constexpr int SMEM = BAR_OFF + 2048;           // + barriers/scan scratch + 1 KiB align
+    static_assert(ROWS % BOX_ROWS == 0 && (CH == 1 || CH == 2 || CH == 4) && NTC % 32 == 0 &&
+                  NTC + 32 <= 1024, "shape");
+};
+#ifndef SHRED_K63_CH
+#define SHRED_K63_CH 2
+#endif
+#ifndef SHRED_K63_NT
+#define SHRED_K63_NT 512
+#endif
+#ifndef SHRED_K32_CH
+#define SHRED_K32_CH 2
+#endif
+#ifndef SHRED_K32_NT
+#define SHRED_K32_NT 512
+#endif
+using CfgK63 = BulkCfg<SHRED_K63_CH, SHRED_K63_NT>;
+using CfgK32 = BulkCfg<SHRED_K32_CH, SHRED_K32_NT>;
 
 // Slot id -> range of window-end positions.  Slots are numbered in stream order:
 // [0, n_head) generic head segments, then the bulk rows, then generic tail segments.
-// Slot groups (one group sum each): bulk mode: group 0 = head slots, 1 + r/ROWS_CTA = bulk rows,
+// Slot groups (one group sum each): bulk mode: group 0 = head slots, 1 + r/rows_cta = bulk rows,
 // nc + 1 = tail slots; generic-only mode (nrows == 0): group = slot / GEN_THREADS.
 struct SlotMap {
     uint64_t head_start; uint64_t head_seg; uint32_t n_head;
     uint32_t nrows;      uint64_t b0;       uint64_t S;
     uint64_t tail_start; uint64_t tail_seg; uint32_t n_tail;
     uint32_t nc;         uint32_t ngroups;  // bulk CTAs; number of groups
+    uint32_t rows_cta;   uint32_t pad;      // rows per bulk CTA
     uint64_t t_end;
 };
 
@@ -70,7 +94,7 @@ __host__ __device__ __forceinline__ uint32_t slot_group(const SlotMap &m, uint32
     if (m.nrows == 0) return slot / GEN_THREADS;
     if (slot < m.n_head) return 0;
     slot -= m.n_head;
-    if (slot < m.nrows) return 1 + slot / ROWS_CTA;
+    if (slot < m.nrows) return 1 + slot / m.rows_cta;
     return m.nc + 1;
 }
 
@@ -387,44 +411,70 @@ __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t min_i,
     }
 }
 
-// One word (4 bytes) of two interleaved chains; hit bits accumulate into mA / mB.
-template <int MODE, bool TEST, int J>
-__device__ __forceinline__ void word4x2(State<MODE> &a, uint32_t ina, uint32_t popa, uint32_t &mA,
-                                        State<MODE> &b, uint32_t inb, uint32_t popb, uint32_t &mB,
-                                        const BulkCtx &c) {
+// One word (4 bytes) of CH interleaved chains; hit bits accumulate into m[ch] (bit 4J+q).
 #if SHRED_HITMODE == 0
-#define SHRED_MARK(q) if (TEST) { mA |= is_marker(a.low(), c) ? (1u << (4 * J + q)) : 0u; \
-                                  mB |= is_marker(b.low(), c) ? (1u << (4 * J + q)) : 0u; }
+#define SHRED_MARK(ch, q) m[ch] |= is_marker(st[ch].low(), c) ? (1u << (4 * J + q)) : 0u;
 #elif SHRED_HITMODE == 2
-#define SHRED_MARK(q) if (TEST) { mA = mA * c.two + not_marker(a.low(), c); \
-                                  mB = mB * c.two + not_marker(b.low(), c); }
+#define SHRED_MARK(ch, q) m[ch] = m[ch] * c.two + not_marker(st[ch].low(), c);
 #else
-#define SHRED_MARK(q) if (TEST) { mA |= (uint32_t)is_marker(a.low(), c); mB |= (uint32_t)is_marker(b.low(), c); }
+#define SHRED_MARK(ch, q) m[ch] |= (uint32_t)is_marker(st[ch].low(), c);
 #endif
-    a.template step<0>(ina, popa, c); b.template step<0>(inb, popb, c);
-    SHRED_MARK(0)
-    a.template step<1>(ina, popa, c); b.template step<1>(inb, popb, c);
-    SHRED_MARK(1)
-    a.template step<2>(ina, popa, c); b.template step<2>(inb, popb, c);
-    SHRED_MARK(2)
-    a.template step<3>(ina, popa, c); b.template step<3>(inb, popb, c);
-    SHRED_MARK(3)
-#undef SHRED_MARK
+template <int MODE, int CH, bool TEST, int J>
+__device__ __forceinline__ void word4xN(State<MODE> (&st)[CH], const uint32_t (&in)[CH],
+                                        const uint32_t (&pop)[CH], uint32_t (&m)[CH], const BulkCtx &c) {
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) st[ch].template step<0>(in[ch], pop[ch], c);
+    if (TEST) {
+#pragma unroll
+        for (int ch = 0; ch < CH; ++ch) { SHRED_MARK(ch, 0) }
+    }
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) st[ch].template step<1>(in[ch], pop[ch], c);
+    if (TEST) {
+#pragma unroll
+        for (int ch = 0; ch < CH; ++ch) { SHRED_MARK(ch, 1) }
+    }
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) st[ch].template step<2>(in[ch], pop[ch], c);
+    if (TEST) {
+#pragma unroll
+        for (int ch = 0; ch < CH; ++ch) { SHRED_MARK(ch, 2) }
+    }
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) st[ch].template step<3>(in[ch], pop[ch], c);
+    if (TEST) {
+#pragma unroll
+        for (int ch = 0; ch < CH; ++ch) { SHRED_MARK(ch, 3) }
+    }
 }
+#undef SHRED_MARK
 
-// 16 bytes of two chains in one basic block (ILP across the chains), then the rare emission.
-template <int MODE, bool TEST>
-__device__ __forceinline__ void chunk16x2(State<MODE> &a, const uint4 &da, const uint4 &pa,
-                                          State<MODE> &b, const uint4 &db, const uint4 &pb,
-                                          const BulkCtx &c, uint32_t &mA, uint32_t &mB) {
-    mA = 0; mB = 0;
-    word4x2<MODE, TEST, 0>(a, da.x, pa.x, mA, b, db.x, pb.x, mB, c);
-    word4x2<MODE, TEST, 1>(a, da.y, pa.y, mA, b, db.y, pb.y, mB, c);
-    word4x2<MODE, TEST, 2>(a, da.z, pa.z, mA, b, db.z, pb.z, mB, c);
-    word4x2<MODE, TEST, 3>(a, da.w, pa.w, mA, b, db.w, pb.w, mB, c);
+// 16 bytes of CH chains in one basic block (ILP across the chains): d = data chunk,
+// p = the chunk 48 bytes earlier (its bytes leave the window).
+template <int MODE, int CH, bool TEST>
+__device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d)[CH], const uint4 (&p)[CH],
+                                          const BulkCtx &c, uint32_t (&m)[CH]) {
+    uint32_t in[CH], po[CH];
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) m[ch] = 0;
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].x; po[ch] = p[ch].x; }
+    word4xN<MODE, CH, TEST, 0>(st, in, po, m, c);
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].y; po[ch] = p[ch].y; }
+    word4xN<MODE, CH, TEST, 1>(st, in, po, m, c);
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].z; po[ch] = p[ch].z; }
+    word4xN<MODE, CH, TEST, 2>(st, in, po, m, c);
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].w; po[ch] = p[ch].w; }
+    word4xN<MODE, CH, TEST, 3>(st, in, po, m, c);
 #if SHRED_HITMODE == 2
-    // bit 15-j of mA = "position j is not a marker" -> bit j = "position j is a marker"
-    if (TEST) { mA = __brev(~mA) >> 16; mB = __brev(~mB) >> 16; }
+    // bit 15-j = "position j is not a marker" -> bit j = "position j is a marker"
+    if (TEST) {
+#pragma unroll
+        for (int ch = 0; ch < CH; ++ch) m[ch] = __brev(~m[ch]) >> 16;
+    }
 #endif
 }
 
@@ -447,25 +497,25 @@ __device__ __noinline__ uint32_t replay_mask(State<MODE> s, uint4 d, uint4 p, co
 
 struct BulkConst { uint32_t mhi, m256, tmul, rsh, one; };
 
-// The hot kernel.  blockDim = NT consumers + 1 producer warp; one CTA per SM.
-// blockIdx < nc: bulk CTA, rows blockIdx*ROWS_CTA + {tid, tid + NT}; blockIdx == nc: edge CTA.
-// Rounds of ROUND = 32 bytes per row arrive in a 4-stage TMA ring (SWIZZLE_32B: the 8 lanes
-// of a quarter warp read 8 consecutive rows' 16-byte chunks from 8 distinct bank groups).
-// The window is fixed at w = 48 = 3 chunks of 16 B: the byte leaving the window at chunk q is
-// the same byte slot of chunk q-3, kept in registers (R1..R3 = chunks 1..3 of the previous
-// pair of rounds).
-template <int MODE>
-__global__ void __launch_bounds__(NT + 32, 1)
+// The hot kernel.  blockDim = NTC consumers + 1 producer warp; one CTA per SM.
+// blockIdx < nc: bulk CTA, rows blockIdx*ROWS + tid + ch*NTC (ch < CH); blockIdx == nc: the
+// edge CTA.  Rounds of ROUND = 64/CH bytes per row arrive in a 4-stage TMA ring (the 8 lanes
+// of a quarter warp read 8 consecutive rows' 16-byte chunks from 8 distinct bank groups:
+// SWIZZLE_32B for 32-byte rounds, no swizzle for 16-byte rounds).  The window is fixed at
+// w = 48 = 3 chunks of 16 B: the byte leaving the window at chunk q is the same byte slot of
+// chunk q-3, kept in a 4-slot register ring per chain (slot = chunk index mod 4).
+template <int MODE, class C>
+__global__ void __launch_bounds__(C::NTC + 32, 1)
 k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_img,
         const GenTables *__restrict__ gt, Job J, DevParams P, BulkConst K) {
-    static_assert(CHAINS == 2 && ROUND == 32, "kernel written for 2 chains x 32-byte rounds");
+    constexpr int CH = C::CH, NTC = C::NTC, ROUND = C::ROUND, CPR = C::CPR;
     extern __shared__ uint8_t smem_raw[];
     // align the dynamic shared base to 1 KiB (the TMA swizzle pattern is address-based)
     uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
     const uint32_t sbase = smem_u32(smem);
     const uint32_t stages = sbase + TAB_BYTES;
-    const uint32_t bars = sbase + BAR_OFFSET;      // full[s] at +8s, empty[s] at +64+8s
-    uint32_t *ws = reinterpret_cast<uint32_t *>(smem + BAR_OFFSET + 128);
+    const uint32_t bars = sbase + C::BAR_OFF;      // full[s] at +8s, empty[s] at +64+8s
+    uint32_t *ws = reinterpret_cast<uint32_t *>(smem + C::BAR_OFF + 128);
     const int tid = threadIdx.x;
 
     if (blockIdx.x == J.map.nc) {                    // ---- edge CTA: head + tail, generic loop
@@ -473,14 +523,14 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         uint64_t *sU = sT + 256;
         for (int i = tid; i < 256; i += blockDim.x) { sT[i] = gt->T[i]; sU[i] = gt->U[i]; }
         __syncthreads();
-        if (tid >= NT) return;
+        if (tid >= NTC) return;
         SmemGenTab tab{sT, sU};
         const uint32_t tail0 = J.map.n_head + J.map.nrows;
         const uint32_t ch = (uint32_t)tid < J.map.n_head ? roll_slot(J, P, tab, tid) : 0u;
         const uint32_t ct = (uint32_t)tid < J.map.n_tail ? roll_slot(J, P, tab, tail0 + tid) : 0u;
         uint32_t th, tt;
-        const uint32_t oh = block_exscan(ch, NT, 1, ws, &th);
-        const uint32_t ot = block_exscan(ct, NT, 1, ws, &tt);
+        const uint32_t oh = block_exscan(ch, NTC, 1, ws, &th);
+        const uint32_t ot = block_exscan(ct, NTC, 1, ws, &tt);
         if ((uint32_t)tid < J.map.n_head) { J.counts[tid] = ch; J.local_off[tid] = oh; }
         if ((uint32_t)tid < J.map.n_tail) { J.counts[tail0 + tid] = ct; J.local_off[tail0 + tid] = ot; }
         if (tid == 0) { J.group_sum[0] = th; J.group_sum[J.map.nc + 1] = tt; }
@@ -492,25 +542,25 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     if (tid == 0) {
         for (int s = 0; s < STAGES; ++s) {
             mbar_init(bars + 8 * s, 1);
-            mbar_init(bars + 64 + 8 * s, NT / 32);
+            mbar_init(bars + 64 + 8 * s, NTC / 32);
         }
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
         asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
     }
     __syncthreads();
 
-    const uint32_t row0 = blockIdx.x * ROWS_CTA;
-    const uint32_t nrounds = (uint32_t)(J.map.S / ROUND);     // even (S is a multiple of 64)
+    const uint32_t row0 = blockIdx.x * C::ROWS;
+    const uint32_t nrounds = (uint32_t)(J.map.S / ROUND);     // a multiple of CH (S % 64 == 0)
 
-    if (tid >= NT) {                                 // ---- producer warp
-        if (tid == NT) {
+    if (tid >= NTC) {                                // ---- producer warp
+        if (tid == NTC) {
             for (uint32_t r = 0; r < nrounds; ++r) {
                 const uint32_t s = r % STAGES;
                 if (r >= STAGES) mbar_wait_sleep(bars + 64 + 8 * s, ((r / STAGES) - 1u) & 1u);
-                mbar_expect_tx(bars + 8 * s, STAGE_BYTES);
-                const uint32_t dst = stages + s * STAGE_BYTES;
+                mbar_expect_tx(bars + 8 * s, C::STAGE);
+                const uint32_t dst = stages + s * C::STAGE;
 #pragma unroll
-                for (int q = 0; q < ROWS_CTA / BOX_ROWS; ++q)
+                for (int q = 0; q < C::ROWS / BOX_ROWS; ++q)
                     tma_load_2d(dst + q * BOX_ROWS * ROUND, &tmap, (int)(r * ROUND), (int)(row0 + q * BOX_ROWS),
                                 bars + 8 * s);
             }
@@ -518,13 +568,8 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         return;
     }
 
-    // ---- consumers: thread tid owns rows rA = row0 + tid and rB = row0 + NT + tid
+    // ---- consumers: thread tid owns rows row0 + tid + ch*NTC
     const int lane = tid & 31;
-    const uint32_t rowA = row0 + tid, rowB = row0 + NT + tid;
-    const bool actA = rowA < J.map.nrows, actB = rowB < J.map.nrows;
-    const uint64_t posA0 = J.map.b0 + (uint64_t)rowA * J.map.S;
-    const uint64_t posB0 = J.map.b0 + (uint64_t)rowB * J.map.S;
-
     BulkCtx c;
     c.tab = sbase;
     if (MODE == MODE_K63) {
@@ -535,83 +580,99 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         c.laneU = 128u + (uint32_t)lane * 4u;
     }
     c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh; c.one = K.one; c.two = 2u * K.one;
-    SlotOut oA, oB;
-    const uint32_t slotA = J.map.n_head + rowA, slotB = J.map.n_head + rowB;
-    oA.lst = J.scratch + (uint64_t)slotA * J.cap; oA.cnt = 0; oA.cap = J.cap;
-    oB.lst = J.scratch + (uint64_t)slotB * J.cap; oB.cnt = 0; oB.cap = J.cap;
 
-    State<MODE> sA, sB;
-    uint4 A1 = make_uint4(0, 0, 0, 0), A2 = A1, A3 = A1, B1 = A1, B2 = A1, B3 = A1;
+    bool act[CH];
+    uint64_t pos0[CH];
+    SlotOut o[CH];
+    State<MODE> st[CH];
+    uint4 R[CH][4];                                   // ring: slot q = chunk index mod 4
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) {
+        const uint32_t row = row0 + tid + ch * NTC;
+        act[ch] = row < J.map.nrows;
+        pos0[ch] = J.map.b0 + (uint64_t)row * J.map.S;
+        o[ch].lst = J.scratch + (uint64_t)(J.map.n_head + row) * J.cap;
+        o[ch].cnt = 0; o[ch].cap = J.cap;
+    }
     {
         // warm-up: the 64 bytes before each row (b0 >= p_begin + 64 keeps them inside src)
         const uint4 Z = make_uint4(0, 0, 0, 0);
-        uint4 HA0 = Z, HA1 = Z, HA2 = Z, HA3 = Z, HB0 = Z, HB1 = Z, HB2 = Z, HB3 = Z;
-        if (actA) {
-            const uint4 *h = reinterpret_cast<const uint4 *>(J.src + (posA0 - 64u - J.p_begin));
-            HA0 = __ldg(h + 0); HA1 = __ldg(h + 1); HA2 = __ldg(h + 2); HA3 = __ldg(h + 3);
+#pragma unroll
+        for (int ch = 0; ch < CH; ++ch) {
+#pragma unroll
+            for (int q = 0; q < 4; ++q) R[ch][q] = Z;
+            if (act[ch]) {
+                const uint4 *h = reinterpret_cast<const uint4 *>(J.src + (pos0[ch] - 64u - J.p_begin));
+#pragma unroll
+                for (int q = 0; q < 4; ++q) R[ch][q] = __ldg(h + q);
+            }
         }
-        if (actB) {
-            const uint4 *h = reinterpret_cast<const uint4 *>(J.src + (posB0 - 64u - J.p_begin));
-            HB0 = __ldg(h + 0); HB1 = __ldg(h + 1); HB2 = __ldg(h + 2); HB3 = __ldg(h + 3);
+        uint32_t m[CH];
+#pragma unroll
+        for (int q = 0; q < 4; ++q) {
+            uint4 d[CH], p[CH];
+#pragma unroll
+            for (int ch = 0; ch < CH; ++ch) { d[ch] = R[ch][q]; p[ch] = (q == 3) ? R[ch][0] : Z; }
+            chunk16xN<MODE, CH, false>(st, d, p, c, m);
         }
-        uint32_t mA, mB;
-        chunk16x2<MODE, false>(sA, HA0, Z, sB, HB0, Z, c, mA, mB);
-        chunk16x2<MODE, false>(sA, HA1, Z, sB, HB1, Z, c, mA, mB);
-        chunk16x2<MODE, false>(sA, HA2, Z, sB, HB2, Z, c, mA, mB);
-        chunk16x2<MODE, false>(sA, HA3, HA0, sB, HB3, HB0, c, mA, mB);
-        A1 = HA1; A2 = HA2; A3 = HA3; B1 = HB1; B2 = HB2; B3 = HB3;
     }
 
-    const uint32_t swz = ((uint32_t)tid >> 2) & 1u;         // SWIZZLE_32B: chunk ^= (row >> 2) & 1
-    const uint32_t offA = (uint32_t)tid * ROUND, offB = (uint32_t)(NT + tid) * ROUND;
-    for (uint32_t r = 0; r < nrounds; r += 2) {
-        const uint32_t s0 = r % STAGES, s1 = (r + 1) % STAGES;
-        mbar_wait(bars + 8 * s0, (r / STAGES) & 1u);
-        const uint32_t b0s = stages + s0 * STAGE_BYTES;
-        const uint4 DA0 = lds128(b0s + offA + ((0u ^ swz) << 4));
-        const uint4 DA1 = lds128(b0s + offA + ((1u ^ swz) << 4));
-        const uint4 DB0 = lds128(b0s + offB + ((0u ^ swz) << 4));
-        const uint4 DB1 = lds128(b0s + offB + ((1u ^ swz) << 4));
-        __syncwarp();
-        if (lane == 0) mbar_arrive(bars + 64 + 8 * s0);
-        mbar_wait(bars + 8 * s1, ((r + 1) / STAGES) & 1u);
-        const uint32_t b1s = stages + s1 * STAGE_BYTES;
-        const uint4 DA2 = lds128(b1s + offA + ((0u ^ swz) << 4));
-        const uint4 DA3 = lds128(b1s + offA + ((1u ^ swz) << 4));
-        const uint4 DB2 = lds128(b1s + offB + ((0u ^ swz) << 4));
-        const uint4 DB3 = lds128(b1s + offB + ((1u ^ swz) << 4));
-        __syncwarp();
-        if (lane == 0) mbar_arrive(bars + 64 + 8 * s1);
-
-        const uint64_t pA = posA0 + (uint64_t)r * ROUND, pB = posB0 + (uint64_t)r * ROUND;
-        uint32_t mA, mB;
-#if SHRED_HITMODE == 0
-#define SHRED_CHUNK(DA, PA, DB, PB, OFF)                                                   \
-        chunk16x2<MODE, true>(sA, DA, PA, sB, DB, PB, c, mA, mB);                         \
-        if (mA && actA) emit_mask(mA, pA + OFF, J.min_i, J.c_limit, oA);                  \
-        if (mB && actB) emit_mask(mB, pB + OFF, J.min_i, J.c_limit, oB);
-#else
-#define SHRED_CHUNK(DA, PA, DB, PB, OFF)                                                   \
-        {                                                                                  \
-            const State<MODE> a0 = sA, b0 = sB;                                            \
-            chunk16x2<MODE, true>(sA, DA, PA, sB, DB, PB, c, mA, mB);                     \
-            if (mA && actA) emit_mask(replay_mask<MODE>(a0, DA, PA, c), pA + OFF, J.min_i, J.c_limit, oA); \
-            if (mB && actB) emit_mask(replay_mask<MODE>(b0, DB, PB, c), pB + OFF, J.min_i, J.c_limit, oB); \
-        }
+    // TMA swizzle of the 16-byte chunk index (rows of ROUND bytes; tid + ch*NTC has the same
+    // low bits as tid): SWIZZLE_64B: ^ (row >> 1) & 3, SWIZZLE_32B: ^ (row >> 2) & 1, 16 B: none
+    const uint32_t swz = (ROUND == 64) ? (((uint32_t)tid >> 1) & 3u)
+                       : (ROUND == 32) ? (((uint32_t)tid >> 2) & 1u) : 0u;
+    for (uint32_t r = 0; r < nrounds; r += CH) {
+#pragma unroll
+        for (int qr = 0; qr < CH; ++qr) {             // round r + qr: chunks qr*CPR .. +CPR-1
+            const uint32_t s = (r + qr) % STAGES;
+            mbar_wait(bars + 8 * s, ((r + qr) / STAGES) & 1u);
+            const uint32_t sb = stages + s * C::STAGE;
+            uint4 D[CH][CPR];
+#pragma unroll
+            for (int ch = 0; ch < CH; ++ch)
+#pragma unroll
+                for (int u = 0; u < CPR; ++u)
+                    D[ch][u] = lds128(sb + (uint32_t)(tid + ch * NTC) * ROUND + (((uint32_t)u ^ swz) << 4));
+            __syncwarp();
+            if (lane == 0) mbar_arrive(bars + 64 + 8 * s);
+#pragma unroll
+            for (int u = 0; u < CPR; ++u) {
+                const int cq = qr * CPR + u;          // chunk index mod 4 (compile time)
+                uint4 d[CH], p[CH];
+                uint32_t m[CH];
+#pragma unroll
+                for (int ch = 0; ch < CH; ++ch) { d[ch] = D[ch][u]; p[ch] = R[ch][(cq + 1) & 3]; }
+#if SHRED_HITMODE == 1
+                State<MODE> s0[CH];
+#pragma unroll
+                for (int ch = 0; ch < CH; ++ch) s0[ch] = st[ch];
 #endif
-        SHRED_CHUNK(DA0, A1, DB0, B1, 0)
-        SHRED_CHUNK(DA1, A2, DB1, B2, 16)
-        SHRED_CHUNK(DA2, A3, DB2, B3, 32)
-        SHRED_CHUNK(DA3, DA0, DB3, DB0, 48)
-#undef SHRED_CHUNK
-        A1 = DA1; A2 = DA2; A3 = DA3; B1 = DB1; B2 = DB2; B3 = DB3;
+                chunk16xN<MODE, CH, true>(st, d, p, c, m);
+#pragma unroll
+                for (int ch = 0; ch < CH; ++ch) {
+                    R[ch][cq] = D[ch][u];
+#if SHRED_HITMODE == 1
+                    if (m[ch] && act[ch]) m[ch] = replay_mask<MODE>(s0[ch], d[ch], p[ch], c);
+#endif
+                    if (m[ch] && act[ch])
+                        emit_mask(m[ch], pos0[ch] + (uint64_t)(r + qr) * ROUND + 16u * u, J.min_i, J.c_limit, o[ch]);
+                }
+            }
+        }
     }
-    uint32_t totA, totB;
-    const uint32_t offsA = block_exscan(actA ? oA.cnt : 0u, NT, 1, ws, &totA);
-    const uint32_t offsB = block_exscan(actB ? oB.cnt : 0u, NT, 1, ws, &totB);
-    if (actA) { J.counts[slotA] = oA.cnt; J.local_off[slotA] = offsA; }
-    if (actB) { J.counts[slotB] = oB.cnt; J.local_off[slotB] = totA + offsB; }
-    if (tid == 0) J.group_sum[1 + blockIdx.x] = totA + totB;
+    uint32_t base = 0;
+#pragma unroll
+    for (int ch = 0; ch < CH; ++ch) {
+        uint32_t tot;
+        const uint32_t off = block_exscan(act[ch] ? o[ch].cnt : 0u, NTC, 1, ws, &tot);
+        if (act[ch]) {
+            const uint32_t slot = J.map.n_head + row0 + tid + ch * NTC;
+            J.counts[slot] = o[ch].cnt;
+            J.local_off[slot] = base + off;
+        }
+        base += tot;
+    }
+    if (tid == 0) J.group_sum[1 + blockIdx.x] = base;
 }
 
 // ------------------------------------------------------------------------------ k_total

@@ -196,6 +196,10 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
     const uint64_t GS = 64;                    // head/tail segment (edge CTA)
 
     // bulk region: aligned start b0 >= max(t_begin, p_begin + 64), rows of S bytes
+    const bool k63 = ctx->path == SHRED_PATH_K63;
+    const uint64_t ROWS_CTA = k63 ? CfgK63::ROWS : CfgK32::ROWS;
+    const uint64_t NTC = k63 ? CfgK63::NTC : CfgK32::NTC;
+    const uint64_t ROUND = k63 ? CfgK63::ROUND : CfgK32::ROUND;
     pl.bulk = false;
     uint64_t S = 0, nrows = 0, b0 = t_end;
     if ((ctx->path == SHRED_PATH_K63 || ctx->path == SHRED_PATH_K32) && len >= 4096) {
@@ -210,7 +214,7 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
             S = (S + 63) / 64 * 64;                // an even number of ROUND-byte rounds
             if (S < 256) S = 256;
             nrows = blen / S;
-            if (nrows > 0 && nrows < (1ull << 31) && S < (1ull << 39) && (b0 - t_begin) <= GS * NT)
+            if (nrows > 0 && nrows < (1ull << 31) && S < (1ull << 39) && (b0 - t_begin) <= GS * NTC)
                 pl.bulk = true;
         }
     }
@@ -231,11 +235,12 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
         m.b0 = b0; m.S = S; m.nrows = (uint32_t)nrows;
         m.tail_start = b0 + nrows * S;
         const uint64_t tl = t_end - m.tail_start;
-        uint64_t ts = (tl + NT - 1) / NT;
+        uint64_t ts = (tl + NTC - 1) / NTC;
         ts = ts < GS ? GS : (ts + 15) / 16 * 16;
         m.tail_seg = ts;
         m.n_tail = (uint32_t)((tl + ts - 1) / ts);
         m.nc = (uint32_t)((nrows + ROWS_CTA - 1) / ROWS_CTA);
+        m.rows_cta = (uint32_t)ROWS_CTA;
         m.ngroups = m.nc + 2;
         pl.bulk_ctas = m.nc + 1;               // + the edge CTA (head + tail, group sums 0, nc+1)
         // 2-D tensor map [nrows][S] over the bulk bytes
@@ -246,7 +251,8 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
         CUresult r = ctx->encode(&pl.tmap, CU_TENSOR_MAP_DATA_TYPE_UINT8, 2,
                                  (void *)(src + (b0 - p_begin)), gdim, gstride, box, estr,
                                  CU_TENSOR_MAP_INTERLEAVE_NONE,
-                                 ROUND == 64 ? CU_TENSOR_MAP_SWIZZLE_64B : CU_TENSOR_MAP_SWIZZLE_32B,
+                                 ROUND == 64 ? CU_TENSOR_MAP_SWIZZLE_64B
+                                             : (ROUND == 32 ? CU_TENSOR_MAP_SWIZZLE_32B : CU_TENSOR_MAP_SWIZZLE_NONE),
                                  CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
         if (r != CUDA_SUCCESS) return fail(ctx, SHRED_ECUDA, "cuTensorMapEncodeTiled failed (%d)", (int)r);
     }
@@ -296,11 +302,11 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         K.rsh = (uint32_t)(ctx->p.magic << m);
         K.one = 1u;
         if (ctx->path == SHRED_PATH_K63)
-            k1_bulk<MODE_K63><<<pl.bulk_ctas, NT + 32, BULK_SMEM, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen,
-                                                                        pl.J, ctx->dp, K);
+            k1_bulk<MODE_K63, CfgK63><<<pl.bulk_ctas, CfgK63::NTC + 32, CfgK63::SMEM, st>>>(
+                pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
         else
-            k1_bulk<MODE_K32><<<pl.bulk_ctas, NT + 32, BULK_SMEM, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen,
-                                                                        pl.J, ctx->dp, K);
+            k1_bulk<MODE_K32, CfgK32><<<pl.bulk_ctas, CfgK32::NTC + 32, CfgK32::SMEM, st>>>(
+                pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
         LAUNCHED("k1_bulk");
         if (e1) CK(cudaEventRecord(e1, st), "profile record");
     } else {
@@ -533,8 +539,8 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fn, cudaEnableDefault, &q) != cudaSuccess || !fn)
             return bail(SHRED_ECUDA);
         ctx->encode = (EncodeTiledFn)fn;
-        if (cudaFuncSetAttribute(k1_bulk<MODE_K63>, cudaFuncAttributeMaxDynamicSharedMemorySize, BULK_SMEM) != cudaSuccess ||
-            cudaFuncSetAttribute(k1_bulk<MODE_K32>, cudaFuncAttributeMaxDynamicSharedMemorySize, BULK_SMEM) != cudaSuccess)
+        if (cudaFuncSetAttribute(k1_bulk<MODE_K63, CfgK63>, cudaFuncAttributeMaxDynamicSharedMemorySize, CfgK63::SMEM) != cudaSuccess ||
+            cudaFuncSetAttribute(k1_bulk<MODE_K32, CfgK32>, cudaFuncAttributeMaxDynamicSharedMemorySize, CfgK32::SMEM) != cudaSuccess)
             return bail(SHRED_ECUDA);
     }
     if (cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking) != cudaSuccess)

@@ -2,7 +2,7 @@
 # A/B the compile-time variants of libshred (built in-tree as libshred_<name>.so): a parity
 # smoke per variant, then the hot-kernel rate for the paper params and the k32 variant.
 mkdir -p gpurun_out
-for v in "" _v_fmahi _v_replay _v_both "$@"; do
+for v in "" "$@"; do
   export SHRED_LIB=$PWD/paper_conf_fast_bhatotiarv12_b200/libshred$v.so
   [ -f "$SHRED_LIB" ] || continue
   echo "== variant '${v:-base}'"
