@@ -1,0 +1,50 @@
+"""Small cases of every kernel path, for compute-sanitizer (memcheck / racecheck / synccheck).
+Checks results against the oracle too, so a silent corruption under the tool is caught."""
+import os
+import sys
+
+import numpy as np
+import torch
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+
+import oracle  # noqa: E402
+import synthgen  # noqa: E402
+import paper_conf_fast_bhatotiarv12_b200 as pkg  # noqa: E402
+
+
+def check(ch, data, off=0):
+    buf = torch.zeros(data.size + off + 64, dtype=torch.uint8, device="cuda")
+    x = buf[off:off + data.size]
+    x.copy_(torch.from_numpy(data))
+    got = ch.chunk(x).cpu().numpy().astype(np.uint64)
+    p = ch.params
+    exp = oracle.chunk(data, oracle.Params(p.poly, p.window, p.divisor, p.magic, p.min_size, p.max_size))
+    assert np.array_equal(got, exp), (p, data.size)
+
+
+def main():
+    n = (1 << 20) + 333
+    data = synthgen.random_bytes(1, n)
+    check(pkg.Chunker(pkg.Params()), data, 3)
+    check(pkg.Chunker(pkg.Params(divisor=64, magic=5)), data)
+    check(pkg.Chunker(pkg.Params(poly=0x104C11DB7)), data, 1)
+    check(pkg.Chunker(pkg.Params(window=32)), data[:200000])
+    check(pkg.Chunker(pkg.Params(min_size=2048, max_size=65536)), data)
+    check(pkg.Chunker(pkg.Params()), synthgen.periodic(b"\x04\xd5", 300000))
+    check(pkg.Chunker(pkg.Params(min_size=3)), synthgen.periodic(b"\x04\xd5", 100000))
+    ch = pkg.Chunker(pkg.Params(divisor=1024, min_size=256, max_size=4096))
+    ch.set_ring(2, 1 << 18)
+    outs = []
+    for a, b in ((0, 1000), (1000, 700001), (700001, n)):
+        outs.append(ch.feed(torch.from_numpy(data[a:b].copy()).pin_memory()).cpu().numpy())
+    outs.append(ch.flush().cpu().numpy())
+    got = np.concatenate(outs).astype(np.uint64)
+    assert np.array_equal(got, oracle.chunk(data, oracle.Params(divisor=1024, min_size=256, max_size=4096)))
+    torch.cuda.synchronize()
+    print("sanitize cases ok")
+
+
+if __name__ == "__main__":
+    main()
