@@ -201,10 +201,20 @@ def main():
     import synthgen
     import paper_conf_fast_bhatotiarv12_b200 as pkg
 
+    # Test-only overrides (exercise the N > 1 code path on a 1-GPU box): SHRED_BENCH_BACKEND=gloo
+    # and SHRED_BENCH_DEVICE=0 put every rank on one device.  Real runs: NCCL, one GPU per rank.
+    backend = os.environ.get("SHRED_BENCH_BACKEND", "nccl")
+    local = int(os.environ.get("SHRED_BENCH_DEVICE", local))
     torch.cuda.set_device(local)
     if world > 1:
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        if backend == "nccl":
+            dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        else:
+            dist.init_process_group(backend)
     dev = torch.device("cuda", local)
+
+    def coll_dev(t):            # gloo exchanges host tensors
+        return t if backend == "nccl" else t.cpu()
     stream = torch.cuda.current_stream()
 
     # ---- inputs (untimed): this rank's shard of stream seed 2 with its halo, and an edited file
@@ -236,7 +246,12 @@ def main():
             ch._check(rc, "shred_candidates_range")
         ch.chunk_async(edited, out1, n1)
         if world > 1:
-            dist.all_gather_into_tensor(counts, n0)       # C2: per-rank candidate counts
+            if backend == "nccl":
+                dist.all_gather_into_tensor(counts, n0)   # C2: per-rank candidate counts
+            else:
+                cc = torch.zeros(world, dtype=torch.int64)
+                dist.all_gather_into_tensor(cc, n0.cpu())
+                counts.copy_(cc)
 
     for _ in range(args.warmup):
         step()
@@ -259,7 +274,7 @@ def main():
     if world > 1:
         dist.barrier()
     ms = e0.elapsed_time(e1)
-    t = torch.tensor([ms], dtype=torch.float64, device=dev)
+    t = coll_dev(torch.tensor([ms], dtype=torch.float64, device=dev))
     if world > 1:
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
     ms_max = float(t.item())
@@ -338,7 +353,7 @@ def main():
         s1.record(stream)
         torch.cuda.synchronize()
         ems = s0.elapsed_time(s1)
-        et = torch.tensor([ems], dtype=torch.float64, device=dev)
+        et = coll_dev(torch.tensor([ems], dtype=torch.float64, device=dev))
         if world > 1:
             dist.all_reduce(et, op=dist.ReduceOp.MAX)
         ems = float(et.item())
