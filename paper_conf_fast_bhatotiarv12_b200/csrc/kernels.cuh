@@ -35,7 +35,8 @@
 #define SHRED_PRODUCER_SLEEP_NS 512
 #endif
 #ifndef SHRED_HITMODE
-#define SHRED_HITMODE 0         // 0: per-byte hit bitmask; 1: chunk predicate + exact replay on hit
+#define SHRED_HITMODE 3         // 3: ISETP + predicated OR per byte (default); 0: ISETP+SEL bitmask;
+                                // 1: chunk predicate + exact replay on hit; 2: FMA-pipe test
 #endif
 
 namespace shred {
@@ -385,6 +386,14 @@ template <> struct State<MODE_K32> {
 
 // marker test: (f mod D) == r  <=>  (f_lo << (32-m)) == (r << (32-m))   (D = 2^m <= 2^32)
 __device__ __forceinline__ bool is_marker(uint32_t lo, const BulkCtx &c) { return lo * c.tmul == c.rsh; }
+// m | BIT if marker else m: ISETP + predicated LOP3 (the PTX predication survives ptxas).
+template <uint32_t BIT>
+__device__ __forceinline__ uint32_t or_if_marker(uint32_t m, uint32_t lo, const BulkCtx &c) {
+    const uint32_t x = lo * c.tmul;
+    asm("{\n .reg .pred p;\n setp.eq.u32 p, %1, %2;\n @p or.b32 %0, %0, %3;\n}"
+        : "+r"(m) : "r"(x), "r"(c.rsh), "n"(BIT));
+    return m;
+}
 // FMA-pipe form: 1 if NOT a marker.  y = (f_lo << (32-m)) - (r << (32-m)) is 0 iff marker;
 // hi32(y * 1 + 0xFFFFFFFF) = (y != 0).
 __device__ __forceinline__ uint32_t not_marker(uint32_t lo, const BulkCtx &c) {
@@ -416,6 +425,8 @@ __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t min_i,
 #define SHRED_MARK(ch, q) m[ch] |= is_marker(st[ch].low(), c) ? (1u << (4 * J + q)) : 0u;
 #elif SHRED_HITMODE == 2
 #define SHRED_MARK(ch, q) m[ch] = m[ch] * c.two + not_marker(st[ch].low(), c);
+#elif SHRED_HITMODE == 3
+#define SHRED_MARK(ch, q) m[ch] = or_if_marker<(1u << (4 * J + q))>(m[ch], st[ch].low(), c);
 #else
 #define SHRED_MARK(ch, q) m[ch] |= (uint32_t)is_marker(st[ch].low(), c);
 #endif
