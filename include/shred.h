@@ -98,9 +98,8 @@ uint64_t    shred_max_cuts(const shred_ctx *ctx, uint64_t len);
 /* One-shot, device-resident chunking of d_in[0..len) as a whole stream.
    Writes the ascending final cuts (candidates, then the size rule if min > 0 or max > 0) to
    d_out[0 .. min(n, cap)) and n to *n_out.  d_in may have any alignment.  len = 0 is valid
-   (n = 0).  Enqueues on `stream`, returns after enqueue — except in bounded mode (min or max
-   set), where it synchronises `stream` once to read the candidate count and size the ordered
-   candidate list the size rule runs over. */
+   (n = 0).  Enqueues on `stream`, returns after enqueue (device scratch may be grown — a
+   synchronous cudaMalloc — the first time a larger input is seen). */
 int shred_chunk(shred_ctx *ctx, const uint8_t *d_in, uint64_t len,
                 uint64_t *d_out, uint64_t cap, uint64_t *n_out, shred_stream_t stream);
 
@@ -128,8 +127,7 @@ int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, ui
    stream into a ring of device slots (double/triple buffering) while the previous slot is
    chunked on `stream`.  Offsets are absolute stream positions.  Only final cuts are emitted:
    a cut at exactly the current stream end is held until the next feed (emitted) or the flush
-   (dropped: c = N is never a cut).  len may be 0.  Bounded mode synchronises `stream` once per
-   piece (as shred_chunk); the next piece's H2D copy is already in flight by then. */
+   (dropped: c = N is never a cut).  len may be 0. */
 int shred_feed (shred_ctx *ctx, const void *in, uint64_t len,
                 uint64_t *d_out, uint64_t cap, uint64_t *n_out, shred_stream_t stream);
 /* End the stream: emits the remaining forced max-size cuts and resets the stream state. */

@@ -133,6 +133,8 @@ struct Aux {
     uint64_t held;              // 1 if a cut at exactly the previous stream end is held
     uint64_t held_val;
     uint64_t overflow;          // sticky: an output did not fit
+    uint64_t dense;             // the ordered candidate list did not fit (size-rule fallback)
+    uint64_t ncand;             // candidates of the current piece (k_scatter; read by sb_*)
     uint64_t pad;
 };
 
@@ -742,6 +744,8 @@ k_scatter(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots,
     const uint64_t total = carry;
     if (blockIdx.x == 0 && tid == 0) {
         aux->total = total;
+        aux->ncand = total;
+        aux->dense = total > dst_cap ? 1ull : 0ull;
         if (n_direct) { *n_direct = total; if (total > dst_cap) aux->overflow = 1; }
     }
     const uint32_t slot = blockIdx.x * blockDim.x + tid;
@@ -794,7 +798,7 @@ __global__ void k_call_end(Aux *aux, uint64_t *n_out, uint64_t cap, volatile uin
 
 __global__ void k_stream_reset(Aux *aux) {
     aux->total = 0; aux->last_cand = 0; aux->out_pos = 0;
-    aux->s = 0; aux->held = 0; aux->held_val = 0;
+    aux->s = 0; aux->held = 0; aux->held_val = 0; aux->dense = 0;
 }
 
 __global__ void k_write_u64(uint64_t *p, uint64_t v) { *p = v; }

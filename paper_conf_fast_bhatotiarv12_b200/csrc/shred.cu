@@ -334,15 +334,18 @@ int launch_scatter(shred_ctx *ctx, Plan &pl, uint64_t *dst, uint64_t dst_cap, Au
 
 bool bounded(const shred_ctx *ctx) { return ctx->p.min_size > 0 || ctx->p.max_size > 0; }
 
-// The size rule over n ascending candidates (n known on the host for the grid sizes; the
-// kernels read the count from n_dev if given).  Appends to dst at aux->out_pos; updates aux.
-int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_dev, uint64_t n,
-                      uint64_t end, int fin, uint64_t *dst, uint64_t cap, Aux *aux, cudaStream_t st) {
-    const uint64_t nb = (n + SB_B - 1) / SB_B;
+// The size rule over ascending candidates.  `nmax` bounds the count for the grid sizes; the
+// kernels read the true count from n_dev if given (else n_host).  Appends to dst at
+// aux->out_pos; updates aux.  With `pl` given, the dense fallback (sb_dense) is enqueued too: it
+// runs only if the ordered list could not hold every candidate.
+int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_dev, uint64_t n_host,
+                      uint64_t nmax, uint64_t end, int fin, uint64_t *dst, uint64_t cap, Aux *aux,
+                      const Plan *pl, cudaStream_t st) {
+    const uint64_t nb = (nmax + SB_B - 1) / SB_B;
     int rc = grow(ctx, ctx->d_sb, ctx->sb_cap, 6 * (nb + 2), "size-rule scratch");
     if (rc) return rc;
     SBArgs A;
-    A.cand = cand; A.n_dev = n_dev; A.n_host = n;
+    A.cand = cand; A.n_dev = n_dev; A.n_host = n_host;
     A.minsz = ctx->p.min_size; A.maxsz = ctx->p.max_size; A.end = end; A.fin = fin;
     uint64_t *b = ctx->d_sb;
     A.spec_exit = b; A.spec_cnt = b + (nb + 2); A.entry = b + 2 * (nb + 2); A.offs = b + 3 * (nb + 2);
@@ -359,23 +362,16 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
     LAUNCHED("sb_plan");
     sb_emit<<<(unsigned)((nb + 1 + SB_THREADS - 1) / SB_THREADS), SB_THREADS, 0, st>>>(A);
     LAUNCHED("sb_emit");
-    return SHRED_OK;
-}
-
-// Bounded mode needs the whole ordered candidate list: read the count back (the one
-// synchronous point of the bounded path) and size the ctx buffer for it.
-int ensure_cand(shred_ctx *ctx, Plan &pl, Aux *aux, cudaStream_t st, uint64_t &total) {
-    if (pl.nslots) {
-        k_total<<<1, 256, 0, st>>>(ctx->d_groups, pl.J.map.ngroups, aux);
-        LAUNCHED("k_total");
-    } else {
-        k_write_u64<<<1, 1, 0, st>>>(&aux->total, 0);
-        LAUNCHED("k_write_u64");
+    if (pl && pl->nslots) {
+        uint64_t maxseg = pl->J.map.S;
+        if (pl->J.map.head_seg > maxseg) maxseg = pl->J.map.head_seg;
+        if (pl->J.map.tail_seg > maxseg) maxseg = pl->J.map.tail_seg;
+        if (maxseg > SBD_WIN) maxseg = SBD_WIN;
+        const size_t smem = (size_t)((maxseg + 31) / 32) * 4;
+        sb_dense<<<1, SBD_THREADS, smem, st>>>(pl->J, ctx->dp, ctx->d_gen, pl->nslots, A);
+        LAUNCHED("sb_dense");
     }
-    CK(cudaMemcpyAsync(ctx->h_pinned, &aux->total, sizeof(uint64_t), cudaMemcpyDeviceToHost, st), "read total");
-    CK(cudaStreamSynchronize(st), "sync total");
-    total = ctx->h_pinned[0];
-    return grow(ctx, ctx->d_cand, ctx->cand_cap, total + 1, "candidate list");
+    return SHRED_OK;
 }
 
 // One piece of a stream (or a whole one-shot stream): window ends [t_begin, t_end).
@@ -398,10 +394,12 @@ int run_piece(shred_ctx *ctx, Aux *aux, const uint8_t *src, uint64_t p_begin, co
         LAUNCHED("k_piece_done");
         return SHRED_OK;
     }
-    uint64_t total = 0;
-    if ((rc = ensure_cand(ctx, pl, aux, st, total))) return rc;
-    if ((rc = launch_scatter(ctx, pl, ctx->d_cand, ctx->cand_cap, aux, 0, nullptr, st))) return rc;
-    return launch_size_bound(ctx, ctx->d_cand, nullptr, total, t_end, final_, dst, dst_cap, aux, st);
+    // ordered candidate list: every slot's complete list fits (dense inputs -> sb_dense)
+    const uint64_t ccap = (uint64_t)pl.nslots * pl.J.cap + 1;
+    if ((rc = grow(ctx, ctx->d_cand, ctx->cand_cap, ccap, "candidate list"))) return rc;
+    if ((rc = launch_scatter(ctx, pl, ctx->d_cand, ccap, aux, 0, nullptr, st))) return rc;
+    return launch_size_bound(ctx, ctx->d_cand, &aux->ncand, 0, ccap, t_end, final_, dst, dst_cap, aux,
+                             &pl, st);
 }
 
 // Kind of a user pointer: 1 = device, 2 = page-locked host, 0 = pageable / unknown.
@@ -543,6 +541,9 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
             cudaFuncSetAttribute(k1_bulk<MODE_K32, CfgK32>, cudaFuncAttributeMaxDynamicSharedMemorySize, CfgK32::SMEM) != cudaSuccess)
             return bail(SHRED_ECUDA);
     }
+    if (cudaFuncSetAttribute(sb_dense, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             (int)(SBD_WIN / 8)) != cudaSuccess)
+        return bail(SHRED_ECUDA);
     if (cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking) != cudaSuccess)
         return bail(SHRED_ECUDA);
     if (cudaDeviceSynchronize() != cudaSuccess) return bail(SHRED_ECUDA);
@@ -622,7 +623,8 @@ int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, ui
     Aux *aux = ctx->d_aux + 0;
     k_stream_reset<<<1, 1, 0, st>>>(aux);
     LAUNCHED("k_stream_reset");
-    if ((rc = launch_size_bound(ctx, d_cand, nullptr, n_cand, total_len, 1, d_out, cap, aux, st))) return rc;
+    if ((rc = launch_size_bound(ctx, d_cand, nullptr, n_cand, n_cand, total_len, 1, d_out, cap, aux,
+                                nullptr, st))) return rc;
     k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, nullptr);
     LAUNCHED("k_call_end");
     return SHRED_OK;

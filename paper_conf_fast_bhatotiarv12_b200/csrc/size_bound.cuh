@@ -71,6 +71,7 @@ __device__ __forceinline__ uint64_t sb_tail_count(uint64_t s, const SBArgs &A) {
 }
 
 __global__ void __launch_bounds__(SB_THREADS) sb_spec(SBArgs A) {
+    if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
     const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
@@ -90,6 +91,7 @@ __global__ void __launch_bounds__(SB_THREADS) sb_spec(SBArgs A) {
 }
 
 __global__ void __launch_bounds__(SB_THREADS) sb_check(SBArgs A) {
+    if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
     const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
@@ -119,6 +121,7 @@ __global__ void __launch_bounds__(SB_THREADS) sb_check(SBArgs A) {
 __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
     __shared__ uint64_t wsum[33];
     __shared__ int all_ok;
+    if (A.aux->dense) return;
     const uint64_t n = sb_n(A);
     const uint32_t nb = (uint32_t)((n + SB_B - 1) / SB_B);
     const uint32_t tid = threadIdx.x;
@@ -211,6 +214,7 @@ __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
 
 // Every block writes its cuts; thread nb writes the forced cuts after the last candidate.
 __global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
+    if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
     const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
@@ -233,6 +237,83 @@ __global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
 #pragma unroll
     for (int j = 0; j < SB_B; ++j)
         if (first + j < last) sb_step(s, v[j], A, held, emit);
+}
+
+// ------------------------------------------------------------------------------ sb_dense
+// Exact fallback when the ordered candidate list could not hold every candidate (only possible
+// when some slot's list overflowed, i.e. dense candidates such as a repeated `04 D5`): one CTA
+// walks the slots in stream order.  Warp 0 owns the rule state; slots whose list is complete
+// are read from it, overflowed slots are re-rolled by all threads into a shared bitmap (in
+// windows of SBD_WIN window ends) that warp 0 then scans in order.
+constexpr int SBD_THREADS = 256;
+constexpr uint64_t SBD_WIN = 1ull << 20;              // window ends per bitmap pass (128 KiB)
+__global__ void __launch_bounds__(SBD_THREADS)
+sb_dense(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots, SBArgs A) {
+    Aux *aux = A.aux;
+    if (!aux->dense) return;
+    extern __shared__ uint32_t bm[];
+    __shared__ uint64_t sT[256], sU[256];
+    for (int i = threadIdx.x; i < 256; i += blockDim.x) { sT[i] = gt->T[i]; sU[i] = gt->U[i]; }
+    __syncthreads();
+    const int tid = threadIdx.x, lane = tid & 31;
+    const bool w0 = tid < 32;
+    uint64_t s = aux->s, off = aux->out_pos;
+    int held = 0;
+    uint64_t *dst = A.dst;
+    const uint64_t cap = A.dst_cap;
+    auto emit = [&](uint64_t v) { if (lane == 0 && off < cap) dst[off] = v; ++off; };
+    if (aux->held) emit(aux->held_val);
+    SmemGenTab tab{sT, sU};
+    for (uint32_t slot = 0; slot < nslots; ++slot) {
+        uint64_t a, b;
+        slot_range(J.map, slot, a, b);
+        const uint32_t cnt = J.counts[slot];
+        if (cnt <= J.cap) {
+            if (w0) {
+                const uint64_t *lst = J.scratch + (uint64_t)slot * J.cap;
+                for (uint32_t j = 0; j < cnt; j += 32) {
+                    const uint64_t v = (j + lane < cnt) ? lst[j + lane] : 0ull;
+                    const uint32_t m = min(32u, cnt - j);
+                    for (uint32_t k = 0; k < m; ++k) sb_step(s, __shfl_sync(0xffffffffu, v, k), A, held, emit);
+                }
+            }
+            continue;
+        }
+        for (uint64_t wa = a; wa < b; wa += SBD_WIN) {
+            const uint64_t wb = min(b, wa + SBD_WIN);
+            const uint32_t nw = (uint32_t)((wb - wa + 31) / 32);
+            for (uint32_t i = tid; i < nw; i += blockDim.x) bm[i] = 0;
+            __syncthreads();
+            const uint64_t per = (wb - wa + blockDim.x - 1) / blockDim.x;
+            const uint64_t ta = wa + per * tid, tb = min(wb, ta + per);
+            if (ta < tb)
+                roll_generic(J, P, tab, ta, tb, [&](uint64_t c) {
+                    const uint64_t k = c - 1 - wa;                 // window end offset in the window
+                    atomicOr(&bm[k >> 5], 1u << (k & 31));
+                });
+            __syncthreads();
+            if (w0) {
+                for (uint32_t i = 0; i < nw; ++i) {
+                    uint32_t word = bm[i];
+                    while (word) {
+                        const int bit = __ffs(word) - 1;
+                        word &= word - 1;
+                        sb_step(s, wa + 32ull * i + (uint64_t)bit + 1, A, held, emit);
+                    }
+                }
+            }
+            __syncthreads();
+        }
+    }
+    if (tid == 0) {
+        const uint64_t mt = sb_tail_count(s, A);
+        for (uint64_t j = 1; j <= mt; ++j) { if (off < cap) dst[off] = s + j * A.maxsz; ++off; }
+        aux->total = off - aux->out_pos - aux->held;
+        aux->out_pos = off;
+        aux->s = s + mt * A.maxsz;
+        aux->held = (uint64_t)held;
+        aux->held_val = held ? A.end : 0;
+    }
 }
 
 }  // namespace shred
