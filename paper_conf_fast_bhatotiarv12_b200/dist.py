@@ -38,6 +38,28 @@ def halo_of(start: int, window: int = 48) -> int:
     return min(window - 1, start)
 
 
+def exchange_halo(own: torch.Tensor, start: int, window: int = 48, group=None) -> torch.Tensor:
+    """C1 for real (non-regenerable) data: rank g gets the last min(w-1, start) bytes of the
+    bytes before its shard from its predecessor, and returns [halo || own] ready for
+    chunk_sharded.  The exchange is one all-gather of each rank's (w-1)-byte tail
+    ((w-1) x world bytes over NCCL/NVLink; ranks must hold contiguous shards in rank order and a
+    shard shorter than w-1 bytes must not follow another short one)."""
+    world = dist.get_world_size(group)
+    rank = dist.get_rank(group)
+    k = window - 1
+    tail = torch.zeros(k, dtype=torch.uint8, device=own.device)
+    m = min(k, own.numel())
+    if m:
+        tail[k - m:] = own[own.numel() - m:]
+    allt = torch.zeros(world * k, dtype=torch.uint8, device=own.device)
+    dist.all_gather_into_tensor(allt, tail, group=group)
+    halo = min(k, start)
+    if rank == 0 or halo == 0:
+        return own.contiguous()
+    prev = allt.view(world, k)[rank - 1]
+    return torch.cat([prev[k - halo:], own]).contiguous()
+
+
 @dataclass
 class ShardResult:
     local: torch.Tensor          # this rank's candidates (absolute offsets, ascending)

@@ -59,6 +59,9 @@ def _worker(rank, world, port, n, seed, params, q):
         halo = sd.halo_of(start, params.window)
         x = torch.from_numpy(synthgen.random_bytes(seed, end - start + halo, start - halo))
         assert np.array_equal(x.numpy(), data[start - halo:end])   # halo regenerated locally
+        own = torch.from_numpy(data[start:end].copy())
+        x2 = sd.exchange_halo(own, start, params.window)            # C1 over the process group
+        assert np.array_equal(x2.numpy(), x.numpy())
         eng = OracleEngine(params, data)
         res = sd.chunk_sharded(x, halo, start, n, eng)
         allc = sd.gather_all(res).numpy()
