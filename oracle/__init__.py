@@ -12,7 +12,8 @@ Functions (each cites the passage it follows; readings Q1..Q17 are listed in DES
 
 * :func:`polymod` — R1, M(x) mod P(x) by long division (Eq. (1)).
 * :func:`window_fp` / :func:`window_fps` — fingerprint of every full window (L444-L454, Q3/Q4/Q10).
-* :func:`candidates` — {c = i+1 : fp_i mod D == r, c < N} (L447-L451, Q5-Q11).
+* :func:`candidates` — {c = i+1 : fp_i mod D == r, c < N} (L447-L451, Q5-Q11); marker = 1
+  gives the "mod p ... lower or equal to a constant" marker set of L249-L251.
 * :func:`size_bound` — min/max rule (L259-L269, Q12-Q15).
 * :func:`chunk` — candidates then size rule: the final cut offsets.
 * :func:`is_irreducible` — Rabin's irreducibility test for ``div(x)`` (L255-L256).
@@ -71,7 +72,7 @@ def _L():
         lib.orc_window_fps.restype = cint
         lib.orc_window_fps.argtypes = [P, u64, u32, u64, cint, P]
         lib.orc_candidates.restype = i64
-        lib.orc_candidates.argtypes = [P, u64, u32, u64, u64, u64, cint, cint, P, u64]
+        lib.orc_candidates.argtypes = [P, u64, u32, u64, u64, u64, cint, cint, cint, P, u64]
         lib.orc_size_bound.restype = i64
         lib.orc_size_bound.argtypes = [P, u64, u64, u64, u64, P, u64]
         _lib = lib
@@ -89,6 +90,7 @@ class Params:
     magic: int = 0x78
     min_size: int = 0
     max_size: int = 0
+    marker: int = 0     # 0: fp mod D == r (L447-L451); 1: fp mod D <= r (L249-L251, variant f4)
 
 
 def _bytes(data) -> np.ndarray:
@@ -154,7 +156,7 @@ def candidates(data, p: Params = Params(), method: int = 2, threads: int | None 
     while True:
         out = np.zeros(cap, dtype=np.uint64)
         n = _L().orc_candidates(a.ctypes.data, a.size, p.window, p.poly, p.divisor, p.magic,
-                                method, threads, out.ctypes.data, cap)
+                                p.marker, method, threads, out.ctypes.data, cap)
         assert n >= 0, "oracle allocation failure"
         if n <= cap:
             return out[:n].copy()

@@ -20,11 +20,13 @@ def window_fp(window: bytes, p: int) -> int:
     return gf2_mod(int.from_bytes(bytes(window), "big"), p)
 
 
-def candidates(data: bytes, p: int, w: int, D: int, r: int) -> list[int]:
-    """Every c = i+1 with w-1 <= i, c < N and fp_i mod D == r (readings Q9-Q11)."""
+def candidates(data: bytes, p: int, w: int, D: int, r: int, marker: int = 0) -> list[int]:
+    """Every c = i+1 with w-1 <= i, c < N and fp_i mod D == r (readings Q9-Q11); marker = 1:
+    fp_i mod D <= r (the "lower or equal to a constant" marker set, L249-L251)."""
     data = bytes(data)
     out = []
     for i in range(w - 1, len(data) - 1):
-        if window_fp(data[i + 1 - w:i + 1], p) % D == r:
+        v = window_fp(data[i + 1 - w:i + 1], p) % D
+        if (v <= r) if marker else (v == r):
             out.append(i + 1)
     return out

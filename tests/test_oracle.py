@@ -312,3 +312,25 @@ def test_synthgen_splitmix_vector(golden_dir):
     full = synthgen.random_bytes(3, 1000)
     for off, ln in ((0, 1), (1, 7), (13, 100), (999, 1), (8, 8)):
         assert np.array_equal(synthgen.random_bytes(3, ln, off), full[off:off + ln])
+
+
+# --------------------------------------------------------------------------- variants (f4)
+@pytest.mark.parametrize("D,r,marker", [(1000, 7, 0), (3, 0, 0), (12345, 999, 1), (256, 3, 1), (7, 6, 1)])
+def test_variant_markers_vs_brute_force(D, r, marker):
+    """Non-power-of-two D and the "mod p <= constant" marker set."""
+    data = synthgen.random_bytes(D + r, 2500)
+    exp = brute.candidates(data.tobytes(), LBFS, 48, D, r, marker)
+    p = Params(divisor=D, magic=r, marker=marker)
+    for method in (1, 2):
+        assert oracle.candidates(data, p, method=method, threads=2).tolist() == exp
+
+
+def test_le_marker_density():
+    """fp mod D <= r on random bytes: density exactly (r+1)/D (fp uniform on GF(2)^63, D | 2^63
+    for powers of two; for other D the bias is < D/2^63)."""
+    n = 2 << 20
+    data = synthgen.random_bytes(33, n)
+    for D, r in ((8192, 1), (10000, 4)):
+        k = oracle.candidates(data, Params(divisor=D, magic=r, marker=1)).size
+        mu = (n - 48) * (r + 1) / D
+        assert abs(k - mu) <= 4 * np.sqrt(mu)
