@@ -49,8 +49,11 @@ typedef struct shred_params {
     uint64_t poly;      /* div(x) over GF(2): bit t = coefficient of x^t; irreducible,
                            8 <= deg <= 63.  Default 0xbfe6b8a5bf378d83 (deg 63, reading Q1).  */
     uint32_t window;    /* w bytes, 1 <= w <= 4096.  Default 48 (L444-L446).                   */
-    uint32_t reserved;  /* must be 0                                                           */
-    uint64_t divisor;   /* D, power of two, 2 <= D <= 2^deg.  Default 8192 ("13 bits", L447).   */
+    uint32_t marker;    /* SHRED_MARKER_EQ (0, default): a cut candidate where fp mod D == r
+                           (L447-L451); SHRED_MARKER_LE (1): where fp mod D <= r, the "value mod
+                           p is lower or equal to a constant" marker set of L249-L251.          */
+    uint64_t divisor;   /* D, 2 <= D <= 2^deg.  Default 8192 ("13 bits", L447).  A power of two
+                           selects the fast paths; any other D runs the generic path.           */
     uint64_t magic;     /* r < D.  Default 0x78 (reading Q6).                                  */
     uint64_t min_size;  /* 0 = off (paper default)                                  */
     uint64_t max_size;  /* 0 = off (= inf).  Else max_size >= max(min_size, 1)                 */
@@ -67,18 +70,21 @@ enum {
     SHRED_ECAPACITY = -5    /* sticky: a streaming call overflowed its output buffer         */
 };
 
+enum { SHRED_MARKER_EQ = 0, SHRED_MARKER_LE = 1 };
+
 /* Kernel paths the ctx selected for its parameters (shred_path). */
 enum {
     SHRED_PATH_K63     = 1, /* deg(P) = 63, D <= 2^32: u64 state, TMA-staged, smem LDS.64 tables */
     SHRED_PATH_K32     = 2, /* deg(P) = 32, D <= 2^32: u32 state, TMA-staged, smem LDS.32 tables */
-    SHRED_PATH_GENERIC = 3  /* any other valid parameters: byte-at-a-time kernel                */
+    SHRED_PATH_GENERIC = 3  /* any other valid parameters (other w or degree, D not a power of two,
+                               D > 2^32, SHRED_MARKER_LE): byte-at-a-time kernel              */
 };
 
 /* Fill *p with the paper defaults (readings Q1, Q5, Q6, Q15): P = 0xbfe6b8a5bf378d83, w = 48,
    D = 8192, r = 0x78, min = 0, max = 0 (off). */
 void        shred_default_params(shred_params *p);
 
-/* Validate *p (degree, irreducibility of P by Ben-Or's test, D power of two, r < D,
+/* Validate *p (degree, irreducibility of P by Ben-Or's test, 2 <= D <= 2^deg, r < D, marker,
    min/max), build the push/pop tables (PAPER.md: "shifting a byte forward") on the
    host, upload them to `device` and create the ctx.  Synchronous.  *out = NULL on error. */
 int         shred_init(const shred_params *p, int device, shred_ctx **out);

@@ -25,7 +25,7 @@ class ShredError(RuntimeError):
 
 
 class _Params(ctypes.Structure):
-    _fields_ = [("poly", ctypes.c_uint64), ("window", ctypes.c_uint32), ("reserved", ctypes.c_uint32),
+    _fields_ = [("poly", ctypes.c_uint64), ("window", ctypes.c_uint32), ("marker", ctypes.c_uint32),
                 ("divisor", ctypes.c_uint64), ("magic", ctypes.c_uint64),
                 ("min_size", ctypes.c_uint64), ("max_size", ctypes.c_uint64)]
 
@@ -39,9 +39,11 @@ class Params:
     magic: int = 0x78
     min_size: int = 0
     max_size: int = 0
+    marker: int = 0          # 0: fp mod D == r (L447-L451); 1: fp mod D <= r (L249-L251)
 
     def _c(self) -> _Params:
-        return _Params(self.poly, self.window, 0, self.divisor, self.magic, self.min_size, self.max_size)
+        return _Params(self.poly, self.window, self.marker, self.divisor, self.magic, self.min_size,
+                       self.max_size)
 
 
 _lib = None

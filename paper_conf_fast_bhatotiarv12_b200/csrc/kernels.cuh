@@ -100,12 +100,21 @@ __host__ __device__ __forceinline__ uint32_t slot_group(const SlotMap &m, uint32
 }
 
 struct DevParams {              // chunking parameters as the kernels need them
-    uint64_t dmask;             // D - 1
+    uint64_t dmask;             // D - 1 (D a power of two)
     uint64_t magic;             // r
     uint64_t kmask;             // 2^k - 1
+    uint64_t divisor;           // D
     uint32_t k;                 // deg P
     uint32_t w;                 // window bytes
+    uint32_t pow2;              // D is a power of two
+    uint32_t marker;            // 0: fp mod D == r; 1: fp mod D <= r
 };
+
+// The marker predicate of the generic path (L247-L251, L447-L451).
+__device__ __forceinline__ bool generic_marker(uint64_t f, const DevParams &P) {
+    const uint64_t v = P.pow2 ? (f & P.dmask) : (f % P.divisor);
+    return P.marker ? (v <= P.magic) : (v == P.magic);
+}
 
 struct Job {
     const uint8_t *src;         // src[0] is stream position p_begin
@@ -225,7 +234,7 @@ __device__ __forceinline__ void roll_generic(const Job &J, const DevParams &P, c
         uint32_t t = (uint32_t)(f >> (P.k - 8u)) & 0xFFu;
         f = ((f << 8) & P.kmask) ^ (uint64_t)b ^ tab.T(t);
         if (pos >= p + P.w) f ^= tab.U(job_byte(J, pos - P.w));
-        if (pos >= seg_start && pos >= J.min_i && (f & P.dmask) == P.magic && pos + 1 < J.c_limit)
+        if (pos >= seg_start && pos >= J.min_i && generic_marker(f, P) && pos + 1 < J.c_limit)
             emit(pos + 1);
     }
 }

@@ -163,9 +163,9 @@ int validate(const shred_params *p, shred_ctx *ctx) {
     if (k < 8 || k > 63) return fail(ctx, SHRED_EINVAL, "deg(poly) = %d, need 8..63", k);
     if (!irreducible(p->poly)) return fail(ctx, SHRED_EINVAL, "poly 0x%llx is reducible", (unsigned long long)p->poly);
     if (p->window < 1 || p->window > 4096) return fail(ctx, SHRED_EINVAL, "window %u not in 1..4096", p->window);
-    if (p->reserved != 0) return fail(ctx, SHRED_EINVAL, "reserved field must be 0");
-    if (p->divisor < 2 || (p->divisor & (p->divisor - 1))) return fail(ctx, SHRED_EINVAL, "divisor must be a power of two >= 2");
-    if (deg64(p->divisor) > k) return fail(ctx, SHRED_EINVAL, "divisor exceeds 2^deg(poly)");
+    if (p->marker > SHRED_MARKER_LE) return fail(ctx, SHRED_EINVAL, "marker must be SHRED_MARKER_EQ or SHRED_MARKER_LE");
+    if (p->divisor < 2) return fail(ctx, SHRED_EINVAL, "divisor must be >= 2");
+    if (k < 63 && p->divisor > (1ull << k)) return fail(ctx, SHRED_EINVAL, "divisor exceeds 2^deg(poly)");
     if (p->magic >= p->divisor) return fail(ctx, SHRED_EINVAL, "magic must be < divisor");
     if (p->max_size && p->max_size < (p->min_size > 1 ? p->min_size : 1))
         return fail(ctx, SHRED_EINVAL, "max_size must be >= max(min_size, 1)");
@@ -483,9 +483,13 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     ctx->dp.kmask = (1ull << k) - 1ull;
     ctx->dp.dmask = p->divisor - 1ull;
     ctx->dp.magic = p->magic;
-    const bool fast_w = (p->window == 48);
-    if (k == 63 && fast_w && p->divisor <= (1ull << 32)) ctx->path = SHRED_PATH_K63;
-    else if (k == 32 && fast_w && p->divisor <= (1ull << 32)) ctx->path = SHRED_PATH_K32;
+    ctx->dp.divisor = p->divisor;
+    ctx->dp.pow2 = (p->divisor & (p->divisor - 1)) == 0 ? 1u : 0u;
+    ctx->dp.marker = p->marker;
+    const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
+    const bool fast = (p->window == 48) && pow2 && p->divisor <= (1ull << 32) && p->marker == SHRED_MARKER_EQ;
+    if (k == 63 && fast) ctx->path = SHRED_PATH_K63;
+    else if (k == 32 && fast) ctx->path = SHRED_PATH_K32;
     else ctx->path = SHRED_PATH_GENERIC;
     if (major != 10) ctx->path = SHRED_PATH_GENERIC;   // the TMA kernels are built for sm_100a only
 

@@ -69,7 +69,8 @@ def test_init_rejects_bad_params_without_touching_the_gpu(libpath):
     bad = [
         _Params((1 << 63) | 1, 48, 0, 8192, 0x78, 0, 0),          # reducible x^63+1
         _Params(0xBFE6B8A5BF378D83, 0, 0, 8192, 0x78, 0, 0),      # w = 0
-        _Params(0xBFE6B8A5BF378D83, 48, 0, 8191, 0x78, 0, 0),     # D not a power of two
+        _Params(0xBFE6B8A5BF378D83, 48, 2, 8192, 0x78, 0, 0),     # unknown marker mode
+        _Params(0xBFE6B8A5BF378D83, 48, 0, 1, 0, 0, 0),           # D < 2
         _Params(0xBFE6B8A5BF378D83, 48, 0, 8192, 8192, 0, 0),     # r >= D
         _Params(0xBFE6B8A5BF378D83, 48, 0, 8192, 0x78, 100, 50),  # max < min
         _Params(0x1F, 48, 0, 4, 0, 0, 0),                         # degree 4 < 8

@@ -31,7 +31,7 @@ def dev(a: np.ndarray, offset: int = 0) -> torch.Tensor:
 
 
 def oparams(p) -> oracle.Params:
-    return oracle.Params(p.poly, p.window, p.divisor, p.magic, p.min_size, p.max_size)
+    return oracle.Params(p.poly, p.window, p.divisor, p.magic, p.min_size, p.max_size, p.marker)
 
 
 def check_chunk(ch, data: np.ndarray, offset: int = 0, method: int = 2):
@@ -247,3 +247,16 @@ def test_bounded_adversarial_stream(pkg):
     per = synthgen.periodic(b"\x04\xd5", n)
     for mn, mx in ((3, 0), (3, 1000), (4097, 65536)):
         check_chunk(pkg.Chunker(pkg.Params(min_size=mn, max_size=mx)), per)
+
+
+# ------------------------------------------------------------------ variants (f4)
+def test_marker_le_and_non_pow2_divisor(pkg):
+    """The "value mod p <= constant" marker set (L249-L251) and divisors that are not powers of
+    two run on the generic path, bit-exact vs the oracle; bounded mode on top."""
+    data = synthgen.random_bytes(31, (2 << 20) + 77)
+    for p in (pkg.Params(divisor=10000, magic=1234), pkg.Params(divisor=8192, magic=1, marker=1),
+              pkg.Params(divisor=12345, magic=3, marker=1), pkg.Params(divisor=3, magic=0),
+              pkg.Params(divisor=5000, magic=4, marker=1, min_size=1000, max_size=20000)):
+        ch = pkg.Chunker(p)
+        assert ch.path == "generic"
+        check_chunk(ch, data)
