@@ -74,10 +74,11 @@ enum { SHRED_MARKER_EQ = 0, SHRED_MARKER_LE = 1 };
 
 /* Kernel paths the ctx selected for its parameters (shred_path). */
 enum {
-    SHRED_PATH_K63     = 1, /* deg(P) = 63, D <= 2^32: u64 state, TMA-staged, smem LDS.64 tables */
-    SHRED_PATH_K32     = 2, /* deg(P) = 32, D <= 2^32: u32 state, TMA-staged, smem LDS.32 tables */
-    SHRED_PATH_GENERIC = 3  /* any other valid parameters (other w or degree, D not a power of two,
-                               D > 2^32, SHRED_MARKER_LE): byte-at-a-time kernel              */
+    SHRED_PATH_K63     = 1, /* deg(P) = 63, w in {16,32,48,64}, D = 2^m <= 2^32 (either marker
+                               set): u64 state, TMA-staged, smem LDS.64 tables                  */
+    SHRED_PATH_K32     = 2, /* deg(P) = 32, same w / D / marker conditions: u32 state, LDS.32    */
+    SHRED_PATH_GENERIC = 3  /* any other valid parameters (other w or degree, D not a power of two
+                               or > 2^32): byte-at-a-time kernel                                */
 };
 
 /* Fill *p with the paper defaults (readings Q1, Q5, Q6, Q15): P = 0xbfe6b8a5bf378d83, w = 48,

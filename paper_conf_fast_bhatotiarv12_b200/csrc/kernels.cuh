@@ -398,11 +398,16 @@ template <> struct State<MODE_K32> {
 // marker test: (f mod D) == r  <=>  (f_lo << (32-m)) == (r << (32-m))   (D = 2^m <= 2^32)
 __device__ __forceinline__ bool is_marker(uint32_t lo, const BulkCtx &c) { return lo * c.tmul == c.rsh; }
 // m | BIT if marker else m: ISETP + predicated LOP3 (the PTX predication survives ptxas).
-template <uint32_t BIT>
+// LE: the "mod D <= r" marker set (L249-L251): (f_lo << (32-m)) <= (r << (32-m)).
+template <uint32_t BIT, bool LE>
 __device__ __forceinline__ uint32_t or_if_marker(uint32_t m, uint32_t lo, const BulkCtx &c) {
     const uint32_t x = lo * c.tmul;
-    asm("{\n .reg .pred p;\n setp.eq.u32 p, %1, %2;\n @p or.b32 %0, %0, %3;\n}"
-        : "+r"(m) : "r"(x), "r"(c.rsh), "n"(BIT));
+    if (LE)
+        asm("{\n .reg .pred p;\n setp.le.u32 p, %1, %2;\n @p or.b32 %0, %0, %3;\n}"
+            : "+r"(m) : "r"(x), "r"(c.rsh), "n"(BIT));
+    else
+        asm("{\n .reg .pred p;\n setp.eq.u32 p, %1, %2;\n @p or.b32 %0, %0, %3;\n}"
+            : "+r"(m) : "r"(x), "r"(c.rsh), "n"(BIT));
     return m;
 }
 // FMA-pipe form: 1 if NOT a marker.  y = (f_lo << (32-m)) - (r << (32-m)) is 0 iff marker;
@@ -437,11 +442,11 @@ __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t min_i,
 #elif SHRED_HITMODE == 2
 #define SHRED_MARK(ch, q) m[ch] = m[ch] * c.two + not_marker(st[ch].low(), c);
 #elif SHRED_HITMODE == 3
-#define SHRED_MARK(ch, q) m[ch] = or_if_marker<(1u << (4 * J + q))>(m[ch], st[ch].low(), c);
+#define SHRED_MARK(ch, q) m[ch] = or_if_marker<(1u << (4 * J + q)), LE>(m[ch], st[ch].low(), c);
 #else
 #define SHRED_MARK(ch, q) m[ch] |= (uint32_t)is_marker(st[ch].low(), c);
 #endif
-template <int MODE, int CH, bool TEST, int J>
+template <int MODE, int CH, bool TEST, int J, bool LE>
 __device__ __forceinline__ void word4xN(State<MODE> (&st)[CH], const uint32_t (&in)[CH],
                                         const uint32_t (&pop)[CH], uint32_t (&m)[CH], const BulkCtx &c) {
 #pragma unroll
@@ -473,7 +478,7 @@ __device__ __forceinline__ void word4xN(State<MODE> (&st)[CH], const uint32_t (&
 
 // 16 bytes of CH chains in one basic block (ILP across the chains): d = data chunk,
 // p = the chunk 48 bytes earlier (its bytes leave the window).
-template <int MODE, int CH, bool TEST>
+template <int MODE, int CH, bool TEST, bool LE>
 __device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d)[CH], const uint4 (&p)[CH],
                                           const BulkCtx &c, uint32_t (&m)[CH]) {
     uint32_t in[CH], po[CH];
@@ -481,16 +486,16 @@ __device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d
     for (int ch = 0; ch < CH; ++ch) m[ch] = 0;
 #pragma unroll
     for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].x; po[ch] = p[ch].x; }
-    word4xN<MODE, CH, TEST, 0>(st, in, po, m, c);
+    word4xN<MODE, CH, TEST, 0, LE>(st, in, po, m, c);
 #pragma unroll
     for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].y; po[ch] = p[ch].y; }
-    word4xN<MODE, CH, TEST, 1>(st, in, po, m, c);
+    word4xN<MODE, CH, TEST, 1, LE>(st, in, po, m, c);
 #pragma unroll
     for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].z; po[ch] = p[ch].z; }
-    word4xN<MODE, CH, TEST, 2>(st, in, po, m, c);
+    word4xN<MODE, CH, TEST, 2, LE>(st, in, po, m, c);
 #pragma unroll
     for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].w; po[ch] = p[ch].w; }
-    word4xN<MODE, CH, TEST, 3>(st, in, po, m, c);
+    word4xN<MODE, CH, TEST, 3, LE>(st, in, po, m, c);
 #if SHRED_HITMODE == 2
     // bit 15-j = "position j is not a marker" -> bit j = "position j is a marker"
     if (TEST) {
@@ -525,8 +530,9 @@ struct BulkConst { uint32_t mhi, m256, tmul, rsh, one; };
 // of a quarter warp read 8 consecutive rows' 16-byte chunks from 8 distinct bank groups:
 // SWIZZLE_32B for 32-byte rounds, no swizzle for 16-byte rounds).  The window is fixed at
 // w = 48 = 3 chunks of 16 B: the byte leaving the window at chunk q is the same byte slot of
-// chunk q-3, kept in a 4-slot register ring per chain (slot = chunk index mod 4).
-template <int MODE, class C>
+// chunk q-3, kept in a 4-slot register ring per chain (slot = chunk index mod 4).  WCH = w/16
+// (w in {16, 32, 48, 64}) generalises the pop distance; LE selects the "mod D <= r" marker set.
+template <int MODE, class C, int WCH, bool LE>
 __global__ void __launch_bounds__(C::NTC + 32, 1)
 k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_img,
         const GenTables *__restrict__ gt, Job J, DevParams P, BulkConst K) {
@@ -634,8 +640,8 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         for (int q = 0; q < 4; ++q) {
             uint4 d[CH], p[CH];
 #pragma unroll
-            for (int ch = 0; ch < CH; ++ch) { d[ch] = R[ch][q]; p[ch] = (q == 3) ? R[ch][0] : Z; }
-            chunk16xN<MODE, CH, false>(st, d, p, c, m);
+            for (int ch = 0; ch < CH; ++ch) { d[ch] = R[ch][q]; p[ch] = (q >= WCH) ? R[ch][q - WCH] : Z; }
+            chunk16xN<MODE, CH, false, LE>(st, d, p, c, m);
         }
     }
 
@@ -663,13 +669,13 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                 uint4 d[CH], p[CH];
                 uint32_t m[CH];
 #pragma unroll
-                for (int ch = 0; ch < CH; ++ch) { d[ch] = D[ch][u]; p[ch] = R[ch][(cq + 1) & 3]; }
+                for (int ch = 0; ch < CH; ++ch) { d[ch] = D[ch][u]; p[ch] = R[ch][(cq + 4 - WCH) & 3]; }
 #if SHRED_HITMODE == 1
                 State<MODE> s0[CH];
 #pragma unroll
                 for (int ch = 0; ch < CH; ++ch) s0[ch] = st[ch];
 #endif
-                chunk16xN<MODE, CH, true>(st, d, p, c, m);
+                chunk16xN<MODE, CH, true, LE>(st, d, p, c, m);
 #pragma unroll
                 for (int ch = 0; ch < CH; ++ch) {
                     R[ch][cq] = D[ch][u];

@@ -73,6 +73,28 @@ void byte_times_xpow(uint64_t P, int k, uint64_t e, uint64_t out[256]) {
     }
 }
 
+typedef void (*K1Fn)(const __grid_constant__ CUtensorMap, const uint4 *, const GenTables *, Job,
+                     DevParams, BulkConst);
+
+template <int MODE, class C>
+K1Fn pick_mode(int wch, bool le) {
+    switch (wch * 2 + (le ? 1 : 0)) {
+        case 2: return k1_bulk<MODE, C, 1, false>;
+        case 3: return k1_bulk<MODE, C, 1, true>;
+        case 4: return k1_bulk<MODE, C, 2, false>;
+        case 5: return k1_bulk<MODE, C, 2, true>;
+        case 6: return k1_bulk<MODE, C, 3, false>;
+        case 7: return k1_bulk<MODE, C, 3, true>;
+        case 8: return k1_bulk<MODE, C, 4, false>;
+        case 9: return k1_bulk<MODE, C, 4, true>;
+        default: return nullptr;
+    }
+}
+// The hot-kernel instance for (deg 63 | 32, w/16, marker set).
+K1Fn pick_k1(bool k63, int wch, bool le) {
+    return k63 ? pick_mode<MODE_K63, CfgK63>(wch, le) : pick_mode<MODE_K32, CfgK32>(wch, le);
+}
+
 typedef CUresult (*EncodeTiledFn)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *,
                                   const cuuint64_t *, const cuuint64_t *, const cuuint32_t *,
                                   const cuuint32_t *, CUtensorMapInterleave, CUtensorMapSwizzle,
@@ -93,6 +115,7 @@ struct shred_ctx {
     uint4 *d_tab_img = nullptr;          // 64 KiB replicated T|U image (fast paths)
     GenTables *d_gen = nullptr;          // plain T/U (generic path, recompute)
     EncodeTiledFn encode = nullptr;
+    K1Fn k1_fn = nullptr;                // the hot-kernel instance for these parameters
     int sm_count = 148;
 
     // scratch (grown on demand, synchronously)
@@ -301,12 +324,9 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
         K.one = 1u;
-        if (ctx->path == SHRED_PATH_K63)
-            k1_bulk<MODE_K63, CfgK63><<<pl.bulk_ctas, CfgK63::NTC + 32, CfgK63::SMEM, st>>>(
-                pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
-        else
-            k1_bulk<MODE_K32, CfgK32><<<pl.bulk_ctas, CfgK32::NTC + 32, CfgK32::SMEM, st>>>(
-                pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
+        const int smem = ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM;
+        const int threads = (ctx->path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC) + 32;
+        ctx->k1_fn<<<pl.bulk_ctas, threads, smem, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
         LAUNCHED("k1_bulk");
         if (e1) CK(cudaEventRecord(e1, st), "profile record");
     } else {
@@ -487,7 +507,8 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     ctx->dp.pow2 = (p->divisor & (p->divisor - 1)) == 0 ? 1u : 0u;
     ctx->dp.marker = p->marker;
     const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
-    const bool fast = (p->window == 48) && pow2 && p->divisor <= (1ull << 32) && p->marker == SHRED_MARKER_EQ;
+    const bool fast_w = p->window == 16 || p->window == 32 || p->window == 48 || p->window == 64;
+    const bool fast = fast_w && pow2 && p->divisor <= (1ull << 32);
     if (k == 63 && fast) ctx->path = SHRED_PATH_K63;
     else if (k == 32 && fast) ctx->path = SHRED_PATH_K32;
     else ctx->path = SHRED_PATH_GENERIC;
@@ -541,8 +562,10 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fn, cudaEnableDefault, &q) != cudaSuccess || !fn)
             return bail(SHRED_ECUDA);
         ctx->encode = (EncodeTiledFn)fn;
-        if (cudaFuncSetAttribute(k1_bulk<MODE_K63, CfgK63>, cudaFuncAttributeMaxDynamicSharedMemorySize, CfgK63::SMEM) != cudaSuccess ||
-            cudaFuncSetAttribute(k1_bulk<MODE_K32, CfgK32>, cudaFuncAttributeMaxDynamicSharedMemorySize, CfgK32::SMEM) != cudaSuccess)
+        ctx->k1_fn = pick_k1(ctx->path == SHRED_PATH_K63, (int)(p->window / 16), p->marker == SHRED_MARKER_LE);
+        if (!ctx->k1_fn ||
+            cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                 ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM) != cudaSuccess)
             return bail(SHRED_ECUDA);
     }
     if (cudaFuncSetAttribute(sb_dense, cudaFuncAttributeMaxDynamicSharedMemorySize,

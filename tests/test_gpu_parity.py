@@ -101,8 +101,8 @@ def test_k32_path(pkg):
 
 
 def test_generic_path_variants(pkg):
-    for p in (pkg.Params(window=32), pkg.Params(window=1, divisor=256, magic=7),
-              pkg.Params(poly=(1 << 63) | 3, window=16, divisor=1024),
+    for p in (pkg.Params(window=33), pkg.Params(window=1, divisor=256, magic=7),
+              pkg.Params(poly=(1 << 63) | 3, window=24, divisor=1024),
               pkg.Params(poly=0x11D, window=7, divisor=64, magic=9),
               pkg.Params(divisor=1 << 40, magic=12345)):
         ch = pkg.Chunker(p)
@@ -254,9 +254,21 @@ def test_marker_le_and_non_pow2_divisor(pkg):
     """The "value mod p <= constant" marker set (L249-L251) and divisors that are not powers of
     two run on the generic path, bit-exact vs the oracle; bounded mode on top."""
     data = synthgen.random_bytes(31, (2 << 20) + 77)
-    for p in (pkg.Params(divisor=10000, magic=1234), pkg.Params(divisor=8192, magic=1, marker=1),
+    for p in (pkg.Params(divisor=10000, magic=1234),
               pkg.Params(divisor=12345, magic=3, marker=1), pkg.Params(divisor=3, magic=0),
               pkg.Params(divisor=5000, magic=4, marker=1, min_size=1000, max_size=20000)):
         ch = pkg.Chunker(p)
         assert ch.path == "generic"
         check_chunk(ch, data)
+
+
+@pytest.mark.parametrize("poly,path", [(LBFS, "k63"), (0x104C11DB7, "k32")])
+@pytest.mark.parametrize("window", [16, 32, 48, 64])
+@pytest.mark.parametrize("marker", [0, 1])
+def test_fast_path_windows_and_le_marker(pkg, poly, path, window, marker):
+    """The hot kernel's instances: w in {16,32,48,64} x {==, <=} marker sets, both degrees."""
+    D, r = (4096, 9) if marker else (1024, 77)
+    p = pkg.Params(poly=poly, window=window, divisor=D, magic=r, marker=marker)
+    ch = pkg.Chunker(p)
+    assert ch.path == path
+    check_chunk(ch, synthgen.random_bytes(window + marker, (3 << 20) + 31), offset=5)
