@@ -307,7 +307,12 @@ def main():
             "scaling": "weak", "vs_baseline": None, "dtype": "u8", "data": "synthetic",
             "config": config(world, per_rank_bytes), "hbm_frac": round(value / world / hbm, 4),
             "roofline": roofline, "clocks": clk.result(), "gpu_launches": launches,
-            "candidates_rank0": n_cand}
+            "candidates_rank0": n_cand,
+            "paper_context": {"note": "PAPER.md numbers on other hardware: context only, not a target",
+                              "gpu": "full Shredder <= 2.5 GB/s (Fig. 12 axis, L1016-L1037), Tesla C2050 "
+                                     "(Fermi, 144 GB/s GDDR5), CUDA 4.0",
+                              "gpu_device_time": "16-256 MB buffers in 11.39-171.4 ms = 1.47-1.57 GB/s (Table 2, L766-L770)",
+                              "cpu_ratio": "GPU > 5x the 12-thread pthreads chunker on 2x Xeon X5650 (L88-L90, L1100-L1102)"}}
 
     # ---- e2e: host-fed through the C ABI (pinned host -> shred_feed -> flush -> D2H)
     if not args.no_e2e:
