@@ -146,6 +146,17 @@ int shred_reset(shred_ctx *ctx);
    each (default 2 x 256 MiB, allocated at the first host feed).  Only between streams. */
 int shred_set_ring(shred_ctx *ctx, int slots, uint64_t slot_bytes);
 
+/* Hashing (dedup step 2: "computing a collision-resistant
+   hash of the chunk"): SHA-256 (FIPS 180-4; the paper names no function) of every chunk of
+   d_in[0..len) delimited by the ascending cuts d_cuts[0 .. *d_ncuts) (e.g. shred_chunk's output,
+   chained on the same stream without a host round trip): chunks [0,c0), [c0,c1), ...,
+   [c_{n-1}, len), i.e. n+1 chunks (none if len = 0).  d_ncuts is device memory or mapped
+   pinned memory; d_cuts must hold all *d_ncuts cuts.  Writes 32 digest bytes per chunk to
+   d_digests (16-byte aligned) for at most max_chunks chunks. */
+int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const uint64_t *d_cuts,
+                      const uint64_t *d_ncuts, uint8_t *d_digests, uint64_t max_chunks,
+                      shred_stream_t stream);
+
 /* Bench/test helper (not the method): writes bytes [offset, offset+len) of the counter-mode
    SplitMix64 stream `seed` into d_buf on `stream`. */
 int shred_synth_fill(uint8_t *d_buf, uint64_t len, uint64_t seed, uint64_t offset,

@@ -17,6 +17,7 @@ Functions (each cites the passage it follows; readings Q1..Q17 are listed in DES
 * :func:`size_bound` — min/max rule (L259-L269, Q12-Q15).
 * :func:`chunk` — candidates then size rule: the final cut offsets.
 * :func:`is_irreducible` — Rabin's irreducibility test for ``div(x)`` (L255-L256).
+* :func:`chunk_digests` — SHA-256 of every chunk (dedup step 2, L229-L238; §8(f) f2).
 
 Parity status: every function is pinned (tests/test_oracle.py); parity with the *paper's own*
 implementation is unpinned because the paper prints no fingerprint, polynomial or boundary.
@@ -180,6 +181,22 @@ def chunk(data, p: Params = Params(), method: int = 2, threads: int | None = Non
     if p.min_size == 0 and p.max_size == 0:
         return c
     return size_bound(c, a.size, p.min_size, p.max_size)
+
+
+def chunk_digests(data, cuts) -> np.ndarray:
+    """SHA-256 of every chunk [0,c0), [c0,c1), ..., [c_{n-1}, N) (dedup step 2, PAPER.md
+    L229-L238).  The library routine hashlib.sha256 is the step (pinned by the
+    FIPS 180 vectors in tests/golden/sha256_fips180.txt).  Returns (n+1, 32) uint8."""
+    import hashlib
+    a = _bytes(data)
+    if a.size == 0:
+        return np.zeros((0, 32), dtype=np.uint8)
+    bounds = [0] + [int(c) for c in cuts] + [a.size]
+    out = np.zeros((len(bounds) - 1, 32), dtype=np.uint8)
+    mv = memoryview(a)
+    for k in range(len(bounds) - 1):
+        out[k] = np.frombuffer(hashlib.sha256(mv[bounds[k]:bounds[k + 1]]).digest(), dtype=np.uint8)
+    return out
 
 
 def is_irreducible(poly: int) -> bool:

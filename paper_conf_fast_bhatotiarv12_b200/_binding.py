@@ -78,6 +78,7 @@ def lib() -> ctypes.CDLL:
             "shred_set_ring": (cint, [vp, cint, u64]),
             "shred_synth_fill": (cint, [vp, u64, u64, u64, vp]),
             "shred_launch_count": (u64, [vp]),
+            "shred_hash_chunks": (cint, [vp, vp, u64, vp, vp, vp, u64, vp]),
             "shred_profile": (cint, [vp, cint]),
             "shred_profile_read": (cint, [vp, ctypes.POINTER(ctypes.c_double), ctypes.POINTER(u64),
                                           ctypes.POINTER(u64)]),
@@ -218,6 +219,25 @@ class Chunker:
         if n > cap:
             raise ShredError(f"capacity {cap} < {n} cuts")
         return out[:n]
+
+    # ---------------------------------------------------------------- hashing (f2)
+    def hash_chunks_async(self, x: torch.Tensor, cuts: torch.Tensor, n_cuts: torch.Tensor,
+                          digests: torch.Tensor, stream=None) -> None:
+        """Enqueue SHA-256 of every chunk delimited by cuts[:n_cuts[0]] (device count)."""
+        assert x.is_cuda and x.dtype == torch.uint8 and x.is_contiguous()
+        assert digests.dtype == torch.uint8 and digests.is_contiguous() and digests.numel() % 32 == 0
+        rc = lib().shred_hash_chunks(self._ctx, x.data_ptr(), x.numel(), cuts.data_ptr(), n_cuts.data_ptr(),
+                                     digests.data_ptr(), digests.numel() // 32, _stream(stream))
+        self._check(rc, "shred_hash_chunks")
+
+    def hash_chunks(self, x: torch.Tensor, cuts: torch.Tensor) -> torch.Tensor:
+        """(len(cuts)+1, 32) uint8 SHA-256 digests of the chunks of x (synchronises)."""
+        n = torch.tensor([cuts.numel()], dtype=torch.int64, device=x.device)
+        out = torch.empty((cuts.numel() + 1) * 32 if x.numel() else 32, dtype=torch.uint8, device=x.device)
+        c = cuts.contiguous() if cuts.numel() else torch.zeros(1, dtype=torch.int64, device=x.device)
+        self.hash_chunks_async(x, c, n, out)
+        torch.cuda.current_stream().synchronize()
+        return out.view(-1, 32)[: (cuts.numel() + 1) if x.numel() else 0]
 
     # ---------------------------------------------------------------- streaming
     def feed_async(self, x: torch.Tensor, out: torch.Tensor, n_out: torch.Tensor, stream=None) -> None:

@@ -1,0 +1,137 @@
+// sha256.cuh — hashing every chunk (dedup step 2,
+// "Hashing: This is the process of computing a collision-resistant hash of the chunk").
+//
+// The paper names no hash function; SHA-256 (FIPS 180-4) is used (reading H1).
+// Chunks are [0, c_0), [c_0, c_1), ..., [c_{n-1}, len): n cuts give n+1 chunks (len > 0).
+//
+// k_hash_chunks: one lane hashes one chunk at a time (Merkle-Damgard is sequential inside a
+// chunk).  Chunk sizes are roughly exponential, so a static chunk-per-lane assignment would
+// leave most lanes of a warp idle while the longest chunk finishes; instead each lane pulls its
+// next chunk from a global queue (one warp-aggregated atomic) as soon as its current one is
+// done, and the warp stays converged on the 64-round compression loop.  Full blocks are
+// loaded as 17 aligned words realigned with funnel shifts; the last one or two blocks of a
+// chunk (0x80 padding + 64-bit length) take a byte-wise path.
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+namespace shred {
+
+__constant__ uint32_t kSha256K[64] = {
+    0x428a2f98u, 0x71374491u, 0xb5c0fbcfu, 0xe9b5dba5u, 0x3956c25bu, 0x59f111f1u, 0x923f82a4u, 0xab1c5ed5u,
+    0xd807aa98u, 0x12835b01u, 0x243185beu, 0x550c7dc3u, 0x72be5d74u, 0x80deb1feu, 0x9bdc06a7u, 0xc19bf174u,
+    0xe49b69c1u, 0xefbe4786u, 0x0fc19dc6u, 0x240ca1ccu, 0x2de92c6fu, 0x4a7484aau, 0x5cb0a9dcu, 0x76f988dau,
+    0x983e5152u, 0xa831c66du, 0xb00327c8u, 0xbf597fc7u, 0xc6e00bf3u, 0xd5a79147u, 0x06ca6351u, 0x14292967u,
+    0x27b70a85u, 0x2e1b2138u, 0x4d2c6dfcu, 0x53380d13u, 0x650a7354u, 0x766a0abbu, 0x81c2c92eu, 0x92722c85u,
+    0xa2bfe8a1u, 0xa81a664bu, 0xc24b8b70u, 0xc76c51a3u, 0xd192e819u, 0xd6990624u, 0xf40e3585u, 0x106aa070u,
+    0x19a4c116u, 0x1e376c08u, 0x2748774cu, 0x34b0bcb5u, 0x391c0cb3u, 0x4ed8aa4au, 0x5b9cca4fu, 0x682e6ff3u,
+    0x748f82eeu, 0x78a5636fu, 0x84c87814u, 0x8cc70208u, 0x90befffau, 0xa4506cebu, 0xbef9a3f7u, 0xc67178f2u};
+
+__device__ __forceinline__ uint32_t rotr(uint32_t x, int n) { return __funnelshift_r(x, x, n); }
+
+// One SHA-256 compression of the 16 big-endian words W into H.
+__device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[16]) {
+    uint32_t a = H[0], b = H[1], c = H[2], d = H[3], e = H[4], f = H[5], g = H[6], h = H[7];
+#pragma unroll
+    for (int t = 0; t < 64; ++t) {
+        uint32_t w;
+        if (t < 16) {
+            w = W[t];
+        } else {
+            const uint32_t w15 = W[(t - 15) & 15], w2 = W[(t - 2) & 15];
+            const uint32_t s0 = rotr(w15, 7) ^ rotr(w15, 18) ^ (w15 >> 3);
+            const uint32_t s1 = rotr(w2, 17) ^ rotr(w2, 19) ^ (w2 >> 10);
+            w = W[t & 15] = W[t & 15] + s0 + W[(t - 7) & 15] + s1;
+        }
+        const uint32_t S1 = rotr(e, 6) ^ rotr(e, 11) ^ rotr(e, 25);
+        const uint32_t ch = (e & f) ^ (~e & g);
+        const uint32_t t1 = h + S1 + ch + kSha256K[t] + w;
+        const uint32_t S0 = rotr(a, 2) ^ rotr(a, 13) ^ rotr(a, 22);
+        const uint32_t mj = (a & b) ^ (a & c) ^ (b & c);
+        const uint32_t t2 = S0 + mj;
+        h = g; g = f; f = e; e = d + t1; d = c; c = b; b = a; a = t1 + t2;
+    }
+    H[0] += a; H[1] += b; H[2] += c; H[3] += d; H[4] += e; H[5] += f; H[6] += g; H[7] += h;
+}
+
+__device__ __forceinline__ void sha256_init(uint32_t (&H)[8]) {
+    H[0] = 0x6a09e667u; H[1] = 0xbb67ae85u; H[2] = 0x3c6ef372u; H[3] = 0xa54ff53au;
+    H[4] = 0x510e527fu; H[5] = 0x9b05688cu; H[6] = 0x1f83d9abu; H[7] = 0x5be0cd19u;
+}
+
+// Block `blk` of the padded message of chunk [a, a+L) (L bytes) into big-endian words W.
+__device__ __forceinline__ void sha256_block(const uint8_t *__restrict__ in, uint64_t in_len, uint64_t a,
+                                             uint64_t L, uint64_t blk, uint32_t (&W)[16]) {
+    const uint64_t m0 = blk * 64;                     // message offset of the block
+    const uint64_t p = a + m0;                        // stream position
+    const uint64_t wa = p & ~3ull;                    // aligned word start
+    if (m0 + 64 <= L && wa + 68 <= in_len) {          // full block, 17 aligned words in bounds
+        const uint32_t *src = reinterpret_cast<const uint32_t *>(in + wa);
+        const uint32_t sh = (uint32_t)(p & 3) * 8;
+        uint32_t prev = __ldg(src);
+#pragma unroll
+        for (int k = 0; k < 16; ++k) {
+            const uint32_t nxt = __ldg(src + k + 1);
+            const uint32_t le = __funnelshift_r(prev, nxt, sh);   // 4 stream bytes, little-endian
+            W[k] = __byte_perm(le, 0, 0x0123);                    // big-endian word
+            prev = nxt;
+        }
+        return;
+    }
+    const uint64_t nblk = (L + 9 + 63) / 64;          // blocks of the padded message
+    const uint64_t lenpos = nblk * 64 - 8;            // where the 64-bit bit length starts
+    const uint64_t bits = L * 8;
+#pragma unroll 1
+    for (int k = 0; k < 16; ++k) {
+        uint32_t v = 0;
+        for (int q = 0; q < 4; ++q) {
+            const uint64_t m = m0 + 4 * k + q;
+            uint32_t byte;
+            if (m < L) byte = in[a + m];
+            else if (m == L) byte = 0x80u;
+            else if (m >= lenpos) byte = (uint32_t)(bits >> (8 * (7 - (m - lenpos)))) & 0xFFu;
+            else byte = 0;
+            v = (v << 8) | byte;
+        }
+        W[k] = v;
+    }
+}
+
+// Hash every chunk.  nchunks = (*n_cuts + 1 if len > 0 else 0); chunk i ends at cuts[i]
+// (i < n) or len.  digests: 32 bytes per chunk (the SHA-256 digest bytes in order).
+// `queue` must be 0 at launch (the host zeroes it).
+__global__ void __launch_bounds__(256)
+k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__restrict__ cuts,
+              const uint64_t *n_cuts, uint64_t max_chunks, uint8_t *__restrict__ digests,
+              unsigned long long *queue) {
+    const uint64_t ncut = *n_cuts;
+    const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
+    uint32_t H[8], W[16];
+    uint64_t chunk = 0, a = 0, L = 0, blk = 0, nblk = 0;
+    bool have = false;
+    while (true) {
+        if (!have) {
+            chunk = atomicAdd(queue, 1ull);
+            if (chunk >= nc) break;
+            a = chunk ? cuts[chunk - 1] : 0;
+            const uint64_t b = chunk < ncut ? cuts[chunk] : len;
+            L = b - a;
+            blk = 0;
+            nblk = (L + 9 + 63) / 64;
+            sha256_init(H);
+            have = true;
+        }
+        sha256_block(in, len, a, L, blk, W);
+        sha256_compress(H, W);
+        if (++blk == nblk) {
+            uint4 *o = reinterpret_cast<uint4 *>(digests + chunk * 32);
+            o[0] = make_uint4(__byte_perm(H[0], 0, 0x0123), __byte_perm(H[1], 0, 0x0123),
+                              __byte_perm(H[2], 0, 0x0123), __byte_perm(H[3], 0, 0x0123));
+            o[1] = make_uint4(__byte_perm(H[4], 0, 0x0123), __byte_perm(H[5], 0, 0x0123),
+                              __byte_perm(H[6], 0, 0x0123), __byte_perm(H[7], 0, 0x0123));
+            have = false;
+        }
+    }
+}
+
+}  // namespace shred

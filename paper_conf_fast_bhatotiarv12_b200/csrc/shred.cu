@@ -8,6 +8,7 @@
 // runs in the kernels of kernels.cuh.
 #include "kernels.cuh"
 #include "size_bound.cuh"
+#include "sha256.cuh"
 #include "../../include/shred.h"
 
 #include <cstdarg>
@@ -127,6 +128,7 @@ struct shred_ctx {
     uint64_t *d_sb = nullptr; uint64_t sb_cap = 0;             // size-rule block scratch
     Aux *d_aux = nullptr;                // [0] one-shot calls, [1] the stream
     uint64_t *h_pinned = nullptr;        // small pinned readback area
+    unsigned long long *d_queue = nullptr;   // work queue of k_hash_chunks
     uint64_t *h_flag = nullptr;          // mapped pinned word: a streaming call overflowed
     uint64_t *d_flag = nullptr;          // its device alias
 
@@ -545,6 +547,7 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         cudaMalloc(&ctx->d_aux, 2 * sizeof(Aux)) != cudaSuccess ||
         cudaMalloc(&ctx->d_carry[0], 4096) != cudaSuccess ||
         cudaMalloc(&ctx->d_carry[1], 4096) != cudaSuccess ||
+        cudaMalloc(&ctx->d_queue, 64) != cudaSuccess ||
         cudaHostAlloc(&ctx->h_pinned, 64, cudaHostAllocDefault) != cudaSuccess ||
         cudaHostAlloc(&ctx->h_flag, 64, cudaHostAllocMapped) != cudaSuccess ||
         cudaHostGetDevicePointer((void **)&ctx->d_flag, ctx->h_flag, 0) != cudaSuccess) {
@@ -590,7 +593,7 @@ void shred_destroy(shred_ctx *ctx) {
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
     cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_counts); cudaFree(ctx->d_local); cudaFree(ctx->d_groups);
     cudaFree(ctx->d_scratch); cudaFree(ctx->d_cand); cudaFree(ctx->d_sb); cudaFree(ctx->d_aux);
-    cudaFree(ctx->d_carry[0]); cudaFree(ctx->d_carry[1]);
+    cudaFree(ctx->d_carry[0]); cudaFree(ctx->d_carry[1]); cudaFree(ctx->d_queue);
     if (ctx->h_pinned) cudaFreeHost(ctx->h_pinned);
     if (ctx->h_flag) cudaFreeHost(ctx->h_flag);
     cudaGetLastError();
@@ -794,6 +797,24 @@ int shred_reset(shred_ctx *ctx) {
     cudaDeviceSynchronize();
     ctx->pos = 0; ctx->carry_len = 0; ctx->carry_idx = 0; ctx->sticky = SHRED_OK;
     ctx->h_flag[0] = 0;
+    return SHRED_OK;
+}
+
+int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const uint64_t *d_cuts,
+                      const uint64_t *d_ncuts, uint8_t *d_digests, uint64_t max_chunks,
+                      shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    if (!d_ncuts || (len && !d_in) || (max_chunks && !d_digests))
+        return fail(ctx, SHRED_EINVAL, "null pointer");
+    if (((uintptr_t)d_digests & 15u) != 0) return fail(ctx, SHRED_EINVAL, "d_digests must be 16-byte aligned");
+    if (!len || !max_chunks) return SHRED_OK;
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    k_write_u64<<<1, 1, 0, st>>>((uint64_t *)ctx->d_queue, 0);
+    LAUNCHED("k_write_u64");
+    k_hash_chunks<<<ctx->sm_count * 4, 256, 0, st>>>(d_in, len, d_cuts, d_ncuts, max_chunks, d_digests,
+                                                      ctx->d_queue);
+    LAUNCHED("k_hash_chunks");
     return SHRED_OK;
 }
 

@@ -1,0 +1,59 @@
+"""f2: SHA-256 of every chunk on the GPU vs the oracle (hashlib per chunk, FIPS-180-pinned)."""
+import numpy as np
+import pytest
+import torch
+
+import oracle
+import synthgen
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def pkg():
+    import paper_conf_fast_bhatotiarv12_b200 as P
+    return P
+
+
+def test_padding_edge_lengths(pkg):
+    """Chunk lengths around the 55/56/64-byte padding edges, 1-byte chunks, unaligned starts."""
+    lens = [1, 1, 2, 3, 54, 55, 56, 57, 63, 64, 65, 119, 120, 121, 127, 128, 129, 1000, 4095, 4096, 4097]
+    rng = np.random.default_rng(3)
+    lens = lens + [int(x) for x in rng.integers(1, 3000, 200)]
+    cuts = np.cumsum(lens)[:-1]
+    n = int(np.sum(lens))
+    data = synthgen.random_bytes(5, n)
+    ch = pkg.Chunker(pkg.Params())
+    got = ch.hash_chunks(torch.from_numpy(data).cuda(), torch.from_numpy(cuts.astype(np.int64)).cuda())
+    exp = oracle.chunk_digests(data, cuts)
+    assert np.array_equal(got.cpu().numpy(), exp)
+
+
+def test_single_chunk_and_fips_message(pkg):
+    ch = pkg.Chunker(pkg.Params())
+    for m in (b"abc", b"abcdbcdecdefdefgefghfghighijhijkijkljklmklmnlmnomnopnopq", b"a" * 1000000):
+        x = torch.frombuffer(bytearray(m), dtype=torch.uint8).cuda()
+        got = ch.hash_chunks(x, torch.zeros(0, dtype=torch.int64).cuda())
+        assert got.shape == (1, 32)
+        assert np.array_equal(got.cpu().numpy(), oracle.chunk_digests(np.frombuffer(m, np.uint8), []))
+
+
+@pytest.mark.parametrize("bounded", [False, True])
+def test_chunk_then_hash_on_device(pkg, bounded):
+    """Chunking -> hashing chained on one stream (the cut count never leaves the device)."""
+    n = (8 << 20) + 333
+    data = synthgen.random_bytes(7, n)
+    p = pkg.Params(divisor=2048, min_size=512 if bounded else 0, max_size=16384 if bounded else 0)
+    ch = pkg.Chunker(p)
+    x = torch.from_numpy(data).cuda()
+    cuts = torch.empty(n // 256, dtype=torch.int64, device="cuda")
+    ncut = torch.zeros(1, dtype=torch.int64, device="cuda")
+    dig = torch.empty(n // 256 * 32, dtype=torch.uint8, device="cuda")
+    ch.chunk_async(x, cuts, ncut)
+    ch.hash_chunks_async(x, cuts, ncut, dig)
+    torch.cuda.synchronize()
+    k = int(ncut.item())
+    c = cuts[:k].cpu().numpy()
+    assert np.array_equal(c.astype(np.uint64), oracle.chunk(data, oracle.Params(divisor=2048, min_size=p.min_size,
+                                                                                 max_size=p.max_size)))
+    assert np.array_equal(dig[:(k + 1) * 32].view(-1, 32).cpu().numpy(), oracle.chunk_digests(data, c))

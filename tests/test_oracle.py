@@ -334,3 +334,25 @@ def test_le_marker_density():
         k = oracle.candidates(data, Params(divisor=D, magic=r, marker=1)).size
         mu = (n - 48) * (r + 1) / D
         assert abs(k - mu) <= 4 * np.sqrt(mu)
+
+
+# --------------------------------------------------------------------------- hashing (f2)
+def test_sha256_oracle_fips180_vectors(golden_dir):
+    import hashlib
+    rows = _golden(golden_dir, "sha256_fips180.txt")
+    msgs = {"EMPTY": b"", "MILLION_A": b"a" * 1000000}
+    for spec, digest in rows:
+        m = msgs.get(spec, spec.encode())
+        assert hashlib.sha256(m).hexdigest() == digest
+        # through the chunk interface: one chunk = the whole message
+        if m:
+            assert oracle.chunk_digests(np.frombuffer(m, np.uint8), [])[0].tobytes().hex() == digest
+
+
+def test_chunk_digests_boundaries():
+    data = synthgen.random_bytes(3, 1000)
+    d = oracle.chunk_digests(data, [10, 500, 999])
+    assert d.shape == (4, 32)
+    import hashlib
+    assert d[1].tobytes() == hashlib.sha256(data[10:500].tobytes()).digest()
+    assert d[3].tobytes() == hashlib.sha256(data[999:].tobytes()).digest()
