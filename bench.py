@@ -403,6 +403,25 @@ def main():
             v32 = timed(c32, base)
             line["k32_variant"] = {"value": round(v32, 2), "unit": "GB/s", "hbm_frac": round(v32 / hbm, 4),
                                    "params": "P=0x104C11DB7 (deg 32, irreducible), other params as paper"}
+            # f2: SHA-256 of every chunk, alone and chained after chunking (no host round trip)
+            dig = torch.empty((cap + 1) * 32, dtype=torch.uint8, device=dev)
+            ch.chunk_async(base, out0, n0)
+            ch.hash_chunks_async(base, out0, n0, dig)
+            torch.cuda.synchronize()
+            h0, h1, h2 = (torch.cuda.Event(enable_timing=True) for _ in range(3))
+            h0.record(stream)
+            for _ in range(3):
+                ch.hash_chunks_async(base, out0, n0, dig)
+            h1.record(stream)
+            for _ in range(3):
+                ch.chunk_async(base, out0, n0)
+                ch.hash_chunks_async(base, out0, n0, dig)
+            h2.record(stream)
+            torch.cuda.synchronize()
+            line["hash_sha256"] = {"value": round(3 * base.numel() / (h0.elapsed_time(h1) * 1e-3) / 1e9, 2),
+                                   "unit": "GB/s", "chunks": int(n0.item()) + 1,
+                                   "chunk_plus_hash": round(3 * base.numel() / (h1.elapsed_time(h2) * 1e-3) / 1e9, 2),
+                                   "note": "SURVEY §8(f) f2: SHA-256 per chunk of the 1 GiB base file"}
         except Exception as e:  # side numbers must never break the headline line
             line["extra_error"] = repr(e)
 

@@ -4,16 +4,17 @@
 // The paper names no hash function; SHA-256 (FIPS 180-4) is used (reading H1).
 // Chunks are [0, c_0), [c_0, c_1), ..., [c_{n-1}, len): n cuts give n+1 chunks (len > 0).
 //
-// k_hash_chunks: one lane hashes one chunk at a time (Merkle-Damgard is sequential inside a
-// chunk).  Chunk sizes are roughly exponential, so a static chunk-per-lane assignment would
-// leave most lanes of a warp idle while the longest chunk finishes; instead each lane pulls its
-// next chunk from a global queue (one warp-aggregated atomic) as soon as its current one is
-// done, and the warp stays converged on the 64-round compression loop.  Full blocks are
-// loaded as 17 aligned words realigned with funnel shifts; the last one or two blocks of a
-// chunk (0x80 padding + 64-bit length) take a byte-wise path.
+// k_hash_chunks: one lane hashes one chunk (Merkle-Damgard is sequential inside a chunk).
+// Chunk sizes are roughly exponential, so chunks are first counting-sorted by length
+// (k_hash_hist / k_hash_scan / k_hash_scatter, 128-byte buckets, longest first) and warps take
+// 32 consecutive sorted chunks at a time: the lanes of a warp have near-equal lengths and the
+// longest chunks start first (LPT).  Full blocks are loaded as 17 aligned words realigned with
+// funnel shifts; the last one or two blocks of a chunk (0x80 padding + 64-bit length) take a
+// byte-wise path.
 #pragma once
 #include <cstdint>
 #include <cuda_runtime.h>
+#include "kernels.cuh"
 
 namespace shred {
 
@@ -97,40 +98,89 @@ __device__ __forceinline__ void sha256_block(const uint8_t *__restrict__ in, uin
     }
 }
 
+// ---- length-sorted work list (LPT): chunk sizes are ~exponential, so lanes of one warp must
+// hash chunks of similar length or the warp idles on its longest lane.  A counting sort by
+// length bucket (descending) makes warps take 32 consecutive similar-length chunks, longest
+// first.
+constexpr int HB = 1024;                 // length buckets of 128 bytes; the last holds >= 128 KiB
+
+__device__ __forceinline__ uint32_t hash_bucket(uint64_t L) {
+    const uint64_t k = L >> 7;
+    return (uint32_t)(HB - 1 - (k < (uint64_t)(HB - 1) ? k : (uint64_t)(HB - 1)));   // descending
+}
+
+__device__ __forceinline__ void chunk_bounds(const uint64_t *cuts, uint64_t ncut, uint64_t len, uint64_t i,
+                                             uint64_t &a, uint64_t &b) {
+    a = i ? cuts[i - 1] : 0;
+    b = i < ncut ? cuts[i] : len;
+}
+
+__global__ void k_hash_hist(const uint64_t *__restrict__ cuts, const uint64_t *n_cuts, uint64_t len,
+                            uint64_t max_chunks, uint32_t *hist) {
+    const uint64_t ncut = *n_cuts;
+    const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nc; i += (uint64_t)gridDim.x * blockDim.x) {
+        uint64_t a, b;
+        chunk_bounds(cuts, ncut, len, i, a, b);
+        atomicAdd(&hist[hash_bucket(b - a)], 1u);
+    }
+}
+
+// One CTA: exclusive scan of the HB bucket counts (in place) and reset of the work queue.
+__global__ void __launch_bounds__(HB) k_hash_scan(uint32_t *hist, unsigned long long *queue) {
+    __shared__ uint32_t ws[33];
+    const uint32_t v = hist[threadIdx.x];
+    uint32_t tot;
+    const uint32_t off = block_exscan(v, HB, 1, ws, &tot);
+    hist[threadIdx.x] = off;
+    if (threadIdx.x == 0) *queue = 0;
+}
+
+__global__ void k_hash_scatter(const uint64_t *__restrict__ cuts, const uint64_t *n_cuts, uint64_t len,
+                               uint64_t max_chunks, uint32_t *offs, uint32_t *order) {
+    const uint64_t ncut = *n_cuts;
+    const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nc; i += (uint64_t)gridDim.x * blockDim.x) {
+        uint64_t a, b;
+        chunk_bounds(cuts, ncut, len, i, a, b);
+        order[atomicAdd(&offs[hash_bucket(b - a)], 1u)] = (uint32_t)i;
+    }
+}
+
 // Hash every chunk.  nchunks = (*n_cuts + 1 if len > 0 else 0); chunk i ends at cuts[i]
 // (i < n) or len.  digests: 32 bytes per chunk (the SHA-256 digest bytes in order).
-// `queue` must be 0 at launch (the host zeroes it).
+// Warps take 32 consecutive entries of the length-sorted `order` at a time from `queue`.
 __global__ void __launch_bounds__(256)
 k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__restrict__ cuts,
               const uint64_t *n_cuts, uint64_t max_chunks, uint8_t *__restrict__ digests,
-              unsigned long long *queue) {
+              const uint32_t *__restrict__ order, unsigned long long *queue) {
     const uint64_t ncut = *n_cuts;
     const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
+    const int lane = threadIdx.x & 31;
     uint32_t H[8], W[16];
-    uint64_t chunk = 0, a = 0, L = 0, blk = 0, nblk = 0;
-    bool have = false;
     while (true) {
-        if (!have) {
-            chunk = atomicAdd(queue, 1ull);
-            if (chunk >= nc) break;
-            a = chunk ? cuts[chunk - 1] : 0;
-            const uint64_t b = chunk < ncut ? cuts[chunk] : len;
-            L = b - a;
-            blk = 0;
-            nblk = (L + 9 + 63) / 64;
+        unsigned long long base = 0;
+        if (lane == 0) base = atomicAdd(queue, 32ull);
+        base = __shfl_sync(0xffffffffu, base, 0);
+        if (base >= nc) break;
+        const uint64_t j = base + (uint64_t)lane;
+        if (j < nc) {
+            const uint64_t chunk = order[j];
+            uint64_t a, b;
+            chunk_bounds(cuts, ncut, len, chunk, a, b);
+            const uint64_t L = b - a, nblk = (L + 9 + 63) / 64;
             sha256_init(H);
-            have = true;
-        }
-        sha256_block(in, len, a, L, blk, W);
-        sha256_compress(H, W);
-        if (++blk == nblk) {
+            for (uint64_t blk = 0; blk < nblk; ++blk) {
+                sha256_block(in, len, a, L, blk, W);
+                sha256_compress(H, W);
+            }
             uint4 *o = reinterpret_cast<uint4 *>(digests + chunk * 32);
             o[0] = make_uint4(__byte_perm(H[0], 0, 0x0123), __byte_perm(H[1], 0, 0x0123),
                               __byte_perm(H[2], 0, 0x0123), __byte_perm(H[3], 0, 0x0123));
             o[1] = make_uint4(__byte_perm(H[4], 0, 0x0123), __byte_perm(H[5], 0, 0x0123),
                               __byte_perm(H[6], 0, 0x0123), __byte_perm(H[7], 0, 0x0123));
-            have = false;
         }
+        __syncwarp();
     }
 }
 

@@ -129,6 +129,8 @@ struct shred_ctx {
     Aux *d_aux = nullptr;                // [0] one-shot calls, [1] the stream
     uint64_t *h_pinned = nullptr;        // small pinned readback area
     unsigned long long *d_queue = nullptr;   // work queue of k_hash_chunks
+    uint32_t *d_hhist = nullptr;             // k_hash_* length buckets
+    uint32_t *d_order = nullptr; uint64_t order_cap = 0;   // length-sorted chunk order
     uint64_t *h_flag = nullptr;          // mapped pinned word: a streaming call overflowed
     uint64_t *d_flag = nullptr;          // its device alias
 
@@ -548,6 +550,7 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         cudaMalloc(&ctx->d_carry[0], 4096) != cudaSuccess ||
         cudaMalloc(&ctx->d_carry[1], 4096) != cudaSuccess ||
         cudaMalloc(&ctx->d_queue, 64) != cudaSuccess ||
+        cudaMalloc(&ctx->d_hhist, HB * sizeof(uint32_t)) != cudaSuccess ||
         cudaHostAlloc(&ctx->h_pinned, 64, cudaHostAllocDefault) != cudaSuccess ||
         cudaHostAlloc(&ctx->h_flag, 64, cudaHostAllocMapped) != cudaSuccess ||
         cudaHostGetDevicePointer((void **)&ctx->d_flag, ctx->h_flag, 0) != cudaSuccess) {
@@ -593,7 +596,7 @@ void shred_destroy(shred_ctx *ctx) {
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
     cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_counts); cudaFree(ctx->d_local); cudaFree(ctx->d_groups);
     cudaFree(ctx->d_scratch); cudaFree(ctx->d_cand); cudaFree(ctx->d_sb); cudaFree(ctx->d_aux);
-    cudaFree(ctx->d_carry[0]); cudaFree(ctx->d_carry[1]); cudaFree(ctx->d_queue);
+    cudaFree(ctx->d_carry[0]); cudaFree(ctx->d_carry[1]); cudaFree(ctx->d_queue); cudaFree(ctx->d_hhist); cudaFree(ctx->d_order);
     if (ctx->h_pinned) cudaFreeHost(ctx->h_pinned);
     if (ctx->h_flag) cudaFreeHost(ctx->h_flag);
     cudaGetLastError();
@@ -810,10 +813,19 @@ int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const u
     if (!len || !max_chunks) return SHRED_OK;
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
-    k_write_u64<<<1, 1, 0, st>>>((uint64_t *)ctx->d_queue, 0);
-    LAUNCHED("k_write_u64");
+    int rc = grow(ctx, ctx->d_order, ctx->order_cap, max_chunks, "hash order");
+    if (rc) return rc;
+    if (max_chunks > 0xFFFFFFFFull) return fail(ctx, SHRED_EINVAL, "max_chunks must be < 2^32");
+    CK(cudaMemsetAsync(ctx->d_hhist, 0, HB * sizeof(uint32_t), st), "hash hist reset");
+    const unsigned gs = (unsigned)(ctx->sm_count * 8);
+    k_hash_hist<<<gs, 256, 0, st>>>(d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist);
+    LAUNCHED("k_hash_hist");
+    k_hash_scan<<<1, HB, 0, st>>>(ctx->d_hhist, ctx->d_queue);
+    LAUNCHED("k_hash_scan");
+    k_hash_scatter<<<gs, 256, 0, st>>>(d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist, ctx->d_order);
+    LAUNCHED("k_hash_scatter");
     k_hash_chunks<<<ctx->sm_count * 4, 256, 0, st>>>(d_in, len, d_cuts, d_ncuts, max_chunks, d_digests,
-                                                      ctx->d_queue);
+                                                      ctx->d_order, ctx->d_queue);
     LAUNCHED("k_hash_chunks");
     return SHRED_OK;
 }
