@@ -301,6 +301,17 @@ def main():
                 "share_of_step": round(k_ms / ms, 4) if ms else None, "peak_source": hbm_src,
                 "note": "algorithmic bytes = 1 B read per input byte (+8 B per candidate, ~0.001 B/B); "
                         "the kernel is bound by the shared-memory lookup datapath below HBM (DESIGN.md)"}
+    # the unit that actually binds: 128 B/clk/SM of shared-memory datapath; per input byte the K63
+    # loop moves 16 B of table lookups + 1 B TMA write + 1 B LDS read (K32: 8 + 1 + 1)
+    smem_bpb = 18.0 if ch.path == "k63" else 10.0
+    clk_mhz = clk.result().get("sm_mhz") or 1965.0
+    nsm = torch.cuda.get_device_properties(dev).multi_processor_count
+    smem_ceiling = nsm * clk_mhz * 1e6 * 128.0 / smem_bpb / 1e9
+    if achieved:
+        roofline["smem_datapath"] = {"ceiling_gbs": round(smem_ceiling, 1), "frac": round(achieved / smem_ceiling, 4),
+                                     "bytes_per_input_byte": smem_bpb, "sms": nsm, "sm_mhz": clk_mhz,
+                                     "source": "128 B/clk/SM SMEM/L1 data path (B300_MICROARCH.md); ncu "
+                                               "l1tex__data_pipe_lsu_wavefronts in profiles/r01_k1_bulk_ncu_full.txt"}
 
     line = {"metric": METRIC, "value": round(value, 2), "unit": "GB/s", "n_gpus": world, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": round(ms_max / args.steps, 4), "higher_is_better": True,
