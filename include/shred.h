@@ -157,6 +157,20 @@ int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const u
                       const uint64_t *d_ncuts, uint8_t *d_digests, uint64_t max_chunks,
                       shred_stream_t stream);
 
+/* Matching (dedup step 3): a device index (hash set) of
+   chunk digests owned by the ctx.  shred_index_reset allocates/clears it for `capacity` distinct
+   digests (rounded up to a power of two, >= 2x).  shred_index_insert looks up every chunk digest
+   produced by shred_hash_chunks (same d_cuts / d_ncuts / len): a chunk is "new" if its digest
+   was not in the index (it is then added).  new_flags (optional, device, 1 byte per chunk) gets
+   1 for new chunks; the running totals {chunks inserted, new chunks, new bytes, inserts that
+   found the index full} are read with shred_index_stats (synchronises).  Of two identical chunks
+   inserted by one call exactly one is new. */
+int shred_index_reset(shred_ctx *ctx, uint64_t capacity);
+int shred_index_insert(shred_ctx *ctx, const uint8_t *d_digests, const uint64_t *d_cuts,
+                       const uint64_t *d_ncuts, uint64_t len, uint64_t max_chunks,
+                       uint8_t *d_new_flags, shred_stream_t stream);
+int shred_index_stats(shred_ctx *ctx, uint64_t stats[4]);
+
 /* Bench/test helper (not the method): writes bytes [offset, offset+len) of the counter-mode
    SplitMix64 stream `seed` into d_buf on `stream`. */
 int shred_synth_fill(uint8_t *d_buf, uint64_t len, uint64_t seed, uint64_t offset,

@@ -199,6 +199,27 @@ def chunk_digests(data, cuts) -> np.ndarray:
     return out
 
 
+class Index:
+    """Matching (dedup step 3, L235-L238): a set of digests; a chunk is new iff its digest was
+    not seen before (plain Python set; test infrastructure)."""
+
+    def __init__(self):
+        self.seen = set()
+        self.chunks = self.new_chunks = self.new_bytes = 0
+
+    def insert(self, digests: np.ndarray, lengths) -> np.ndarray:
+        flags = np.zeros(len(lengths), dtype=np.uint8)
+        for k, (d, ln) in enumerate(zip(digests, lengths)):
+            key = bytes(d)
+            self.chunks += 1
+            if key not in self.seen:
+                self.seen.add(key)
+                flags[k] = 1
+                self.new_chunks += 1
+                self.new_bytes += int(ln)
+        return flags
+
+
 def is_irreducible(poly: int) -> bool:
     """Rabin's irreducibility test for div(x) (L255-L256), degree 1..63."""
     return bool(_L().orc_is_irreducible(poly))

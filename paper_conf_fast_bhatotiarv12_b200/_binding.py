@@ -79,6 +79,9 @@ def lib() -> ctypes.CDLL:
             "shred_synth_fill": (cint, [vp, u64, u64, u64, vp]),
             "shred_launch_count": (u64, [vp]),
             "shred_hash_chunks": (cint, [vp, vp, u64, vp, vp, vp, u64, vp]),
+            "shred_index_reset": (cint, [vp, u64]),
+            "shred_index_insert": (cint, [vp, vp, vp, vp, u64, u64, vp, vp]),
+            "shred_index_stats": (cint, [vp, ctypes.POINTER(u64)]),
             "shred_profile": (cint, [vp, cint]),
             "shred_profile_read": (cint, [vp, ctypes.POINTER(ctypes.c_double), ctypes.POINTER(u64),
                                           ctypes.POINTER(u64)]),
@@ -238,6 +241,23 @@ class Chunker:
         self.hash_chunks_async(x, c, n, out)
         torch.cuda.current_stream().synchronize()
         return out.view(-1, 32)[: (cuts.numel() + 1) if x.numel() else 0]
+
+    # ---------------------------------------------------------------- dedup index (f3)
+    def index_reset(self, capacity: int) -> None:
+        self._check(lib().shred_index_reset(self._ctx, capacity), "shred_index_reset")
+
+    def index_insert_async(self, digests: torch.Tensor, cuts: torch.Tensor, n_cuts: torch.Tensor, length: int,
+                           new_flags: torch.Tensor | None = None, stream=None) -> None:
+        assert digests.dtype == torch.uint8 and digests.is_contiguous()
+        rc = lib().shred_index_insert(self._ctx, digests.data_ptr(), cuts.data_ptr(), n_cuts.data_ptr(), length,
+                                      digests.numel() // 32,
+                                      new_flags.data_ptr() if new_flags is not None else None, _stream(stream))
+        self._check(rc, "shred_index_insert")
+
+    def index_stats(self) -> dict:
+        arr = (ctypes.c_uint64 * 4)()
+        self._check(lib().shred_index_stats(self._ctx, arr), "shred_index_stats")
+        return {"chunks": arr[0], "new_chunks": arr[1], "new_bytes": arr[2], "full": arr[3]}
 
     # ---------------------------------------------------------------- streaming
     def feed_async(self, x: torch.Tensor, out: torch.Tensor, n_out: torch.Tensor, stream=None) -> None:

@@ -9,6 +9,7 @@
 #include "kernels.cuh"
 #include "size_bound.cuh"
 #include "sha256.cuh"
+#include "dedup.cuh"
 #include "../../include/shred.h"
 
 #include <cstdarg>
@@ -131,6 +132,7 @@ struct shred_ctx {
     unsigned long long *d_queue = nullptr;   // work queue of k_hash_chunks
     uint32_t *d_hhist = nullptr;             // k_hash_* length buckets
     uint32_t *d_order = nullptr; uint64_t order_cap = 0;   // length-sorted chunk order
+    DedupTable index{};                  // f3: device hash set of digests (shred_index_*)
     uint64_t *h_flag = nullptr;          // mapped pinned word: a streaming call overflowed
     uint64_t *d_flag = nullptr;          // its device alias
 
@@ -597,6 +599,7 @@ void shred_destroy(shred_ctx *ctx) {
     cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_counts); cudaFree(ctx->d_local); cudaFree(ctx->d_groups);
     cudaFree(ctx->d_scratch); cudaFree(ctx->d_cand); cudaFree(ctx->d_sb); cudaFree(ctx->d_aux);
     cudaFree(ctx->d_carry[0]); cudaFree(ctx->d_carry[1]); cudaFree(ctx->d_queue); cudaFree(ctx->d_hhist); cudaFree(ctx->d_order);
+    cudaFree(ctx->index.tag); cudaFree(ctx->index.key); cudaFree(ctx->index.ready); cudaFree(ctx->index.stats);
     if (ctx->h_pinned) cudaFreeHost(ctx->h_pinned);
     if (ctx->h_flag) cudaFreeHost(ctx->h_flag);
     cudaGetLastError();
@@ -827,6 +830,55 @@ int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const u
     k_hash_chunks<<<ctx->sm_count * 4, 256, 0, st>>>(d_in, len, d_cuts, d_ncuts, max_chunks, d_digests,
                                                       ctx->d_order, ctx->d_queue);
     LAUNCHED("k_hash_chunks");
+    return SHRED_OK;
+}
+
+int shred_index_reset(shred_ctx *ctx, uint64_t capacity) {
+    if (!ctx || capacity == 0 || capacity > (1ull << 36)) return SHRED_EINVAL;
+    DevGuard g(ctx->device);
+    uint64_t cap = 1024;
+    while (cap < 2 * capacity) cap <<= 1;
+    cudaDeviceSynchronize();
+    DedupTable &T = ctx->index;
+    if (T.cap != cap) {
+        cudaFree(T.tag); cudaFree(T.key); cudaFree(T.ready);
+        T.tag = nullptr; T.key = nullptr; T.ready = nullptr; T.cap = 0;
+        if (cudaMalloc(&T.tag, cap * 8) != cudaSuccess || cudaMalloc(&T.key, cap * 32) != cudaSuccess ||
+            cudaMalloc(&T.ready, cap * 4) != cudaSuccess) {
+            cudaGetLastError();
+            return fail(ctx, SHRED_ENOMEM, "index: cudaMalloc failed for %llu slots", (unsigned long long)cap);
+        }
+        T.cap = cap;
+    }
+    if (!T.stats && cudaMalloc(&T.stats, 64) != cudaSuccess) { cudaGetLastError(); return SHRED_ENOMEM; }
+    if (cudaMemset(T.tag, 0, cap * 8) != cudaSuccess || cudaMemset(T.ready, 0, cap * 4) != cudaSuccess ||
+        cudaMemset(T.stats, 0, 64) != cudaSuccess)
+        return fail(ctx, SHRED_ECUDA, "index reset");
+    return SHRED_OK;
+}
+
+int shred_index_insert(shred_ctx *ctx, const uint8_t *d_digests, const uint64_t *d_cuts,
+                       const uint64_t *d_ncuts, uint64_t len, uint64_t max_chunks,
+                       uint8_t *d_new_flags, shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    if (!ctx->index.cap) return fail(ctx, SHRED_ESTATE, "shred_index_reset first");
+    if (!d_ncuts || (max_chunks && !d_digests)) return fail(ctx, SHRED_EINVAL, "null pointer");
+    if (((uintptr_t)d_digests & 15u) != 0) return fail(ctx, SHRED_EINVAL, "d_digests must be 16-byte aligned");
+    if (!len || !max_chunks) return SHRED_OK;
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    k_dedup_insert<<<ctx->sm_count * 8, 256, 0, st>>>(ctx->index, d_digests, d_cuts, d_ncuts, len, max_chunks,
+                                                      d_new_flags);
+    LAUNCHED("k_dedup_insert");
+    return SHRED_OK;
+}
+
+int shred_index_stats(shred_ctx *ctx, uint64_t stats[4]) {
+    if (!ctx || !stats) return SHRED_EINVAL;
+    if (!ctx->index.stats) { for (int i = 0; i < 4; ++i) stats[i] = 0; return SHRED_OK; }
+    DevGuard g(ctx->device);
+    CK(cudaDeviceSynchronize(), "index stats sync");
+    CK(cudaMemcpy(stats, ctx->index.stats, 32, cudaMemcpyDeviceToHost), "index stats");
     return SHRED_OK;
 }
 

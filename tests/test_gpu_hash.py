@@ -57,3 +57,38 @@ def test_chunk_then_hash_on_device(pkg, bounded):
     assert np.array_equal(c.astype(np.uint64), oracle.chunk(data, oracle.Params(divisor=2048, min_size=p.min_size,
                                                                                  max_size=p.max_size)))
     assert np.array_equal(dig[:(k + 1) * 32].view(-1, 32).cpu().numpy(), oracle.chunk_digests(data, c))
+
+
+# ------------------------------------------------------------------ f3: dedup across snapshots
+def test_index_dedup_across_snapshots_vs_oracle(pkg):
+    """chunk -> hash -> index over backup snapshots (configs[4] recipe, 12 MiB master): new-chunk
+    and new-byte counts equal the oracle's set semantics; per-chunk flags agree except among
+    identical digests inserted by the same call (then exactly one is new)."""
+    import tools.snapshots as S
+    n = 12 << 20
+    ch = pkg.Chunker(pkg.Params(divisor=4096))
+    ch.index_reset(1 << 20)
+    oi = oracle.Index()
+    buf = torch.empty(n, dtype=torch.uint8, device="cuda")
+    cuts = torch.empty(n // 512, dtype=torch.int64, device="cuda")
+    ncut = torch.zeros(1, dtype=torch.int64, device="cuda")
+    dig = torch.empty(n // 512 * 32, dtype=torch.uint8, device="cuda")
+    flags = torch.empty(n // 512, dtype=torch.uint8, device="cuda")
+    for s in (0, 1, 3, 5, 0, 9):                                  # snapshot 0 twice: all duplicates
+        S.build_snapshot(buf, 6, s)
+        ch.chunk_async(buf, cuts, ncut)
+        ch.hash_chunks_async(buf, cuts, ncut, dig)
+        ch.index_insert_async(dig, cuts, ncut, n, flags)
+        torch.cuda.synchronize()
+        k = int(ncut.item())
+        c = cuts[:k].cpu().numpy()
+        d = dig[:(k + 1) * 32].view(-1, 32).cpu().numpy()
+        lens = np.diff(np.concatenate([[0], c, [n]]))
+        exp_flags = oi.insert(d, lens)
+        got_flags = flags[:k + 1].cpu().numpy()
+        st = ch.index_stats()
+        assert (st["chunks"], st["new_chunks"], st["new_bytes"], st["full"]) == \
+               (oi.chunks, oi.new_chunks, oi.new_bytes, 0)
+        uniq_batch = {bytes(x) for x in d}
+        if len(uniq_batch) == len(d):                             # no duplicates inside the batch
+            assert np.array_equal(got_flags, exp_flags)
