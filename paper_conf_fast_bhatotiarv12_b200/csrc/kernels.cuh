@@ -9,12 +9,13 @@
 // realised with two 256-entry tables: T (reduces the byte shifted out of the top of the
 // state) and U (removes the byte leaving the window).  See DESIGN.md "Kernels".
 //
-//   k1_bulk<MODE>   TMA-staged hot loop.  One thread = one row of S bytes of the input viewed
-//                   as a 2-D [rows][S] tensor; rounds of 64 B per row arrive in a 4-stage
-//                   shared-memory ring (SWIZZLE_64B, conflict-free LDS.128).  T/U live in
+//   k1_bulk<MODE,C,WCH,LE>  TMA-staged hot loop.  The input is viewed as a 2-D [rows][S]
+//                   tensor; each consumer thread rolls CH = 2 rows (independent chains) in one
+//                   basic block; rounds of 32 B per row arrive in a 4-stage shared-memory ring
+//                   (SWIZZLE_32B, conflict-free LDS.128) fed by a producer warp.  T/U live in
 //                   shared memory, replicated per lane so the data-dependent lookups never
-//                   bank-conflict.  A per-16-byte predicate detects the rare marker hit;
-//                   hits replay that chunk exactly and append c to the thread's slot list.
+//                   bank-conflict.  The marker test sets bits of a per-16-byte hit mask
+//                   (ISETP + predicated OR); rare hits are appended to the row's slot list.
 //                   The last CTA of the launch is the "edge" CTA: it rolls the unaligned head
 //                   and the ragged tail of the range with the generic byte loop.  Every CTA
 //                   ends with a block scan of its slots' counts (local offsets + group sum).
@@ -28,15 +29,12 @@
 #include <cuda.h>
 #include <cuda_runtime.h>
 
-#ifndef SHRED_PUSHHI_FMA
-#define SHRED_PUSHHI_FMA 0      // 1: f_hi shift-in as IMAD.HI + IMAD (FMA pipe) instead of PRMT
-#endif
 #ifndef SHRED_PRODUCER_SLEEP_NS
 #define SHRED_PRODUCER_SLEEP_NS 512
 #endif
 #ifndef SHRED_HITMODE
-#define SHRED_HITMODE 3         // 3: ISETP + predicated OR per byte (default); 0: ISETP+SEL bitmask;
-                                // 1: chunk predicate + exact replay on hit; 2: FMA-pipe test
+#define SHRED_HITMODE 3         // 3: ISETP + predicated OR per byte (default); 0: ISETP + SEL bitmask
+                                // (A/B of these and of removed variants: profiles/r01_ab_variants.txt)
 #endif
 
 namespace shred {
@@ -342,8 +340,6 @@ struct BulkCtx {
     uint32_t m256;      // 256 (row stride of the table image)
     uint32_t tmul;      // 2^(32-m): (f_lo * tmul) keeps the low m bits at the top
     uint32_t rsh;       // r << (32-m)
-    uint32_t one;       // 1 (runtime, keeps IMAD.WIDE on the FMA pipe in SHRED_HITMODE 2)
-    uint32_t two;       // 2 (runtime, shift-accumulate of the hit bits by IMAD)
 };
 
 // One byte step, K63 (deg P = 63, fully reduced u64 state f = fh:fl, f < 2^63):
@@ -358,11 +354,7 @@ __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, 
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
     const uint2 T = lds64(ti);
     const uint2 U = lds64(c.tab + oi);
-#if SHRED_PUSHHI_FMA
-    const uint32_t nh = fh * c.m256 + __umulhi(fl, c.m256);       // (fh << 8) | (fl >> 24)
-#else
     const uint32_t nh = __byte_perm(fh, fl, 0x2107u);
-#endif
     const uint32_t nl = __byte_perm(fl, in, 0x2104u + K);
     fl = nl ^ T.x ^ U.x;
     fh = nh ^ T.y ^ U.y;
@@ -410,13 +402,6 @@ __device__ __forceinline__ uint32_t or_if_marker(uint32_t m, uint32_t lo, const 
             : "+r"(m) : "r"(x), "r"(c.rsh), "n"(BIT));
     return m;
 }
-// FMA-pipe form: 1 if NOT a marker.  y = (f_lo << (32-m)) - (r << (32-m)) is 0 iff marker;
-// hi32(y * 1 + 0xFFFFFFFF) = (y != 0).
-__device__ __forceinline__ uint32_t not_marker(uint32_t lo, const BulkCtx &c) {
-    const uint32_t y = lo * c.tmul - c.rsh;
-    const uint64_t w = (uint64_t)y * (uint64_t)c.one + 0xFFFFFFFFull;
-    return (uint32_t)(w >> 32);
-}
 
 struct SlotOut {
     uint64_t *lst; uint32_t cnt; uint32_t cap;
@@ -439,12 +424,8 @@ __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t min_i,
 // One word (4 bytes) of CH interleaved chains; hit bits accumulate into m[ch] (bit 4J+q).
 #if SHRED_HITMODE == 0
 #define SHRED_MARK(ch, q) m[ch] |= is_marker(st[ch].low(), c) ? (1u << (4 * J + q)) : 0u;
-#elif SHRED_HITMODE == 2
-#define SHRED_MARK(ch, q) m[ch] = m[ch] * c.two + not_marker(st[ch].low(), c);
-#elif SHRED_HITMODE == 3
-#define SHRED_MARK(ch, q) m[ch] = or_if_marker<(1u << (4 * J + q)), LE>(m[ch], st[ch].low(), c);
 #else
-#define SHRED_MARK(ch, q) m[ch] |= (uint32_t)is_marker(st[ch].low(), c);
+#define SHRED_MARK(ch, q) m[ch] = or_if_marker<(1u << (4 * J + q)), LE>(m[ch], st[ch].low(), c);
 #endif
 template <int MODE, int CH, bool TEST, int J, bool LE>
 __device__ __forceinline__ void word4xN(State<MODE> (&st)[CH], const uint32_t (&in)[CH],
@@ -496,33 +477,9 @@ __device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d
 #pragma unroll
     for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].w; po[ch] = p[ch].w; }
     word4xN<MODE, CH, TEST, 3, LE>(st, in, po, m, c);
-#if SHRED_HITMODE == 2
-    // bit 15-j = "position j is not a marker" -> bit j = "position j is a marker"
-    if (TEST) {
-#pragma unroll
-        for (int ch = 0; ch < CH; ++ch) m[ch] = __brev(~m[ch]) >> 16;
-    }
-#endif
 }
 
-// Exact hit mask of one 16-byte chunk of one chain, recomputed from its entry state (the rare
-// path of SHRED_HITMODE 1).
-template <int MODE>
-__device__ __noinline__ uint32_t replay_mask(State<MODE> s, uint4 d, uint4 p, const BulkCtx &c) {
-    const uint32_t dw[4] = {d.x, d.y, d.z, d.w};
-    const uint32_t pw[4] = {p.x, p.y, p.z, p.w};
-    uint32_t m = 0;
-#pragma unroll
-    for (int j = 0; j < 4; ++j) {
-        s.template step<0>(dw[j], pw[j], c); m |= is_marker(s.low(), c) ? (1u << (4 * j + 0)) : 0u;
-        s.template step<1>(dw[j], pw[j], c); m |= is_marker(s.low(), c) ? (1u << (4 * j + 1)) : 0u;
-        s.template step<2>(dw[j], pw[j], c); m |= is_marker(s.low(), c) ? (1u << (4 * j + 2)) : 0u;
-        s.template step<3>(dw[j], pw[j], c); m |= is_marker(s.low(), c) ? (1u << (4 * j + 3)) : 0u;
-    }
-    return m;
-}
-
-struct BulkConst { uint32_t mhi, m256, tmul, rsh, one; };
+struct BulkConst { uint32_t mhi, m256, tmul, rsh; };
 
 // The hot kernel.  blockDim = NTC consumers + 1 producer warp; one CTA per SM.
 // blockIdx < nc: bulk CTA, rows blockIdx*ROWS + tid + ch*NTC (ch < CH); blockIdx == nc: the
@@ -607,7 +564,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         c.laneT = sbase + (uint32_t)lane * 4u;
         c.laneU = 128u + (uint32_t)lane * 4u;
     }
-    c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh; c.one = K.one; c.two = 2u * K.one;
+    c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh;
 
     bool act[CH];
     uint64_t pos0[CH];
@@ -670,18 +627,10 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                 uint32_t m[CH];
 #pragma unroll
                 for (int ch = 0; ch < CH; ++ch) { d[ch] = D[ch][u]; p[ch] = R[ch][(cq + 4 - WCH) & 3]; }
-#if SHRED_HITMODE == 1
-                State<MODE> s0[CH];
-#pragma unroll
-                for (int ch = 0; ch < CH; ++ch) s0[ch] = st[ch];
-#endif
                 chunk16xN<MODE, CH, true, LE>(st, d, p, c, m);
 #pragma unroll
                 for (int ch = 0; ch < CH; ++ch) {
                     R[ch][cq] = D[ch][u];
-#if SHRED_HITMODE == 1
-                    if (m[ch] && act[ch]) m[ch] = replay_mask<MODE>(s0[ch], d[ch], p[ch], c);
-#endif
                     if (m[ch] && act[ch])
                         emit_mask(m[ch], pos0[ch] + (uint64_t)(r + qr) * ROUND + 16u * u, J.min_i, J.c_limit, o[ch]);
                 }

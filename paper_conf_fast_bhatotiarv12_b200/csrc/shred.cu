@@ -329,7 +329,6 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         K.m256 = 256u;
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
-        K.one = 1u;
         const int smem = ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM;
         const int threads = (ctx->path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC) + 32;
         ctx->k1_fn<<<pl.bulk_ctas, threads, smem, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
