@@ -385,7 +385,19 @@ def main():
             torch.cuda.synchronize()
             best = min(best, q0.elapsed_time(q1))
         h2d_peak = (256 << 20) / (best * 1e-3) / 1e9
+        # ring depth 3 (the paper's Fig. 9 pipeline-depth analogue), same step
+        che.set_ring(3, 256 << 20)
+        e2e_step()
+        torch.cuda.synchronize()
+        r0, r1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        r0.record(stream)
+        for _ in range(max(2, args.steps // 2)):
+            e2e_step()
+        r1.record(stream)
+        torch.cuda.synchronize()
+        ev3 = world * per_rank_bytes * max(2, args.steps // 2) / (r0.elapsed_time(r1) * 1e-3) / 1e9
         line["e2e"] = {"value": round(ev, 3), "unit": "GB/s", "h2d_bytes_per_step": per_rank_bytes,
+                       "ring3_value": round(ev3, 3),
                        "d2h_bytes_per_step": d2h[0], "ms_per_step": round(ems / args.steps, 3),
                        "api": "shred_feed(pinned host, 2 x 256 MiB device slots) + shred_flush + D2H of cuts",
                        "h2d_peak_gbs": round(h2d_peak, 2), "frac_of_h2d_peak": round(ev / world / h2d_peak, 4),
@@ -409,7 +421,7 @@ def main():
         try:
             chb = pkg.Chunker(pkg.Params(min_size=2048, max_size=65536), device=local)
             line["bounded_2048_65536"] = {"value": round(timed(chb, base), 2), "unit": "GB/s",
-                                          "note": "size rule on: one host sync (count) + parallel speculative size-rule kernels"}
+                                          "note": "size rule on: parallel speculative size-rule kernels (sb_*), no host sync"}
             c32 = pkg.Chunker(pkg.Params(poly=0x104C11DB7), device=local)
             v32 = timed(c32, base)
             line["k32_variant"] = {"value": round(v32, 2), "unit": "GB/s", "hbm_frac": round(v32 / hbm, 4),
