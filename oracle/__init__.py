@@ -76,6 +76,8 @@ def _L():
         lib.orc_candidates.argtypes = [P, u64, u32, u64, u64, u64, cint, cint, cint, P, u64]
         lib.orc_size_bound.restype = i64
         lib.orc_size_bound.argtypes = [P, u64, u64, u64, u64, P, u64]
+        lib.orc_size_bound_from.restype = i64
+        lib.orc_size_bound_from.argtypes = [P, u64, u64, cint, u64, cint, u64, u64, P, u64, P]
         _lib = lib
     return _lib
 
@@ -172,6 +174,21 @@ def size_bound(cands: np.ndarray, n: int, min_size: int, max_size: int) -> np.nd
     k = _L().orc_size_bound(c.ctypes.data, c.size, n, min_size, max_size, out.ctypes.data, cap)
     assert 0 <= k <= cap
     return out[:k].copy()
+
+
+def size_bound_from(cands: np.ndarray, end: int, fin: bool, s0: int, held0: bool, min_size: int,
+                    max_size: int) -> tuple[np.ndarray, int, bool]:
+    """The size rule from an entry state over one stream range ending at `end` (a fed piece or
+    a byte-range shard): returns (cuts, exit s, exit held).  size_bound(c, N, ..) ==
+    size_bound_from(c, N, True, 0, False, ..)[0]."""
+    c = np.ascontiguousarray(cands, dtype=np.uint64)
+    cap = c.size + (end // max_size + 2 if max_size else 0) + 2
+    out = np.zeros(cap, dtype=np.uint64)
+    st = np.zeros(2, dtype=np.uint64)
+    k = _L().orc_size_bound_from(c.ctypes.data, c.size, end, int(fin), s0, int(held0), min_size, max_size,
+                                 out.ctypes.data, cap, st.ctypes.data)
+    assert 0 <= k <= cap
+    return out[:k].copy(), int(st[0]), bool(st[1])
 
 
 def chunk(data, p: Params = Params(), method: int = 2, threads: int | None = None) -> np.ndarray:

@@ -356,3 +356,24 @@ def test_chunk_digests_boundaries():
     import hashlib
     assert d[1].tobytes() == hashlib.sha256(data[10:500].tobytes()).digest()
     assert d[3].tobytes() == hashlib.sha256(data[999:].tobytes()).digest()
+
+
+
+def test_size_bound_from_composes_over_pieces():
+    """Running the rule piece by piece, each from the previous exit state, equals one run over the
+    whole list (the streaming/sharded reading); the whole-stream case equals orc_size_bound."""
+    rng = np.random.default_rng(8)
+    for trial in range(200):
+        n = int(rng.integers(2, 3000))
+        cands = np.unique(rng.integers(1, n, int(rng.integers(0, 200)))).astype(np.uint64)
+        mn = int(rng.integers(0, 60)); mx = int(rng.choice([0, max(1, mn) + int(rng.integers(0, 120))]))
+        whole = oracle.size_bound(cands, n, mn, mx)
+        w2, _, _ = oracle.size_bound_from(cands, n, True, 0, False, mn, mx)
+        assert np.array_equal(whole, w2)
+        bounds = sorted(set([0, n] + [int(x) for x in rng.integers(1, n, int(rng.integers(1, 5)))]))
+        s, held, got = 0, False, []
+        for a, b in zip(bounds[:-1], bounds[1:]):
+            part = cands[(cands > a) & (cands <= b)]
+            cuts, s, held = oracle.size_bound_from(part, b, b == n, s, held, mn, mx)
+            got += cuts.tolist()
+        assert got == whole.tolist(), (trial, mn, mx, bounds)
