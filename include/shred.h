@@ -128,6 +128,16 @@ int shred_candidates_range(shred_ctx *ctx, const uint8_t *d_in, uint64_t halo, u
 int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, uint64_t total_len,
                      uint64_t *d_out, uint64_t cap, uint64_t *n_out, shred_stream_t stream);
 
+/* The size rule from an explicit entry state over one range of the stream ending at `end`
+   (the per-shard step of the distributed size rule): state_in = {s, held}
+   (s = last cut; held = 1 if a cut at s is not yet emitted; {0, 0} at the stream start).
+   fin = 1 if `end` is the stream end, else a candidate accepted exactly at `end` is held.
+   Cuts go to d_out (cap, n_out as usual); d_state_out (device, 2 x u64) gets the exit
+   {s, held}.  Chaining ranges through their states equals one run over the whole list. */
+int shred_size_bound_state(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, uint64_t end,
+                           int fin, const uint64_t state_in[2], uint64_t *d_out, uint64_t cap,
+                           uint64_t *n_out, uint64_t *d_state_out, shred_stream_t stream);
+
 /* Streaming with carried window and size-rule state (§4.1-§4.2: pinned
    buffers, async transfers, multi-buffering).  `in` is device memory or page-locked host
    memory (pageable host memory -> SHRED_EINVAL).  Host input is copied by the ctx's own copy

@@ -80,6 +80,7 @@ def lib() -> ctypes.CDLL:
             "shred_launch_count": (u64, [vp]),
             "shred_hash_chunks": (cint, [vp, vp, u64, vp, vp, vp, u64, vp]),
             "shred_index_reset": (cint, [vp, u64]),
+            "shred_size_bound_state": (cint, [vp, vp, u64, u64, cint, ctypes.POINTER(u64), vp, u64, vp, vp, vp]),
             "shred_index_insert": (cint, [vp, vp, vp, vp, u64, u64, vp, vp]),
             "shred_index_stats": (cint, [vp, ctypes.POINTER(u64)]),
             "shred_profile": (cint, [vp, cint]),
@@ -222,6 +223,26 @@ class Chunker:
         if n > cap:
             raise ShredError(f"capacity {cap} < {n} cuts")
         return out[:n]
+
+    def size_bound_state(self, cands: torch.Tensor, end: int, fin: bool, s: int, held: bool,
+                         cap: int | None = None) -> tuple[torch.Tensor, int, bool]:
+        """The size rule over one stream range from entry state (s, held): (cuts, exit s, exit held)."""
+        assert cands.dtype == torch.int64 and cands.is_contiguous()
+        dev = torch.device("cuda", self.device)
+        c = cands if cands.is_cuda else cands.to(dev)
+        cap = self.max_cuts(end + 2) + 2 if cap is None else cap
+        out = self._out(cap)
+        st = torch.zeros(2, dtype=torch.int64, device=dev)
+        sin = (ctypes.c_uint64 * 2)(s, int(held))
+        rc = lib().shred_size_bound_state(self._ctx, c.data_ptr() if c.numel() else None, c.numel(), end, int(fin),
+                                          sin, out.data_ptr(), out.numel(), self._n.data_ptr(), st.data_ptr(),
+                                          _stream(None))
+        self._check(rc, "shred_size_bound_state")
+        n = int(self._n.item())
+        if n > cap:
+            raise ShredError(f"capacity {cap} < {n} cuts")
+        sv = st.cpu().tolist()
+        return out[:n], int(sv[0]), bool(sv[1])
 
     # ---------------------------------------------------------------- hashing (f2)
     def hash_chunks_async(self, x: torch.Tensor, cuts: torch.Tensor, n_cuts: torch.Tensor,

@@ -767,6 +767,16 @@ __global__ void k_stream_reset(Aux *aux) {
 
 __global__ void k_write_u64(uint64_t *p, uint64_t v) { *p = v; }
 
+// Entry / exit of shred_size_bound_state.
+__global__ void k_state_in(Aux *aux, uint64_t s, uint64_t held) {
+    aux->total = 0; aux->last_cand = 0; aux->out_pos = 0; aux->dense = 0;
+    aux->s = s; aux->held = held; aux->held_val = held ? s : 0;
+}
+__global__ void k_state_out(const Aux *aux, uint64_t *state, uint64_t *n_out, uint64_t cap) {
+    state[0] = aux->s; state[1] = aux->held;
+    *n_out = aux->out_pos;
+}
+
 // New carry = the last min(keep, old_len + len) bytes of (old carry || src[0..len)).
 __global__ void k_carry(const uint8_t *old_c, uint32_t old_len, const uint8_t *src, uint64_t len,
                         uint8_t *new_c, uint32_t keep) {

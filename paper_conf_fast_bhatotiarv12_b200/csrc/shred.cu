@@ -665,6 +665,26 @@ int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, ui
     return SHRED_OK;
 }
 
+int shred_size_bound_state(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, uint64_t end,
+                           int fin, const uint64_t state_in[2], uint64_t *d_out, uint64_t cap,
+                           uint64_t *n_out, uint64_t *d_state_out, shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    int rc = check_out(ctx, d_out, cap, n_out);
+    if (rc) return rc;
+    if ((n_cand && !d_cand) || !state_in || !d_state_out) return fail(ctx, SHRED_EINVAL, "null pointer");
+    if (state_in[0] > end) return fail(ctx, SHRED_EINVAL, "entry state beyond the range end");
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    Aux *aux = ctx->d_aux + 0;
+    k_state_in<<<1, 1, 0, st>>>(aux, state_in[0], state_in[1] ? 1ull : 0ull);
+    LAUNCHED("k_state_in");
+    if ((rc = launch_size_bound(ctx, d_cand, nullptr, n_cand, n_cand, end, fin ? 1 : 0, d_out, cap, aux,
+                                nullptr, st))) return rc;
+    k_state_out<<<1, 1, 0, st>>>(aux, d_state_out, n_out, cap);
+    LAUNCHED("k_state_out");
+    return SHRED_OK;
+}
+
 // ---------------------------------------------------------------------------- streaming
 int shred_set_ring(shred_ctx *ctx, int slots, uint64_t slot_bytes) {
     if (!ctx) return SHRED_EINVAL;

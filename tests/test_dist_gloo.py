@@ -35,6 +35,11 @@ class OracleEngine:
         c = c[(c >= start + 1) & (c < total_len)]                 # window ends i >= start
         return torch.from_numpy(c)
 
+    def size_bound_state(self, cands, end, fin, s, held):
+        c, s2, h2 = oracle.size_bound_from(cands.numpy().astype(np.uint64), end, fin, s, held,
+                                           self.params.min_size, self.params.max_size)
+        return torch.from_numpy(c.astype(np.int64)), s2, h2
+
     def size_bound(self, cands, total_len):
         return torch.from_numpy(oracle.size_bound(cands.numpy().astype(np.uint64), total_len,
                                                   self.params.min_size, self.params.max_size).astype(np.int64))
@@ -48,7 +53,7 @@ def _free_port():
     return p
 
 
-def _worker(rank, world, port, n, seed, params, q):
+def _worker(rank, world, port, n, seed, params, q, mode="chain"):
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
     dist.init_process_group("gloo", rank=rank, world_size=world)
@@ -63,19 +68,19 @@ def _worker(rank, world, port, n, seed, params, q):
         x2 = sd.exchange_halo(own, start, params.window)            # C1 over the process group
         assert np.array_equal(x2.numpy(), x.numpy())
         eng = OracleEngine(params, data)
-        res = sd.chunk_sharded(x, halo, start, n, eng)
+        res = sd.chunk_sharded(x, halo, start, n, eng, mode=mode)
         allc = sd.gather_all(res).numpy()
         q.put((rank, res.base, res.total, res.local.numpy().tolist(), allc.tolist(),
-               None if res.cuts is None else res.cuts.numpy().tolist()))
+               None if res.cuts is None else res.cuts.numpy().tolist(), res.cut_base, res.rounds))
     finally:
         dist.destroy_process_group()
 
 
-def _run(world, n, seed, params):
+def _run(world, n, seed, params, mode="chain"):
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    procs = [ctx.Process(target=_worker, args=(r, world, port, n, seed, params, q)) for r in range(world)]
+    procs = [ctx.Process(target=_worker, args=(r, world, port, n, seed, params, q, mode)) for r in range(world)]
     for p in procs:
         p.start()
     out = [q.get(timeout=300) for _ in range(world)]
@@ -92,7 +97,7 @@ def test_sharded_unbounded_matches_whole_stream(world):
     exp = oracle.candidates(synthgen.random_bytes(7, n), params).astype(np.int64).tolist()
     out = _run(world, n, 7, params)
     cat = []
-    for rank, base, total, local, allc, cuts in out:
+    for rank, base, total, local, allc, cuts, cut_base, rounds in out:
         assert base == len(cat)
         assert total == len(exp)
         cat += local
@@ -101,14 +106,63 @@ def test_sharded_unbounded_matches_whole_stream(world):
     assert cat == exp
 
 
-def test_sharded_bounded_global_size_rule():
+@pytest.mark.parametrize("world,mode", [(2, "gather"), (2, "chain"), (3, "chain")])
+def test_sharded_bounded_global_size_rule(world, mode):
     n = (1 << 20) + 999
     params = oracle.Params(divisor=512, min_size=128, max_size=4096)
     data = synthgen.random_bytes(9, n)
     exp = oracle.chunk(data, params).astype(np.int64).tolist()
-    out = _run(2, n, 9, params)
-    for rank, base, total, local, allc, cuts in out:
-        assert cuts == exp
+    out = _run(world, n, 9, params, mode)
+    if mode == "gather":
+        for rank, base, total, local, allc, cuts, cut_base, rounds in out:
+            assert cuts == exp
+    else:
+        cat = []
+        for rank, base, total, local, allc, cuts, cut_base, rounds in out:
+            assert cut_base == len(cat)
+            assert rounds <= world
+            cat += cuts
+        assert cat == exp
+
+
+def test_sharded_chain_adversarial_phase_lock():
+    """Periodic candidates 2 bytes apart with min = 3: entry guesses are out of phase, so the
+    chain needs extra rounds; the result is still exact."""
+    n = 300000
+    params = oracle.Params(divisor=8192, min_size=3, max_size=0)
+    ctx = mp.get_context("spawn")
+    data = synthgen.periodic(b"\x04\xd5", n)
+    exp = oracle.chunk(data, params).astype(np.int64).tolist()
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_worker_periodic, args=(r, 3, port, n, params, q)) for r in range(3)]
+    for p in procs:
+        p.start()
+    out = sorted(q.get(timeout=300) for _ in range(3))
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    cat = []
+    for rank, cuts, cut_base in out:
+        assert cut_base == len(cat)
+        cat += cuts
+    assert cat == exp
+
+
+def _worker_periodic(rank, world, port, n, params, q):
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        from paper_conf_fast_bhatotiarv12_b200 import dist as sd
+        data = synthgen.periodic(b"\x04\xd5", n)
+        start, end = sd.shard_bounds(n, world, rank, align=4096)
+        halo = sd.halo_of(start, params.window)
+        x = torch.from_numpy(data[start - halo:end].copy())
+        res = sd.chunk_sharded(x, halo, start, n, OracleEngine(params, data), mode="chain")
+        q.put((rank, res.cuts.numpy().tolist(), res.cut_base))
+    finally:
+        dist.destroy_process_group()
 
 
 def test_shard_bounds_cover_the_stream():

@@ -139,6 +139,26 @@ def test_virtual_shards_concatenate_to_chunk(pkg, G):
     assert np.array_equal(cuts.astype(np.uint64), oracle.size_bound(exp, n, 256, 8192))
 
 
+def test_size_bound_state_chains_over_virtual_shards(pkg):
+    """shred_size_bound_state: chaining the rule over shard ranges through the exit states equals
+    the whole-stream rule (the per-rank step of the distributed size rule, f1)."""
+    n = (9 << 20) + 321
+    data = synthgen.random_bytes(17, n)
+    p = pkg.Params(divisor=1024, min_size=256, max_size=8192)
+    ch = pkg.Chunker(p)
+    cand = oracle.candidates(data, oracle.Params(divisor=1024)).astype(np.int64)
+    exp = oracle.size_bound(cand.astype(np.uint64), n, 256, 8192)
+    for G in (1, 3, 8):
+        bounds = [n * g // G for g in range(G + 1)]
+        s, held, got = 0, False, []
+        for g in range(G):
+            a, b = bounds[g], bounds[g + 1]
+            part = torch.from_numpy(cand[(cand > a) & (cand <= b)].copy())
+            cuts, s, held = ch.size_bound_state(part, b, b == n, s, held)
+            got.append(cuts.cpu().numpy())
+        assert np.array_equal(np.concatenate(got).astype(np.uint64), exp)
+
+
 # ------------------------------------------------------------------ streaming (config 3 shape)
 def _feed_all(ch, data, sizes, pinned):
     outs = []
