@@ -426,6 +426,23 @@ def main():
             v32 = timed(c32, base)
             line["k32_variant"] = {"value": round(v32, 2), "unit": "GB/s", "hbm_frac": round(v32 / hbm, 4),
                                    "params": "P=0x104C11DB7 (deg 32, irreducible), other params as paper"}
+            # configs[0]: 1 MiB per call, launch-latency bound -> report microseconds per call
+            small = base[: 1 << 20]
+            o_s = torch.empty(4096, dtype=torch.int64, device=dev)
+            n_s = torch.zeros(1, dtype=torch.int64, device=dev)
+            for _ in range(10):
+                ch.chunk_async(small, o_s, n_s)
+            torch.cuda.synchronize()
+            q0, q1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            q0.record(stream)
+            for _ in range(200):
+                ch.chunk_async(small, o_s, n_s)
+            q1.record(stream)
+            torch.cuda.synchronize()
+            us = q0.elapsed_time(q1) * 1e3 / 200
+            line["config1_1mib"] = {"us_per_call": round(us, 2), "gbs": round((1 << 20) / (us * 1e-6) / 1e9, 1),
+                                    "candidates": int(n_s.item()),
+                                    "note": "configs[0] size, device-resident, back-to-back calls on one stream"}
             # f2: SHA-256 of every chunk, alone and chained after chunking (no host round trip)
             dig = torch.empty((cap + 1) * 32, dtype=torch.uint8, device=dev)
             ch.chunk_async(base, out0, n0)

@@ -241,7 +241,7 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
             const uint64_t target = (uint64_t)(ctx->sm_count > 1 ? ctx->sm_count - 1 : 1) * ROWS_CTA;
             S = (blen + target - 1) / target;
             S = (S + 63) / 64 * 64;                // an even number of ROUND-byte rounds
-            if (S < 256) S = 256;
+            if (S < 64) S = 64;                    // small inputs: more rows, latency-bound anyway
             nrows = blen / S;
             if (nrows > 0 && nrows < (1ull << 31) && S < (1ull << 39) && (b0 - t_begin) <= GS * NTC)
                 pl.bulk = true;
