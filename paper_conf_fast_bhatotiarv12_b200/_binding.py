@@ -283,7 +283,7 @@ class Chunker:
     # ---------------------------------------------------------------- streaming
     def feed_async(self, x: torch.Tensor, out: torch.Tensor, n_out: torch.Tensor, stream=None) -> None:
         assert x.dtype == torch.uint8 and x.is_contiguous()
-        assert x.is_cuda or x.is_pinned(), "host input must be pinned"
+        assert x.numel() == 0 or x.is_cuda or x.is_pinned(), "host input must be pinned"
         rc = lib().shred_feed(self._ctx, x.data_ptr(), x.numel(), out.data_ptr(), out.numel(),
                               n_out.data_ptr(), _stream(stream))
         self._check(rc, "shred_feed")

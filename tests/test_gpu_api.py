@@ -119,3 +119,28 @@ def test_profile_hook_counts_hot_launches(pkg):
     ch.profile(False)
     ms, launches, nbytes = ch.profile_read()
     assert launches == 2 and ms > 0 and nbytes == 2 * x.numel()
+
+
+def test_feed_edge_cases_mixed_sources_and_empty(pkg):
+    """Zero-length feeds change nothing; device and pinned-host pieces can be mixed in one stream;
+    an empty shard range yields no candidates."""
+    n = (2 << 20) + 17
+    data = synthgen.random_bytes(25, n)
+    for p in (pkg.Params(divisor=1024), pkg.Params(divisor=1024, min_size=300, max_size=5000)):
+        ch = pkg.Chunker(p)
+        ch.set_ring(2, 1 << 19)
+        outs = []
+        a = 0
+        for k, b in enumerate((0, 1000, 1000, 300000, 1500000, n)):
+            piece = torch.from_numpy(data[a:b].copy())
+            x = piece.cuda() if k % 2 else piece.pin_memory()
+            outs.append(ch.feed(x).cpu().numpy())
+            a = b
+        outs.append(ch.feed(torch.zeros(0, dtype=torch.uint8).cuda()).cpu().numpy())
+        outs.append(ch.flush().cpu().numpy())
+        got = np.concatenate(outs).astype(np.uint64)
+        exp = oracle.chunk(data, oracle.Params(divisor=1024, min_size=p.min_size, max_size=p.max_size))
+        assert np.array_equal(got, exp)
+    ch = pkg.Chunker(pkg.Params())
+    x = torch.from_numpy(data[:47].copy()).cuda()
+    assert ch.candidates_range(x, 47, 47, n).numel() == 0      # halo only, empty range
