@@ -378,10 +378,8 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
     A.dst = dst; A.dst_cap = cap; A.aux = aux;
     const unsigned g = (unsigned)((nb + SB_THREADS - 1) / SB_THREADS);
     if (nb) {
-        sb_spec<<<g, SB_THREADS, 0, st>>>(A);
-        LAUNCHED("sb_spec");
-        sb_check<<<g, SB_THREADS, 0, st>>>(A);
-        LAUNCHED("sb_check");
+        sb_spec_check<<<g, SB_THREADS, 0, st>>>(A);
+        LAUNCHED("sb_spec_check");
     }
     sb_plan<<<1, 1024, 0, st>>>(A);
     LAUNCHED("sb_plan");

@@ -8,11 +8,11 @@
 // It is sequential in s, but the state is a single number and two runs over the same
 // candidates that ever reach the same s stay identical afterwards.  The parallel form
 // (exact for any input):
-//   sb_spec   block b of SB_B candidates runs speculatively from g_b = c[first-1] (i.e. "the
-//             previous candidate was accepted"); block 0 runs from the true initial state.
-//             -> spec exit state, spec count.
-//   sb_check  block b runs from e_b = spec exit of block b-1 in lockstep with its speculation
-//             until the two states coincide (sync) -> count delta; no sync -> not ok.
+//   sb_spec_check  block b of SB_B candidates runs speculatively from g_b = c[first-1] (i.e.
+//             "the previous candidate was accepted"; block 0 from the true initial state)
+//             -> spec exit state, spec count; and, in lockstep, from e_b = the spec exit of
+//             block b-1 (recomputed by the same thread) until the two states coincide (sync)
+//             -> count delta; no sync -> not ok.
 //   sb_plan   one CTA: if every block synced, entries = spec exits and the offsets are a scan
 //             of the counts; otherwise warp 0 walks the blocks in order, re-walking the ones
 //             whose assumed entry does not hold (exact; serial only through those blocks).
@@ -26,7 +26,7 @@
 
 namespace shred {
 
-constexpr int SB_B = 32;            // candidates per block (one thread; prefetched into registers)
+constexpr int SB_B = 16;            // candidates per block (one thread; prefetched into registers)
 constexpr int SB_THREADS = 128;
 
 struct SBArgs {
@@ -70,7 +70,9 @@ __device__ __forceinline__ uint64_t sb_tail_count(uint64_t s, const SBArgs &A) {
     return (A.end - s - 1) / A.maxsz;
 }
 
-__global__ void __launch_bounds__(SB_THREADS) sb_spec(SBArgs A) {
+// sb_spec + sb_check fused: thread b runs the speculation of block b-1 (to get its exit X),
+// then block b from its own guess and, in lockstep, from X until the two states coincide.
+__global__ void __launch_bounds__(SB_THREADS) sb_spec_check(SBArgs A) {
     if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
@@ -78,87 +80,84 @@ __global__ void __launch_bounds__(SB_THREADS) sb_spec(SBArgs A) {
     if (b >= nb) return;
     const uint64_t first = b * SB_B, last = min(n, first + SB_B);
     uint64_t v[SB_B];
+    uint64_t X = 0;
+    int hX = 0;
+    if (b) {                                  // speculation of block b-1 (its guess, or exact for 0)
+        const uint64_t pf = first - SB_B;
+#pragma unroll
+        for (int j = 0; j < SB_B; ++j) v[j] = A.cand[pf + j];
+        X = (b - 1) ? A.cand[pf - 1] : A.aux->s;
+#pragma unroll
+        for (int j = 0; j < SB_B; ++j) sb_step(X, v[j], A, hX, NoEmit{});
+    }
 #pragma unroll
     for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
-    uint64_t s = b ? A.cand[first - 1] : A.aux->s;
-    uint64_t cnt = 0;
-    int held = 0;
-#pragma unroll
-    for (int j = 0; j < SB_B; ++j)
-        if (first + j < last) cnt += sb_step(s, v[j], A, held, NoEmit{});
-    A.spec_exit[b] = s;
-    A.spec_cnt[b] = cnt;
-}
-
-__global__ void __launch_bounds__(SB_THREADS) sb_check(SBArgs A) {
-    if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
-    const uint64_t n = sb_n(A);
-    const uint64_t nb = (n + SB_B - 1) / SB_B;
-    const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
-    if (b >= nb) return;
-    if (b == 0) { A.ok[0] = 1; A.delta[0] = 0; return; }
-    const uint64_t first = b * SB_B, last = min(n, first + SB_B);
-    uint64_t s1 = A.spec_exit[b - 1], s2 = A.cand[first - 1];
-    int64_t c1 = 0, c2 = 0;
-    int h1 = 0, h2 = 0;
-    uint32_t ok = (s1 == s2);
-    uint64_t v[SB_B];
-#pragma unroll
-    for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
+    uint64_t sg = b ? A.cand[first - 1] : A.aux->s;       // this block's guess
+    int hg = 0, ht = 0;
+    uint64_t cg = 0;
+    int64_t ct = 0, cg_sync = 0;
+    bool synced = (b == 0) || (X == sg && hX == 0);
+    uint64_t st = X;
 #pragma unroll
     for (int j = 0; j < SB_B; ++j) {
-        if (first + j < last && !ok) {
-            c1 += (int64_t)sb_step(s1, v[j], A, h1, NoEmit{});
-            c2 += (int64_t)sb_step(s2, v[j], A, h2, NoEmit{});
-            ok = (s1 == s2) && (h1 == h2);
+        if (first + j < last) {
+            const uint64_t k = sb_step(sg, v[j], A, hg, NoEmit{});
+            cg += k;
+            if (!synced) {
+                ct += (int64_t)sb_step(st, v[j], A, ht, NoEmit{});
+                cg_sync += (int64_t)k;
+                synced = (st == sg) && (ht == hg);
+            }
         }
     }
-    A.ok[b] = ok;
-    A.delta[b] = c1 - c2;
+    A.spec_exit[b] = sg;
+    A.spec_cnt[b] = cg;
+    A.ok[b] = synced ? 1u : 0u;
+    A.delta[b] = ct - cg_sync;
 }
 
-// One CTA: entries, offsets, totals and the streaming state.
+// One CTA: entries, offsets, totals and the streaming state.  Each thread owns a contiguous
+// range of blocks; one block scan of the range sums gives every block's offset.
 __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
+    __shared__ uint32_t ws[33];
     __shared__ uint64_t wsum[33];
-    __shared__ int all_ok;
     if (A.aux->dense) return;
     const uint64_t n = sb_n(A);
     const uint32_t nb = (uint32_t)((n + SB_B - 1) / SB_B);
     const uint32_t tid = threadIdx.x;
-    if (tid == 0) all_ok = 1;
-    __syncthreads();
-    for (uint32_t b = tid; b < nb; b += blockDim.x)
-        if (!A.ok[b]) all_ok = 0;
-    __syncthreads();
+    const uint32_t per = (nb + blockDim.x - 1) / blockDim.x;
+    const uint32_t ba = min(nb, tid * per), bb = min(nb, ba + per);
+    uint64_t sum = 0;
+    uint32_t bad = 0;
+    for (uint32_t b = ba; b < bb; ++b) {
+        sum += (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]);
+        bad |= A.ok[b] ^ 1u;
+    }
+    const int all_ok = __syncthreads_and(bad == 0);
     Aux *aux = A.aux;
     const uint64_t held_prev = aux->held;
     const uint64_t base0 = aux->out_pos + held_prev;
     if (all_ok) {
-        // exclusive scan of true counts, in chunks of 1024 with a carry
-        uint64_t carry = 0;
-        for (uint32_t b0 = 0; b0 < nb; b0 += blockDim.x) {
-            const uint32_t b = b0 + tid;
-            const uint64_t v = b < nb ? (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]) : 0ull;
-            uint64_t incl = v;
-            for (int d = 1; d < 32; d <<= 1) {
-                uint64_t u = __shfl_up_sync(0xffffffffu, incl, d);
-                if ((tid & 31) >= (uint32_t)d) incl += u;
-            }
-            if ((tid & 31) == 31) wsum[tid >> 5] = incl;
-            __syncthreads();
-            if (tid == 0) {
-                uint64_t r = 0;
-                for (int w = 0; w < 32; ++w) { uint64_t x = wsum[w]; wsum[w] = r; r += x; }
-                wsum[32] = r;
-            }
-            __syncthreads();
-            if (b < nb) {
-                A.offs[b] = base0 + carry + wsum[tid >> 5] + incl - v;
-                A.entry[b] = b ? A.spec_exit[b - 1] : aux->s;
-            }
-            carry += wsum[32];
-            __syncthreads();
+        uint64_t incl = sum;
+        for (int d = 1; d < 32; d <<= 1) {
+            uint64_t u = __shfl_up_sync(0xffffffffu, incl, d);
+            if ((tid & 31) >= (uint32_t)d) incl += u;
         }
+        if ((tid & 31) == 31) wsum[tid >> 5] = incl;
+        __syncthreads();
+        if (tid == 0) {
+            uint64_t r = 0;
+            for (int w = 0; w < 32; ++w) { uint64_t x = wsum[w]; wsum[w] = r; r += x; }
+            wsum[32] = r;
+        }
+        __syncthreads();
+        uint64_t off = base0 + wsum[tid >> 5] + incl - sum;
+        for (uint32_t b = ba; b < bb; ++b) {
+            A.offs[b] = off;
+            A.entry[b] = b ? A.spec_exit[b - 1] : aux->s;
+            off += (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]);
+        }
+        const uint64_t carry = wsum[32];
         if (tid == 0) {
             const uint64_t s_last = nb ? A.spec_exit[nb - 1] : aux->s;
             // the held flag of the piece: the last candidate accepted exactly at `end`
