@@ -342,10 +342,10 @@ struct BulkCtx {
     uint32_t rsh;       // r << (32-m)
 };
 
-// One byte step, K63 (deg P = 63, fully reduced u64 state f = fh:fl, f < 2^63):
-//   t = f >> 55;  f <- (f << 8 mod 2^64) ^ B ^ T[t] ^ U[o]
-//   T[t] = (t x^63 mod P) ^ ((t & 1) << 63) cancels the bit the shift leaves at 2^63,
-//   U[o] = o x^{8w} mod P.   Shift-in by two byte permutes (PRMT).
+// One byte step, u64 state (deg P = k in 41..63; the paper's reading k = 63), f = fh:fl < 2^k:
+//   t = f >> (k-8) = mulhi(fh, 2^(72-k));  f <- (f << 8 mod 2^64) ^ B ^ T[t] ^ U[o]
+//   T[t] = (t x^k mod P) ^ ((t << k) mod 2^64) cancels the byte the shift leaves at bits
+//   k..k+7 (k = 63: the one bit at 2^63), U[o] = o x^{8w} mod P.  Shift-in by two PRMTs.
 template <int K>
 __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, uint32_t pop,
                                        const BulkCtx &c) {
@@ -360,7 +360,8 @@ __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, 
     fh = nh ^ T.y ^ U.y;
 }
 
-// One byte step, K32 (deg P = 32, u32 state): f <- (f << 8) ^ B ^ T[f >> 24] ^ U[o].
+// One byte step, u32 state (deg P = k in 9..32): t = mulhi(f, 2^(40-k)) = f >> (k-8),
+// f <- (f << 8 mod 2^32) ^ B ^ T[t] ^ U[o], T[t] = (t x^k mod P) ^ ((t << k) mod 2^32).
 template <int K>
 __device__ __forceinline__ void step32(uint32_t &f, uint32_t in, uint32_t pop, const BulkCtx &c) {
     const uint32_t ti = __umulhi(f, c.mhi) * c.m256 + c.laneT;

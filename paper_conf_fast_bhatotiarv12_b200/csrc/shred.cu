@@ -325,7 +325,8 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         }
         const int m = 32 - (int)__builtin_ctzll(ctx->p.divisor);     // D = 2^(32-m')
         BulkConst K;
-        K.mhi = ctx->path == SHRED_PATH_K63 ? 512u : 256u;
+        // top byte t = f >> (k-8): u64 state mulhi(f_hi, 2^(72-k)); u32 state mulhi(f, 2^(40-k))
+        K.mhi = ctx->path == SHRED_PATH_K63 ? (1u << (72 - ctx->k)) : (1u << (40 - ctx->k));
         K.m256 = 256u;
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
@@ -512,8 +513,9 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
     const bool fast_w = p->window == 16 || p->window == 32 || p->window == 48 || p->window == 64;
     const bool fast = fast_w && pow2 && p->divisor <= (1ull << 32);
-    if (k == 63 && fast) ctx->path = SHRED_PATH_K63;
-    else if (k == 32 && fast) ctx->path = SHRED_PATH_K32;
+    // u64-state kernel: deg 41..63 (t = mulhi(f_hi, 2^(72-k))); u32-state kernel: deg 9..32
+    if (k >= 41 && k <= 63 && fast) ctx->path = SHRED_PATH_K63;
+    else if (k >= 9 && k <= 32 && fast) ctx->path = SHRED_PATH_K32;
     else ctx->path = SHRED_PATH_GENERIC;
     if (major != 10) ctx->path = SHRED_PATH_GENERIC;   // the TMA kernels are built for sm_100a only
 
@@ -524,11 +526,11 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     GenTables gt;
     for (int t = 0; t < 256; ++t) { gt.T[t] = Tk[t]; gt.U[t] = U[t]; }
     std::vector<uint8_t> img(TAB_BYTES, 0);
+    // Fast-path T entries carry the cancel term (t << k) mod 2^W: after (f << 8) mod 2^W the top
+    // byte t of f sits at bits k..k+7 (those below W); T[t] removes it and adds t x^k mod P.
     if (ctx->path == SHRED_PATH_K63) {
-        uint64_t T63[256];
-        byte_times_xpow(p->poly, k, 63, T63);                     // t x^63 mod P
         for (int t = 0; t < 256; ++t) {
-            uint64_t tv = T63[t] ^ ((uint64_t)(t & 1) << 63);     // cancel bit left at 2^63
+            uint64_t tv = Tk[t] ^ ((uint64_t)t << k);             // W = 64 (k = 63: (t&1) << 63)
             for (int r = 0; r < 16; ++r) {
                 memcpy(&img[t * 256 + r * 8], &tv, 8);
                 memcpy(&img[t * 256 + 128 + r * 8], &U[t], 8);
@@ -536,7 +538,7 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         }
     } else if (ctx->path == SHRED_PATH_K32) {
         for (int t = 0; t < 256; ++t) {
-            uint32_t tv = (uint32_t)Tk[t], uv = (uint32_t)U[t];
+            uint32_t tv = (uint32_t)(Tk[t] ^ ((uint64_t)t << k)), uv = (uint32_t)U[t];   // W = 32
             for (int r = 0; r < 32; ++r) {
                 memcpy(&img[t * 256 + r * 4], &tv, 4);
                 memcpy(&img[t * 256 + 128 + r * 4], &uv, 4);

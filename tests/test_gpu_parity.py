@@ -292,3 +292,24 @@ def test_fast_path_windows_and_le_marker(pkg, poly, path, window, marker):
     ch = pkg.Chunker(p)
     assert ch.path == path
     check_chunk(ch, synthgen.random_bytes(window + marker, (3 << 20) + 31), offset=5)
+
+
+def _dense_irreducible(deg, seed):
+    rng = np.random.default_rng(seed)
+    while True:
+        low = int(rng.integers(0, 1 << min(deg, 62))) | 1
+        p = (1 << deg) | (low & ((1 << deg) - 1))
+        if oracle.is_irreducible(p):
+            return p
+
+
+@pytest.mark.parametrize("deg", [8, 9, 12, 16, 24, 31, 32, 33, 40, 41, 48, 57, 62, 63])
+def test_polynomial_degrees(pkg, deg):
+    """Any degree: u32-state fast kernel for 9..32, u64-state for 41..63, generic otherwise
+    (T tables with the (t << k) cancel term); dense random irreducible P, bit-exact."""
+    P = _dense_irreducible(deg, deg)
+    D = 1 << min(10, deg - 1)
+    p = pkg.Params(poly=P, divisor=D, magic=D // 3)
+    ch = pkg.Chunker(p)
+    assert ch.path == ("k32" if 9 <= deg <= 32 else "k63" if deg >= 41 else "generic")
+    check_chunk(ch, synthgen.random_bytes(deg, (2 << 20) + 123), offset=deg % 16)
