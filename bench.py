@@ -458,7 +458,21 @@ def main():
                 ch.hash_chunks_async(base, out0, n0, dig)
             h2.record(stream)
             torch.cuda.synchronize()
+            # the same on bounded chunks (min 2048 / max 65536): the longest chunk is capped
+            ob = torch.empty(cap, dtype=torch.int64, device=dev)
+            nb_ = torch.zeros(1, dtype=torch.int64, device=dev)
+            chb.chunk_async(base, ob, nb_)
+            chb.hash_chunks_async(base, ob, nb_, dig)
+            torch.cuda.synchronize()
+            g0, g1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            g0.record(stream)
+            for _ in range(3):
+                chb.hash_chunks_async(base, ob, nb_, dig)
+            g1.record(stream)
+            torch.cuda.synchronize()
+            hb = round(3 * base.numel() / (g0.elapsed_time(g1) * 1e-3) / 1e9, 2)
             line["hash_sha256"] = {"value": round(3 * base.numel() / (h0.elapsed_time(h1) * 1e-3) / 1e9, 2),
+                                   "bounded_chunks_value": hb,
                                    "unit": "GB/s", "chunks": int(n0.item()) + 1,
                                    "chunk_plus_hash": round(3 * base.numel() / (h1.elapsed_time(h2) * 1e-3) / 1e9, 2),
                                    "note": "SURVEY §8(f) f2: SHA-256 per chunk of the 1 GiB base file"}

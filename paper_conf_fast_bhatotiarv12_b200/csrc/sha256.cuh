@@ -147,9 +147,19 @@ __global__ void k_hash_scatter(const uint64_t *__restrict__ cuts, const uint64_t
     }
 }
 
+__device__ __forceinline__ void sha256_store(uint8_t *digests, uint64_t chunk, const uint32_t (&H)[8]) {
+    uint4 *o = reinterpret_cast<uint4 *>(digests + chunk * 32);
+    o[0] = make_uint4(__byte_perm(H[0], 0, 0x0123), __byte_perm(H[1], 0, 0x0123),
+                      __byte_perm(H[2], 0, 0x0123), __byte_perm(H[3], 0, 0x0123));
+    o[1] = make_uint4(__byte_perm(H[4], 0, 0x0123), __byte_perm(H[5], 0, 0x0123),
+                      __byte_perm(H[6], 0, 0x0123), __byte_perm(H[7], 0, 0x0123));
+}
+
 // Hash every chunk.  nchunks = (*n_cuts + 1 if len > 0 else 0); chunk i ends at cuts[i]
 // (i < n) or len.  digests: 32 bytes per chunk (the SHA-256 digest bytes in order).
 // Warps take 32 consecutive entries of the length-sorted `order` at a time from `queue`.
+// Launched with one warp per SM sub-partition: the sequential SHA chain of the longest chunks
+// bounds the run, so few warps (each issuing at full rate) beat many (profiles/r01_hash_ab.txt).
 __global__ void __launch_bounds__(256)
 k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__restrict__ cuts,
               const uint64_t *n_cuts, uint64_t max_chunks, uint8_t *__restrict__ digests,
@@ -174,11 +184,7 @@ k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__re
                 sha256_block(in, len, a, L, blk, W);
                 sha256_compress(H, W);
             }
-            uint4 *o = reinterpret_cast<uint4 *>(digests + chunk * 32);
-            o[0] = make_uint4(__byte_perm(H[0], 0, 0x0123), __byte_perm(H[1], 0, 0x0123),
-                              __byte_perm(H[2], 0, 0x0123), __byte_perm(H[3], 0, 0x0123));
-            o[1] = make_uint4(__byte_perm(H[4], 0, 0x0123), __byte_perm(H[5], 0, 0x0123),
-                              __byte_perm(H[6], 0, 0x0123), __byte_perm(H[7], 0, 0x0123));
+            sha256_store(digests, chunk, H);
         }
         __syncwarp();
     }

@@ -10,6 +10,13 @@
 #include "size_bound.cuh"
 #include "sha256.cuh"
 #include "dedup.cuh"
+
+#ifndef SHRED_HASH_CTAS_PER_SM
+#define SHRED_HASH_CTAS_PER_SM 1
+#endif
+#ifndef SHRED_HASH_THREADS
+#define SHRED_HASH_THREADS 128                // one warp per SM sub-partition
+#endif
 #include "../../include/shred.h"
 
 #include <cstdarg>
@@ -846,7 +853,7 @@ int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const u
     LAUNCHED("k_hash_scan");
     k_hash_scatter<<<gs, 256, 0, st>>>(d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist, ctx->d_order);
     LAUNCHED("k_hash_scatter");
-    k_hash_chunks<<<ctx->sm_count * 4, 256, 0, st>>>(d_in, len, d_cuts, d_ncuts, max_chunks, d_digests,
+    k_hash_chunks<<<ctx->sm_count * SHRED_HASH_CTAS_PER_SM, SHRED_HASH_THREADS, 0, st>>>(d_in, len, d_cuts, d_ncuts, max_chunks, d_digests,
                                                       ctx->d_order, ctx->d_queue);
     LAUNCHED("k_hash_chunks");
     return SHRED_OK;
