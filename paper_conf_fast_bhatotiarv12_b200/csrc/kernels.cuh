@@ -108,9 +108,13 @@ struct DevParams {              // chunking parameters as the kernels need them
     uint32_t marker;            // 0: fp mod D == r; 1: fp mod D <= r
 };
 
-// The marker predicate of the generic path (L247-L251, L447-L451).
+// The marker predicate of the generic path (L247-L251, L447-L451).  The 64-bit modulo is a
+// software division: keep it behind a real branch so power-of-two divisors never pay for it.
+__device__ __noinline__ uint64_t mod_u64(uint64_t f, uint64_t d) { return f % d; }
 __device__ __forceinline__ bool generic_marker(uint64_t f, const DevParams &P) {
-    const uint64_t v = P.pow2 ? (f & P.dmask) : (f % P.divisor);
+    uint64_t v;
+    if (P.pow2) v = f & P.dmask;
+    else v = mod_u64(f, P.divisor);
     return P.marker ? (v <= P.magic) : (v == P.magic);
 }
 
@@ -199,6 +203,11 @@ __device__ __forceinline__ bool mbar_try_wait(uint32_t bar, uint32_t parity) {
 // instructions).
 __device__ __forceinline__ void mbar_wait_sleep(uint32_t bar, uint32_t parity) {
     while (!mbar_try_wait(bar, parity)) __nanosleep(SHRED_PRODUCER_SLEEP_NS);
+}
+// 1-D bulk copy global -> shared (TMA engine), completing on an mbarrier.
+__device__ __forceinline__ void bulk_g2s(uint32_t dst, const void *src, uint32_t bytes, uint32_t bar) {
+    asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];"
+                 :: "r"(dst), "l"(src), "r"(bytes), "r"(bar) : "memory");
 }
 __device__ __forceinline__ void tma_load_2d(uint32_t dst, const CUtensorMap *map, int x, int y,
                                             uint32_t bar) {
@@ -523,15 +532,21 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         return;
     }
 
-    for (int i = tid; i < TAB_BYTES / 16; i += blockDim.x)
-        reinterpret_cast<uint4 *>(smem)[i] = tab_img[i];
+    // the 64 KiB T|U image arrives by TMA bulk copies (tabbar), overlapping the set-up below
+    const uint32_t tabbar = bars + 120;
     if (tid == 0) {
         for (int s = 0; s < STAGES; ++s) {
             mbar_init(bars + 8 * s, 1);
             mbar_init(bars + 64 + 8 * s, NTC / 32);
         }
+        mbar_init(tabbar, 1);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
         asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+        mbar_expect_tx(tabbar, TAB_BYTES);
+#pragma unroll
+        for (int q = 0; q < 4; ++q)
+            bulk_g2s(sbase + q * (TAB_BYTES / 4), reinterpret_cast<const uint8_t *>(tab_img) + q * (TAB_BYTES / 4),
+                     TAB_BYTES / 4, tabbar);
     }
     __syncthreads();
 
@@ -580,6 +595,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         o[ch].lst = J.scratch + (uint64_t)(J.map.n_head + row) * J.cap;
         o[ch].cnt = 0; o[ch].cap = J.cap;
     }
+    mbar_wait(tabbar, 0);                             // T|U image resident
     {
         // warm-up: the 64 bytes before each row (b0 >= p_begin + 64 keeps them inside src)
         const uint4 Z = make_uint4(0, 0, 0, 0);

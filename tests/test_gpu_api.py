@@ -144,3 +144,33 @@ def test_feed_edge_cases_mixed_sources_and_empty(pkg):
     ch = pkg.Chunker(pkg.Params())
     x = torch.from_numpy(data[:47].copy()).cuda()
     assert ch.candidates_range(x, 47, 47, n).numel() == 0      # halo only, empty range
+
+
+@pytest.mark.parametrize("bounded", [False, True])
+def test_cuda_graph_capture_and_replay(pkg, bounded):
+    """A shred_chunk call (after a warm-up call sized its scratch) can be captured into a CUDA
+    graph and replayed: the launch-bound small-input case (configs[0]) without per-call launch
+    overhead.  Replays on new bytes (same buffer) give the new exact result."""
+    n = (1 << 20) + 77
+    p = pkg.Params(min_size=2048, max_size=65536) if bounded else pkg.Params()
+    ch = pkg.Chunker(p)
+    x = torch.empty(n, dtype=torch.uint8, device="cuda")
+    out = torch.empty(4096, dtype=torch.int64, device="cuda")
+    cnt = torch.zeros(1, dtype=torch.int64, device="cuda")
+    pkg.synth_fill(x, 1)
+    s = torch.cuda.Stream()
+    with torch.cuda.stream(s):
+        ch.chunk_async(x, out, cnt, stream=s)                # warm-up: sizes the ctx scratch
+    torch.cuda.synchronize()
+    g = torch.cuda.CUDAGraph()
+    with torch.cuda.graph(g, stream=s):
+        ch.chunk_async(x, out, cnt, stream=s)
+    op = oracle.Params(min_size=p.min_size, max_size=p.max_size)
+    for seed in (1, 2, 3):
+        pkg.synth_fill(x, seed)
+        torch.cuda.synchronize()
+        g.replay()
+        torch.cuda.synchronize()
+        k = int(cnt.item())
+        exp = oracle.chunk(synthgen.random_bytes(seed, n), op)
+        assert np.array_equal(out[:k].cpu().numpy().astype(np.uint64), exp)
