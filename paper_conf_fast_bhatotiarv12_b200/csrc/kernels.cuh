@@ -39,7 +39,7 @@
 
 namespace shred {
 
-enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3 };
+enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3, MODE_K32B = 4 };   // K32B: deg 16/24/32
 
 constexpr int STAGES      = 4;                 // TMA ring depth
 constexpr int BOX_ROWS    = 256;               // rows per TMA box (hardware max 256)
@@ -349,6 +349,7 @@ struct BulkCtx {
     uint32_t m256;      // 256 (row stride of the table image)
     uint32_t tmul;      // 2^(32-m): (f_lo * tmul) keeps the low m bits at the top
     uint32_t rsh;       // r << (32-m)
+    uint32_t tsel;      // K32B: PRMT selector 0x55s4 placing byte s = (k-8)/8 of f at bits 8..15
 };
 
 // One byte step, u64 state (deg P = k in 41..63; the paper's reading k = 63), f = fh:fl < 2^k:
@@ -371,9 +372,13 @@ __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, 
 
 // One byte step, u32 state (deg P = k in 9..32): t = mulhi(f, 2^(40-k)) = f >> (k-8),
 // f <- (f << 8 mod 2^32) ^ B ^ T[t] ^ U[o], T[t] = (t x^k mod P) ^ ((t << k) mod 2^32).
-template <int K>
+template <int K, bool BYTEIDX>
 __device__ __forceinline__ void step32(uint32_t &f, uint32_t in, uint32_t pop, const BulkCtx &c) {
-    const uint32_t ti = __umulhi(f, c.mhi) * c.m256 + c.laneT;
+    uint32_t ti;
+    if (BYTEIDX)   // deg 16/24/32: t = f >> (k-8) is a whole byte -> one PRMT builds (t << 8) | lane*4
+        ti = c.tab + __byte_perm(f, c.laneT - c.tab, c.tsel);
+    else
+        ti = __umulhi(f, c.mhi) * c.m256 + c.laneT;
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
     const uint32_t T = lds32(ti);
     const uint32_t U = lds32(c.tab + oi);
@@ -392,7 +397,14 @@ template <> struct State<MODE_K63> {
 template <> struct State<MODE_K32> {
     uint32_t f = 0;
     template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
-        step32<K>(f, in, pop, c);
+        step32<K, false>(f, in, pop, c);
+    }
+    __device__ __forceinline__ uint32_t low() const { return f; }
+};
+template <> struct State<MODE_K32B> {
+    uint32_t f = 0;
+    template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
+        step32<K, true>(f, in, pop, c);
     }
     __device__ __forceinline__ uint32_t low() const { return f; }
 };
@@ -489,7 +501,7 @@ __device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d
     word4xN<MODE, CH, TEST, 3, LE>(st, in, po, m, c);
 }
 
-struct BulkConst { uint32_t mhi, m256, tmul, rsh; };
+struct BulkConst { uint32_t mhi, m256, tmul, rsh, tsel; };
 
 // The hot kernel.  blockDim = NTC consumers + 1 producer warp; one CTA per SM.
 // blockIdx < nc: bulk CTA, rows blockIdx*ROWS + tid + ch*NTC (ch < CH); blockIdx == nc: the
@@ -580,7 +592,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         c.laneT = sbase + (uint32_t)lane * 4u;
         c.laneU = 128u + (uint32_t)lane * 4u;
     }
-    c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh;
+    c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh; c.tsel = K.tsel;
 
     bool act[CH];
     uint64_t pos0[CH];

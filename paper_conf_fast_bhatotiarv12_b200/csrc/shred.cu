@@ -99,9 +99,11 @@ K1Fn pick_mode(int wch, bool le) {
         default: return nullptr;
     }
 }
-// The hot-kernel instance for (deg 63 | 32, w/16, marker set).
-K1Fn pick_k1(bool k63, int wch, bool le) {
-    return k63 ? pick_mode<MODE_K63, CfgK63>(wch, le) : pick_mode<MODE_K32, CfgK32>(wch, le);
+// The hot-kernel instance for (u64 state | u32 state with a whole-byte top byte | u32 state,
+// w/16, marker set).
+K1Fn pick_k1(bool k63, bool byteidx, int wch, bool le) {
+    if (k63) return pick_mode<MODE_K63, CfgK63>(wch, le);
+    return byteidx ? pick_mode<MODE_K32B, CfgK32>(wch, le) : pick_mode<MODE_K32, CfgK32>(wch, le);
 }
 
 typedef CUresult (*EncodeTiledFn)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *,
@@ -337,6 +339,7 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         K.m256 = 256u;
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
+        K.tsel = 0x5504u | ((uint32_t)((ctx->k - 8) / 8) << 4);         // byte (k-8)/8 -> bits 8..15
         const int smem = ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM;
         const int threads = (ctx->path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC) + 32;
         ctx->k1_fn<<<pl.bulk_ctas, threads, smem, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
@@ -576,7 +579,9 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fn, cudaEnableDefault, &q) != cudaSuccess || !fn)
             return bail(SHRED_ECUDA);
         ctx->encode = (EncodeTiledFn)fn;
-        ctx->k1_fn = pick_k1(ctx->path == SHRED_PATH_K63, (int)(p->window / 16), p->marker == SHRED_MARKER_LE);
+        const bool byteidx = ctx->path == SHRED_PATH_K32 && (k == 16 || k == 24 || k == 32);
+        ctx->k1_fn = pick_k1(ctx->path == SHRED_PATH_K63, byteidx, (int)(p->window / 16),
+                             p->marker == SHRED_MARKER_LE);
         if (!ctx->k1_fn ||
             cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM) != cudaSuccess)
