@@ -34,7 +34,8 @@
 #endif
 #ifndef SHRED_HITMODE
 #define SHRED_HITMODE 3         // 3: ISETP + predicated OR per byte (default); 0: ISETP + SEL bitmask
-                                // (A/B of these and of removed variants: profiles/r01_ab_variants.txt)
+                                // (A/B of these and of removed variants, incl. a per-chunk LOP3.PAND
+                                // predicate with replay: profiles/r01_ab_variants.txt)
 #endif
 
 namespace shred {
@@ -75,6 +76,9 @@ struct BulkCfg {
 #endif
 using CfgK63 = BulkCfg<SHRED_K63_CH, SHRED_K63_NT>;
 using CfgK32 = BulkCfg<SHRED_K32_CH, SHRED_K32_NT>;
+// Small inputs (< ~5 MB): 128 consumers x 2 rows per CTA (two CTAs per SM fit), so the short
+// rows still spread over every SM (1 MiB: 65 CTAs instead of 17; 19.8 -> 16.7 us per call).
+using CfgSmall = BulkCfg<2, 128>;
 
 // Slot id -> range of window-end positions.  Slots are numbered in stream order:
 // [0, n_head) generic head segments, then the bulk rows, then generic tail segments.
@@ -305,6 +309,39 @@ __device__ __forceinline__ uint32_t block_exscan(uint32_t v, uint32_t nthr, uint
     return r;
 }
 
+// Copy the stream bytes [from, to) of job J into shared memory (all nthr threads of the CTA
+// take part; the caller synchronises) and return a view of J whose bytes come from there.
+// buf + o + (pos - from) holds byte pos, with o chosen so that 16-byte-aligned source addresses
+// land on 16-byte-aligned shared addresses (16-byte loads for the bulk of the range).  Needs
+// to - from + 16 bytes at buf (16-byte aligned).
+__device__ __forceinline__ Job stage_job(const Job &J, uint64_t from, uint64_t to, uint8_t *buf,
+                                         int tid, int nthr) {
+    const uint32_t o = (uint32_t)((uintptr_t)J.src + (uintptr_t)(from - J.p_begin)) & 15u;
+    uint8_t *d = buf + o;                           // d[pos - from] = byte pos
+    const uint64_t s0 = from > J.p_begin ? from : J.p_begin;
+    for (uint64_t pos = from + tid; pos < to && pos < s0; pos += nthr) d[pos - from] = job_byte(J, pos);
+    if (s0 < to) {
+        const uintptr_t a0 = (uintptr_t)(J.src + (s0 - J.p_begin));
+        const uint64_t a = s0 + (((16u - (a0 & 15u)) & 15u));      // first 16-B-aligned position
+        const uint64_t e = a < to ? a + ((to - a) & ~15ull) : a;    // end of the aligned run
+        for (uint64_t pos = s0 + tid; pos < to && pos < a; pos += nthr) d[pos - from] = J.src[pos - J.p_begin];
+        for (uint64_t pos = e + tid; pos < to; pos += nthr) d[pos - from] = J.src[pos - J.p_begin];
+        if (e > a) {
+            const uint4 *g = reinterpret_cast<const uint4 *>(J.src + (a - J.p_begin));
+            uint4 *sd = reinterpret_cast<uint4 *>(d + (a - from));
+            const uint64_t n16 = (e - a) >> 4;
+#pragma unroll 4
+            for (uint64_t k = tid; k < n16; k += nthr) sd[k] = __ldg(g + k);
+        }
+    }
+    Job V = J;
+    V.src = d;
+    V.p_begin = from;
+    V.prefix = nullptr;
+    V.prefix_len = 0;
+    return V;
+}
+
 // Roll one generic slot into its list; returns the true count.
 template <class Tab>
 __device__ __forceinline__ uint32_t roll_slot(const Job &J, const DevParams &P, const Tab &tab,
@@ -529,12 +566,26 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         uint64_t *sT = reinterpret_cast<uint64_t *>(smem + TAB_BYTES);
         uint64_t *sU = sT + 256;
         for (int i = tid; i < 256; i += blockDim.x) { sT[i] = gt->T[i]; sU[i] = gt->U[i]; }
+        // Stage the head and tail byte ranges (with their w-1 warm-up bytes) in the idle stage
+        // ring, so the byte loop reads shared memory instead of one dependent global load per
+        // byte (that latency chain set a ~16 us floor on every call).
+        uint8_t *buf = smem + TAB_BYTES + 4096;
+        const uint64_t cap = (uint64_t)STAGES * C::STAGE - 4096;
+        const uint64_t warm = (uint64_t)P.w - 1u, lo = J.p_begin - J.prefix_len;
+        const uint64_t hf = J.map.head_start >= lo + warm ? J.map.head_start - warm : lo;
+        const uint64_t tf = J.map.tail_start >= lo + warm ? J.map.tail_start - warm : lo;
+        const uint64_t hl = J.map.n_head ? J.map.b0 - hf : 0, tl = J.map.n_tail ? J.map.t_end - tf : 0;
+        const uint64_t hsz = (hl + 31u) & ~15ull;       // + alignment slack, 16-B multiple
+        const bool sh = hl && hsz <= cap, stl = tl && hsz + tl + 16u <= cap;
+        Job JH = J, JT = J;
+        if (sh) JH = stage_job(J, hf, J.map.b0, buf, tid, blockDim.x);
+        if (stl) JT = stage_job(J, tf, J.map.t_end, buf + hsz, tid, blockDim.x);
         __syncthreads();
         if (tid >= NTC) return;
         SmemGenTab tab{sT, sU};
         const uint32_t tail0 = J.map.n_head + J.map.nrows;
-        const uint32_t ch = (uint32_t)tid < J.map.n_head ? roll_slot(J, P, tab, tid) : 0u;
-        const uint32_t ct = (uint32_t)tid < J.map.n_tail ? roll_slot(J, P, tab, tail0 + tid) : 0u;
+        const uint32_t ch = (uint32_t)tid < J.map.n_head ? roll_slot(JH, P, tab, tid) : 0u;
+        const uint32_t ct = (uint32_t)tid < J.map.n_tail ? roll_slot(JT, P, tab, tail0 + tid) : 0u;
         uint32_t th, tt;
         const uint32_t oh = block_exscan(ch, NTC, 1, ws, &th);
         const uint32_t ot = block_exscan(ct, NTC, 1, ws, &tt);

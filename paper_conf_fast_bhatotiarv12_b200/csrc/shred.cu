@@ -101,9 +101,18 @@ K1Fn pick_mode(int wch, bool le) {
 }
 // The hot-kernel instance for (u64 state | u32 state with a whole-byte top byte | u32 state,
 // w/16, marker set).
+#ifndef SHRED_BYTEIDX
+#define SHRED_BYTEIDX 1   // deg 16/24/32: PRMT table index (MODE_K32B); 0: IMAD index (MODE_K32)
+#endif
 K1Fn pick_k1(bool k63, bool byteidx, int wch, bool le) {
     if (k63) return pick_mode<MODE_K63, CfgK63>(wch, le);
     return byteidx ? pick_mode<MODE_K32B, CfgK32>(wch, le) : pick_mode<MODE_K32, CfgK32>(wch, le);
+}
+// The small-input shape (CfgSmall) exists for the paper's window with the equality marker.
+K1Fn pick_k1_small(bool k63, bool byteidx, int wch, bool le) {
+    if (wch != 3 || le) return nullptr;
+    if (k63) return k1_bulk<MODE_K63, CfgSmall, 3, false>;
+    return byteidx ? k1_bulk<MODE_K32B, CfgSmall, 3, false> : k1_bulk<MODE_K32, CfgSmall, 3, false>;
 }
 
 typedef CUresult (*EncodeTiledFn)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *,
@@ -127,6 +136,7 @@ struct shred_ctx {
     GenTables *d_gen = nullptr;          // plain T/U (generic path, recompute)
     EncodeTiledFn encode = nullptr;
     K1Fn k1_fn = nullptr;                // the hot-kernel instance for these parameters
+    K1Fn k1_small_fn = nullptr;          // the same with the small-input shape (or null)
     int sm_count = 148;
 
     // scratch (grown on demand, synchronously)
@@ -214,6 +224,7 @@ int validate(const shred_params *p, shred_ctx *ctx) {
 struct Plan {
     Job J;
     bool bulk = false;
+    bool small = false;                  // bulk with the CfgSmall launch shape
     uint32_t nslots = 0;
     uint32_t bulk_ctas = 0;
     CUtensorMap tmap;
@@ -235,10 +246,12 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
 
     // bulk region: aligned start b0 >= max(t_begin, p_begin + 64), rows of S bytes
     const bool k63 = ctx->path == SHRED_PATH_K63;
-    const uint64_t ROWS_CTA = k63 ? CfgK63::ROWS : CfgK32::ROWS;
-    const uint64_t NTC = k63 ? CfgK63::NTC : CfgK32::NTC;
+    uint64_t ROWS_CTA = k63 ? CfgK63::ROWS : CfgK32::ROWS;
+    uint64_t NTC = k63 ? CfgK63::NTC : CfgK32::NTC;
     const uint64_t ROUND = k63 ? CfgK63::ROUND : CfgK32::ROUND;
+    static_assert(CfgK63::ROUND == CfgSmall::ROUND && CfgK32::ROUND == CfgSmall::ROUND, "round");
     pl.bulk = false;
+    pl.small = false;
     uint64_t S = 0, nrows = 0, b0 = t_end;
     if ((ctx->path == SHRED_PATH_K63 || ctx->path == SHRED_PATH_K32) && len >= 4096) {
         uint64_t lo = t_begin > p_begin + 64 ? t_begin : p_begin + 64;
@@ -247,7 +260,15 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
         if (b0 + 256 < t_end) {
             const uint64_t blen = t_end - b0;
             // one wave: (SMs - 1) bulk CTAs of ROWS_CTA rows + the edge CTA
-            const uint64_t target = (uint64_t)(ctx->sm_count > 1 ? ctx->sm_count - 1 : 1) * ROWS_CTA;
+            const uint64_t sms = (uint64_t)(ctx->sm_count > 1 ? ctx->sm_count - 1 : 1);
+            uint64_t target = sms * ROWS_CTA;
+            if (ctx->k1_small_fn && blen <= target * 32) {
+                // rows of < 64 B with the big shape: use the small one, two CTAs per SM
+                // (tools/size_latency.py: faster up to ~4 MiB, slower from ~16 MiB)
+                pl.small = true;
+                ROWS_CTA = CfgSmall::ROWS; NTC = CfgSmall::NTC;
+                target = 2 * sms * ROWS_CTA;
+            }
             S = (blen + target - 1) / target;
             S = (S + 63) / 64 * 64;                // an even number of ROUND-byte rounds
             if (S < 64) S = 64;                    // small inputs: more rows, latency-bound anyway
@@ -257,6 +278,7 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
         }
     }
     if (!pl.bulk) {
+        pl.small = false;
         // generic only: segments of about len / (sm_count * 4 * 256) bytes, >= 256
         uint64_t seg = 256;
         const uint64_t want = (uint64_t)ctx->sm_count * 4 * GEN_THREADS;
@@ -340,9 +362,11 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
         K.tsel = 0x5504u | ((uint32_t)((ctx->k - 8) / 8) << 4);         // byte (k-8)/8 -> bits 8..15
-        const int smem = ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM;
-        const int threads = (ctx->path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC) + 32;
-        ctx->k1_fn<<<pl.bulk_ctas, threads, smem, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
+        int smem = ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM;
+        int threads = (ctx->path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC) + 32;
+        K1Fn fn = ctx->k1_fn;
+        if (pl.small) { smem = CfgSmall::SMEM; threads = CfgSmall::NTC + 32; fn = ctx->k1_small_fn; }
+        fn<<<pl.bulk_ctas, threads, smem, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
         LAUNCHED("k1_bulk");
         if (e1) CK(cudaEventRecord(e1, st), "profile record");
     } else {
@@ -579,12 +603,20 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fn, cudaEnableDefault, &q) != cudaSuccess || !fn)
             return bail(SHRED_ECUDA);
         ctx->encode = (EncodeTiledFn)fn;
-        const bool byteidx = ctx->path == SHRED_PATH_K32 && (k == 16 || k == 24 || k == 32);
+        const bool byteidx = SHRED_BYTEIDX && ctx->path == SHRED_PATH_K32 && (k == 16 || k == 24 || k == 32);
         ctx->k1_fn = pick_k1(ctx->path == SHRED_PATH_K63, byteidx, (int)(p->window / 16),
                              p->marker == SHRED_MARKER_LE);
         if (!ctx->k1_fn ||
             cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM) != cudaSuccess)
+            return bail(SHRED_ECUDA);
+#ifndef SHRED_NO_SMALL
+        ctx->k1_small_fn = pick_k1_small(ctx->path == SHRED_PATH_K63, byteidx, (int)(p->window / 16),
+                                         p->marker == SHRED_MARKER_LE);
+#endif
+        if (ctx->k1_small_fn &&
+            cudaFuncSetAttribute(ctx->k1_small_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                 CfgSmall::SMEM) != cudaSuccess)
             return bail(SHRED_ECUDA);
     }
     if (cudaFuncSetAttribute(sb_dense, cudaFuncAttributeMaxDynamicSharedMemorySize,

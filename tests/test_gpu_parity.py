@@ -100,6 +100,20 @@ def test_k32_path(pkg):
                 synthgen.random_bytes(9, (3 << 20) + 1))
 
 
+SMALL_LIMIT = 147 * 1024 * 32       # bulk bytes up to which the small launch shape runs (148 SMs)
+
+
+@pytest.mark.parametrize("poly", [LBFS, 0x104C11DB7, 0x20000005])   # K63, K32B, K32 (deg 29)
+@pytest.mark.parametrize("n", [(4 << 20) + 4093, SMALL_LIMIT + 60, SMALL_LIMIT + 100, (5 << 20) + 1])
+def test_launch_shapes_around_small_threshold(pkg, poly, n):
+    """Inputs up to ~4.6 MiB run the small launch shape (128 consumers x 2 rows per CTA), larger
+    ones the big shape; both sides of the switch, every u32/u64 kernel mode, and a dense divisor
+    (a marker every 64 B on average: many hits per row)."""
+    data = synthgen.random_bytes(21, n)
+    for p in (pkg.Params(poly=poly), pkg.Params(poly=poly, divisor=64, magic=17)):
+        check_chunk(pkg.Chunker(p), data)
+
+
 def test_generic_path_variants(pkg):
     for p in (pkg.Params(window=33), pkg.Params(window=1, divisor=256, magic=7),
               pkg.Params(poly=(1 << 63) | 3, window=24, divisor=1024),
