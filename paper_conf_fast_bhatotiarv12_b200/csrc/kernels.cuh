@@ -150,7 +150,7 @@ struct Aux {
     uint64_t overflow;          // sticky: an output did not fit
     uint64_t dense;             // the ordered candidate list did not fit (size-rule fallback)
     uint64_t ncand;             // candidates of the current piece (k_scatter; read by sb_*)
-    uint64_t pad;
+    uint64_t sb_fast;           // sb_plan: 1 = every block synced (two-level scan offsets)
 };
 
 // ------------------------------------------------------------------------------ PTX helpers

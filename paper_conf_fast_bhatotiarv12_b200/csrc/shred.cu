@@ -402,7 +402,7 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
                       uint64_t nmax, uint64_t end, int fin, uint64_t *dst, uint64_t cap, Aux *aux,
                       const Plan *pl, cudaStream_t st) {
     const uint64_t nb = (nmax + SB_B - 1) / SB_B;
-    int rc = grow(ctx, ctx->d_sb, ctx->sb_cap, 6 * (nb + 2), "size-rule scratch");
+    int rc = grow(ctx, ctx->d_sb, ctx->sb_cap, 9 * (nb + 2), "size-rule scratch");
     if (rc) return rc;
     SBArgs A;
     A.cand = cand; A.n_dev = n_dev; A.n_host = n_host;
@@ -410,15 +410,21 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
     uint64_t *b = ctx->d_sb;
     A.spec_exit = b; A.spec_cnt = b + (nb + 2); A.entry = b + 2 * (nb + 2); A.offs = b + 3 * (nb + 2);
     A.delta = (int64_t *)(b + 4 * (nb + 2)); A.ok = (uint32_t *)(b + 5 * (nb + 2));
+    A.cta_sum = b + 6 * (nb + 2); A.cta_ok = b + 7 * (nb + 2); A.cta_off = b + 8 * (nb + 2);
     A.dst = dst; A.dst_cap = cap; A.aux = aux;
-    const unsigned g = (unsigned)((nb + SB_THREADS - 1) / SB_THREADS);
+    // tiles of SB_THREADS blocks, at most 8 CTAs per SM (grid-stride over the true tile count)
+    const uint64_t gmax = (uint64_t)ctx->sm_count * 8;
+    uint64_t g = (nb + SB_THREADS - 1) / SB_THREADS;
+    if (g > gmax) g = gmax;
     if (nb) {
-        sb_spec_check<<<g, SB_THREADS, 0, st>>>(A);
+        sb_spec_check<<<(unsigned)g, SB_THREADS, 0, st>>>(A);
         LAUNCHED("sb_spec_check");
     }
     sb_plan<<<1, 1024, 0, st>>>(A);
     LAUNCHED("sb_plan");
-    sb_emit<<<(unsigned)((nb + 1 + SB_THREADS - 1) / SB_THREADS), SB_THREADS, 0, st>>>(A);
+    uint64_t ge = (nb + 1 + SB_THREADS - 1) / SB_THREADS;
+    if (ge > gmax) ge = gmax;
+    sb_emit<<<(unsigned)ge, SB_THREADS, 0, st>>>(A);
     LAUNCHED("sb_emit");
     if (pl && pl->nslots) {
         uint64_t maxseg = pl->J.map.S;

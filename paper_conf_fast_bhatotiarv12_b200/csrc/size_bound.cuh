@@ -13,9 +13,11 @@
 //             -> spec exit state, spec count; and, in lockstep, from e_b = the spec exit of
 //             block b-1 (recomputed by the same thread) until the two states coincide (sync)
 //             -> count delta; no sync -> not ok.
+//             Each CTA also reduces its blocks' counts and sync flags (cta_sum, cta_ok).
 //   sb_plan   one CTA: if every block synced, entries = spec exits and the offsets are a scan
-//             of the counts; otherwise warp 0 walks the blocks in order, re-walking the ones
-//             whose assumed entry does not hold (exact; serial only through those blocks).
+//             of the per-CTA sums (two-level scan: sb_emit adds the in-CTA prefix); otherwise
+//             warp 0 walks the blocks in order, re-walking the ones whose assumed entry does not
+//             hold (exact; serial only through those blocks) and writes every entry and offset.
 //   sb_emit   every block re-runs from its true entry and writes its cuts at its offset; one
 //             extra thread writes the forced cuts after the last candidate.
 // Streaming: `fin` = 1 for a whole stream (cuts < end = N); fin = 0 for a fed piece: an accepted
@@ -26,7 +28,10 @@
 
 namespace shred {
 
-constexpr int SB_B = 16;            // candidates per block (one thread; prefetched into registers)
+#ifndef SHRED_SB_B
+#define SHRED_SB_B 16
+#endif
+constexpr int SB_B = SHRED_SB_B;    // candidates per block (one thread; prefetched into registers)
 constexpr int SB_THREADS = 128;
 
 struct SBArgs {
@@ -39,6 +44,7 @@ struct SBArgs {
     uint64_t *spec_exit, *spec_cnt, *entry, *offs;   // [nb] each
     int64_t *delta;
     uint32_t *ok;
+    uint64_t *cta_sum, *cta_ok, *cta_off;            // [ncta] per spec_check CTA (two-level scan)
     uint64_t *dst; uint64_t dst_cap;
     Aux *aux;                       // s, held, held_val, out_pos (streaming state)
 };
@@ -72,48 +78,70 @@ __device__ __forceinline__ uint64_t sb_tail_count(uint64_t s, const SBArgs &A) {
 
 // sb_spec + sb_check fused: thread b runs the speculation of block b-1 (to get its exit X),
 // then block b from its own guess and, in lockstep, from X until the two states coincide.
+// Tiles of SB_THREADS blocks; CTA i takes tiles i, i + gridDim.x, ... (the grid is sized for the
+// capacity bound, the tile count comes from the true count on the device).
 __global__ void __launch_bounds__(SB_THREADS) sb_spec_check(SBArgs A) {
     if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
-    const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
-    if (b >= nb) return;
-    const uint64_t first = b * SB_B, last = min(n, first + SB_B);
-    uint64_t v[SB_B];
-    uint64_t X = 0;
-    int hX = 0;
-    if (b) {                                  // speculation of block b-1 (its guess, or exact for 0)
-        const uint64_t pf = first - SB_B;
+    for (uint64_t tile = blockIdx.x; tile * SB_THREADS < nb; tile += gridDim.x) {
+    const uint64_t b = tile * SB_THREADS + threadIdx.x;
+    uint64_t cnt = 0;
+    bool synced = true;
+    if (b < nb) {
+        const uint64_t first = b * SB_B, last = min(n, first + SB_B);
+        uint64_t v[SB_B];
+        uint64_t X = 0;
+        int hX = 0;
+        if (b) {                              // speculation of block b-1 (its guess, or exact for 0)
+            const uint64_t pf = first - SB_B;
 #pragma unroll
-        for (int j = 0; j < SB_B; ++j) v[j] = A.cand[pf + j];
-        X = (b - 1) ? A.cand[pf - 1] : A.aux->s;
+            for (int j = 0; j < SB_B; ++j) v[j] = A.cand[pf + j];
+            X = (b - 1) ? A.cand[pf - 1] : A.aux->s;
 #pragma unroll
-        for (int j = 0; j < SB_B; ++j) sb_step(X, v[j], A, hX, NoEmit{});
-    }
+            for (int j = 0; j < SB_B; ++j) sb_step(X, v[j], A, hX, NoEmit{});
+        }
 #pragma unroll
-    for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
-    uint64_t sg = b ? A.cand[first - 1] : A.aux->s;       // this block's guess
-    int hg = 0, ht = 0;
-    uint64_t cg = 0;
-    int64_t ct = 0, cg_sync = 0;
-    bool synced = (b == 0) || (X == sg && hX == 0);
-    uint64_t st = X;
+        for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
+        uint64_t sg = b ? A.cand[first - 1] : A.aux->s;       // this block's guess
+        int hg = 0, ht = 0;
+        uint64_t cg = 0;
+        int64_t ct = 0, cg_sync = 0;
+        synced = (b == 0) || (X == sg && hX == 0);
+        uint64_t st = X;
 #pragma unroll
-    for (int j = 0; j < SB_B; ++j) {
-        if (first + j < last) {
-            const uint64_t k = sb_step(sg, v[j], A, hg, NoEmit{});
-            cg += k;
-            if (!synced) {
-                ct += (int64_t)sb_step(st, v[j], A, ht, NoEmit{});
-                cg_sync += (int64_t)k;
-                synced = (st == sg) && (ht == hg);
+        for (int j = 0; j < SB_B; ++j) {
+            if (first + j < last) {
+                const uint64_t k = sb_step(sg, v[j], A, hg, NoEmit{});
+                cg += k;
+                if (!synced) {
+                    ct += (int64_t)sb_step(st, v[j], A, ht, NoEmit{});
+                    cg_sync += (int64_t)k;
+                    synced = (st == sg) && (ht == hg);
+                }
             }
         }
+        A.spec_exit[b] = sg;
+        A.spec_cnt[b] = cg;
+        A.ok[b] = synced ? 1u : 0u;
+        A.delta[b] = ct - cg_sync;
+        cnt = (uint64_t)((int64_t)cg + ct - cg_sync);
     }
-    A.spec_exit[b] = sg;
-    A.spec_cnt[b] = cg;
-    A.ok[b] = synced ? 1u : 0u;
-    A.delta[b] = ct - cg_sync;
+    // per-CTA sum of the counts (valid if every block synced) and AND of the sync flags
+    __shared__ uint64_t red[SB_THREADS / 32];
+    uint64_t x = cnt;
+    for (int d = 16; d; d >>= 1) x += __shfl_xor_sync(0xffffffffu, x, d);
+    const int all = __syncthreads_and(synced ? 1 : 0);
+    if ((threadIdx.x & 31) == 0) red[threadIdx.x >> 5] = x;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        uint64_t t = 0;
+        for (int w = 0; w < SB_THREADS / 32; ++w) t += red[w];
+        A.cta_sum[tile] = t;
+        A.cta_ok[tile] = all ? 1u : 0u;
+    }
+    __syncthreads();                          // red reused by the next tile
+    }
 }
 
 // One CTA: entries, offsets, totals and the streaming state.  Each thread owns a contiguous
@@ -125,13 +153,14 @@ __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
     const uint64_t n = sb_n(A);
     const uint32_t nb = (uint32_t)((n + SB_B - 1) / SB_B);
     const uint32_t tid = threadIdx.x;
-    const uint32_t per = (nb + blockDim.x - 1) / blockDim.x;
-    const uint32_t ba = min(nb, tid * per), bb = min(nb, ba + per);
+    const uint32_t nc = (nb + SB_THREADS - 1) / SB_THREADS;         // spec_check CTAs with blocks
+    const uint32_t per = (nc + blockDim.x - 1) / blockDim.x;
+    const uint32_t ca = min(nc, tid * per), cb = min(nc, ca + per);
     uint64_t sum = 0;
     uint32_t bad = 0;
-    for (uint32_t b = ba; b < bb; ++b) {
-        sum += (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]);
-        bad |= A.ok[b] ^ 1u;
+    for (uint32_t c = ca; c < cb; ++c) {
+        sum += A.cta_sum[c];
+        bad |= (uint32_t)(A.cta_ok[c] ^ 1u);
     }
     const int all_ok = __syncthreads_and(bad == 0);
     Aux *aux = A.aux;
@@ -152,10 +181,9 @@ __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
         }
         __syncthreads();
         uint64_t off = base0 + wsum[tid >> 5] + incl - sum;
-        for (uint32_t b = ba; b < bb; ++b) {
-            A.offs[b] = off;
-            A.entry[b] = b ? A.spec_exit[b - 1] : aux->s;
-            off += (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]);
+        for (uint32_t c = ca; c < cb; ++c) {        // sb_emit adds the in-CTA prefix
+            A.cta_off[c] = off;
+            off += A.cta_sum[c];
         }
         const uint64_t carry = wsum[32];
         if (tid == 0) {
@@ -165,11 +193,13 @@ __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
             if (!A.fin && n > 0 && A.cand[n - 1] == A.end && s_last == A.end) held_new = 1;
             const uint64_t mt = sb_tail_count(s_last, A);
             if (held_prev && aux->out_pos < A.dst_cap) A.dst[aux->out_pos] = aux->held_val;
+            A.entry[0] = aux->s;                  // block 0's entry (the others: spec exits)
             aux->out_pos = base0 + carry + mt;
             aux->s = s_last + mt * A.maxsz;
             aux->held = (uint64_t)held_new;
             aux->held_val = held_new ? A.end : 0;
             aux->total = carry + mt;
+            aux->sb_fast = 1;
             A.offs[nb] = base0 + carry;           // the tail's forced cuts start here
             A.entry[nb] = s_last;
         }
@@ -200,6 +230,7 @@ __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
         }
     }
     if (lane != 0) return;
+    aux->sb_fast = 0;
     const uint64_t mt = sb_tail_count(s, A);
     if (held_prev && aux->out_pos < A.dst_cap) A.dst[aux->out_pos] = aux->held_val;
     A.offs[nb] = off;
@@ -216,26 +247,48 @@ __global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
     if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
-    const uint64_t b = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x;
-    if (b > nb) return;
-    uint64_t s = A.entry[b];
-    uint64_t o = A.offs[b];
-    uint64_t *dst = A.dst;
-    const uint64_t cap = A.dst_cap;
-    auto emit = [&](uint64_t v) { if (o < cap) dst[o] = v; ++o; };
-    if (b == nb) {
-        const uint64_t mt = sb_tail_count(s, A);
-        for (uint64_t j = 1; j <= mt; ++j) emit(s + j * A.maxsz);
-        return;
+    const bool fast = A.aux->sb_fast != 0;
+    __shared__ uint64_t ws[SB_THREADS / 32 + 1];
+    for (uint64_t tile = blockIdx.x; tile * SB_THREADS <= nb; tile += gridDim.x) {
+        const uint64_t b = tile * SB_THREADS + threadIdx.x;
+        uint64_t s = 0, o = 0;
+        if (fast) {
+            // entry = the previous block's spec exit; offset = tile offset + in-tile exclusive prefix
+            const uint64_t v = b < nb ? (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]) : 0ull;
+            uint64_t incl = v;
+            for (int d = 1; d < 32; d <<= 1) {
+                uint64_t u = __shfl_up_sync(0xffffffffu, incl, d);
+                if ((threadIdx.x & 31) >= (uint32_t)d) incl += u;
+            }
+            if ((threadIdx.x & 31) == 31) ws[threadIdx.x >> 5] = incl;
+            __syncthreads();
+            uint64_t pre = 0;
+            for (uint32_t w = 0; w < (threadIdx.x >> 5); ++w) pre += ws[w];
+            __syncthreads();                  // ws reused by the next tile
+            if (b == nb) { s = A.entry[nb]; o = A.offs[nb]; }
+            else if (b < nb) { s = b ? A.spec_exit[b - 1] : A.entry[0]; o = A.cta_off[tile] + pre + incl - v; }
+        } else if (b <= nb) {
+            s = A.entry[b];
+            o = A.offs[b];
+        }
+        if (b > nb) continue;
+        uint64_t *dst = A.dst;
+        const uint64_t cap = A.dst_cap;
+        auto emit = [&](uint64_t v) { if (o < cap) dst[o] = v; ++o; };
+        if (b == nb) {
+            const uint64_t mt = sb_tail_count(s, A);
+            for (uint64_t j = 1; j <= mt; ++j) emit(s + j * A.maxsz);
+            continue;
+        }
+        const uint64_t first = b * SB_B, last = min(n, first + SB_B);
+        uint64_t v[SB_B];
+#pragma unroll
+        for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
+        int held = 0;
+#pragma unroll
+        for (int j = 0; j < SB_B; ++j)
+            if (first + j < last) sb_step(s, v[j], A, held, emit);
     }
-    const uint64_t first = b * SB_B, last = min(n, first + SB_B);
-    uint64_t v[SB_B];
-#pragma unroll
-    for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
-    int held = 0;
-#pragma unroll
-    for (int j = 0; j < SB_B; ++j)
-        if (first + j < last) sb_step(s, v[j], A, held, emit);
 }
 
 // ------------------------------------------------------------------------------ sb_dense
