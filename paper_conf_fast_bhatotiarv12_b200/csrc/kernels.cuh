@@ -40,7 +40,9 @@
 
 namespace shred {
 
-enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3, MODE_K32B = 4 };   // K32B: deg 16/24/32
+// K63: u64 state, deg 41..63; K40: u64 state, deg 33..40; K32: u32 state, deg 9..32;
+// K32B: u32 state, deg 16/24/32 (whole-byte top byte)
+enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3, MODE_K32B = 4, MODE_K40 = 5 };
 
 constexpr int STAGES      = 4;                 // TMA ring depth
 constexpr int BOX_ROWS    = 256;               // rows per TMA box (hardware max 256)
@@ -382,7 +384,7 @@ struct BulkCtx {
     uint32_t tab;       // shared address of the T|U image
     uint32_t laneT;     // K63: tab + (lane&15)*8           K32: tab + lane*4
     uint32_t laneU;     // K63: 128 + (lane&15)*8 (byte)     K32: 128 + lane*4 (byte)
-    uint32_t mhi;       // K63: 2^9 (f_hi >> 23 = mulhi(f_hi, 2^9))   K32: 2^8 (f >> 24)
+    uint32_t mhi;       // K63: 2^(72-k) (t = mulhi(f_hi, mhi))  K40: k-8 (funnel shift)  K32: 2^(40-k)
     uint32_t m256;      // 256 (row stride of the table image)
     uint32_t tmul;      // 2^(32-m): (f_lo * tmul) keeps the low m bits at the top
     uint32_t rsh;       // r << (32-m)
@@ -393,10 +395,11 @@ struct BulkCtx {
 //   t = f >> (k-8) = mulhi(fh, 2^(72-k));  f <- (f << 8 mod 2^64) ^ B ^ T[t] ^ U[o]
 //   T[t] = (t x^k mod P) ^ ((t << k) mod 2^64) cancels the byte the shift leaves at bits
 //   k..k+7 (k = 63: the one bit at 2^63), U[o] = o x^{8w} mod P.  Shift-in by two PRMTs.
-template <int K>
+// deg 33..40 (FUNNEL): the top byte straddles the two words, t = funnel(fl, fh) >> (k-8).
+template <int K, bool FUNNEL = false>
 __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, uint32_t pop,
                                        const BulkCtx &c) {
-    const uint32_t t  = __umulhi(fh, c.mhi);
+    const uint32_t t  = FUNNEL ? __funnelshift_rc(fl, fh, c.mhi) : __umulhi(fh, c.mhi);
     const uint32_t ti = t * c.m256 + c.laneT;
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
     const uint2 T = lds64(ti);
@@ -428,6 +431,13 @@ template <> struct State<MODE_K63> {
     uint32_t fl = 0, fh = 0;
     template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
         step63<K>(fl, fh, in, pop, c);
+    }
+    __device__ __forceinline__ uint32_t low() const { return fl; }
+};
+template <> struct State<MODE_K40> {
+    uint32_t fl = 0, fh = 0;
+    template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
+        step63<K, true>(fl, fh, in, pop, c);
     }
     __device__ __forceinline__ uint32_t low() const { return fl; }
 };
@@ -538,7 +548,37 @@ __device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d
     word4xN<MODE, CH, TEST, 3, LE>(st, in, po, m, c);
 }
 
-struct BulkConst { uint32_t mhi, m256, tmul, rsh, tsel; };
+struct BulkConst {
+    uint32_t mhi, m256, tmul, rsh, tsel;
+    uint32_t fu, fsel;  // FN windows (w % 16 != 0): e = 16*ceil(w/16) - w = 4*fu + v, fsel = PRMT
+                        // selector of bytes v..v+3 (0x3210 + 0x1111 v)
+};
+
+// The 16 bytes leaving the window at chunk q are bytes [16(q-A) + e, +16), A = WCH = ceil(w/16),
+// e = 16A - w: chunk q-A itself (w a multiple of 16), else a byte funnel of chunks q-A (lo) and
+// q-A+1 (hi) at the uniform offset e (one switch per chunk for every chain, 4 PRMTs per chain).
+template <bool FN, int CH>
+__device__ __forceinline__ void pops16(const uint4 (&lo)[CH], const uint4 (&hi)[CH], uint4 (&p)[CH],
+                                       const BulkConst &K) {
+    if (!FN) {
+#pragma unroll
+        for (int ch = 0; ch < CH; ++ch) p[ch] = lo[ch];
+        return;
+    }
+#define SHRED_FUN(a, b, c, d, e)                                                              \
+    for (int ch = 0; ch < CH; ++ch) {                                                        \
+        const uint32_t C[8] = {lo[ch].x, lo[ch].y, lo[ch].z, lo[ch].w, hi[ch].x, hi[ch].y, hi[ch].z, hi[ch].w}; \
+        p[ch] = make_uint4(__byte_perm(C[a], C[b], K.fsel), __byte_perm(C[b], C[c], K.fsel),  \
+                           __byte_perm(C[c], C[d], K.fsel), __byte_perm(C[d], C[e], K.fsel)); \
+    }
+    switch (K.fu) {
+        case 0: SHRED_FUN(0, 1, 2, 3, 4) break;
+        case 1: SHRED_FUN(1, 2, 3, 4, 5) break;
+        case 2: SHRED_FUN(2, 3, 4, 5, 6) break;
+        default: SHRED_FUN(3, 4, 5, 6, 7) break;
+    }
+#undef SHRED_FUN
+}
 
 // The hot kernel.  blockDim = NTC consumers + 1 producer warp; one CTA per SM.
 // blockIdx < nc: bulk CTA, rows blockIdx*ROWS + tid + ch*NTC (ch < CH); blockIdx == nc: the
@@ -548,7 +588,7 @@ struct BulkConst { uint32_t mhi, m256, tmul, rsh, tsel; };
 // w = 48 = 3 chunks of 16 B: the byte leaving the window at chunk q is the same byte slot of
 // chunk q-3, kept in a 4-slot register ring per chain (slot = chunk index mod 4).  WCH = w/16
 // (w in {16, 32, 48, 64}) generalises the pop distance; LE selects the "mod D <= r" marker set.
-template <int MODE, class C, int WCH, bool LE>
+template <int MODE, class C, int WCH, bool LE, bool FN = false>
 __global__ void __launch_bounds__(C::NTC + 32, 1)
 k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_img,
         const GenTables *__restrict__ gt, Job J, DevParams P, BulkConst K) {
@@ -636,7 +676,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     const int lane = tid & 31;
     BulkCtx c;
     c.tab = sbase;
-    if (MODE == MODE_K63) {
+    if (MODE == MODE_K63 || MODE == MODE_K40) {
         c.laneT = sbase + (uint32_t)(lane & 15) * 8u;
         c.laneU = 128u + (uint32_t)(lane & 15) * 8u;
     } else {
@@ -677,7 +717,14 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         for (int q = 0; q < 4; ++q) {
             uint4 d[CH], p[CH];
 #pragma unroll
-            for (int ch = 0; ch < CH; ++ch) { d[ch] = R[ch][q]; p[ch] = (q >= WCH) ? R[ch][q - WCH] : Z; }
+            uint4 lo[CH], hi[CH];
+#pragma unroll
+            for (int ch = 0; ch < CH; ++ch) {
+                d[ch] = R[ch][q];
+                lo[ch] = (q >= WCH) ? R[ch][q - WCH] : Z;
+                hi[ch] = (q + 1 >= WCH) ? R[ch][q + 1 - WCH] : Z;
+            }
+            pops16<FN, CH>(lo, hi, p, K);
             chunk16xN<MODE, CH, false, LE>(st, d, p, c, m);
         }
     }
@@ -706,7 +753,16 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                 uint4 d[CH], p[CH];
                 uint32_t m[CH];
 #pragma unroll
-                for (int ch = 0; ch < CH; ++ch) { d[ch] = D[ch][u]; p[ch] = R[ch][(cq + 4 - WCH) & 3]; }
+                for (int ch = 0; ch < CH; ++ch) { d[ch] = D[ch][u]; }
+                {
+                    uint4 lo[CH], hi[CH];
+#pragma unroll
+                    for (int ch = 0; ch < CH; ++ch) {
+                        lo[ch] = R[ch][(cq + 4 - WCH) & 3];
+                        hi[ch] = (WCH == 1) ? D[ch][u] : R[ch][(cq + 5 - WCH) & 3];
+                    }
+                    pops16<FN, CH>(lo, hi, p, K);
+                }
                 chunk16xN<MODE, CH, true, LE>(st, d, p, c, m);
 #pragma unroll
                 for (int ch = 0; ch < CH; ++ch) {

@@ -86,7 +86,17 @@ typedef void (*K1Fn)(const __grid_constant__ CUtensorMap, const uint4 *, const G
                      DevParams, BulkConst);
 
 template <int MODE, class C>
-K1Fn pick_mode(int wch, bool le) {
+K1Fn pick_mode(int wch, bool le, bool fn) {
+    if (fn) {                                // windows that are not a multiple of 16: '==' marker
+        if (le) return nullptr;
+        switch (wch) {
+            case 1: return k1_bulk<MODE, C, 1, false, true>;
+            case 2: return k1_bulk<MODE, C, 2, false, true>;
+            case 3: return k1_bulk<MODE, C, 3, false, true>;
+            case 4: return k1_bulk<MODE, C, 4, false, true>;
+            default: return nullptr;
+        }
+    }
     switch (wch * 2 + (le ? 1 : 0)) {
         case 2: return k1_bulk<MODE, C, 1, false>;
         case 3: return k1_bulk<MODE, C, 1, true>;
@@ -99,19 +109,20 @@ K1Fn pick_mode(int wch, bool le) {
         default: return nullptr;
     }
 }
-// The hot-kernel instance for (u64 state | u32 state with a whole-byte top byte | u32 state,
-// w/16, marker set).
+// The hot-kernel instance for (u64 state: deg 41..63 | deg 33..40; u32 state with a whole-byte
+// top byte | u32 state; ceil(w/16), marker set, w % 16 != 0).
 #ifndef SHRED_BYTEIDX
 #define SHRED_BYTEIDX 1   // deg 16/24/32: PRMT table index (MODE_K32B); 0: IMAD index (MODE_K32)
 #endif
-K1Fn pick_k1(bool k63, bool byteidx, int wch, bool le) {
-    if (k63) return pick_mode<MODE_K63, CfgK63>(wch, le);
-    return byteidx ? pick_mode<MODE_K32B, CfgK32>(wch, le) : pick_mode<MODE_K32, CfgK32>(wch, le);
+K1Fn pick_k1(int k, bool byteidx, int wch, bool le, bool fn) {
+    if (k >= 41) return pick_mode<MODE_K63, CfgK63>(wch, le, fn);
+    if (k >= 33) return pick_mode<MODE_K40, CfgK63>(wch, le, fn);
+    return byteidx ? pick_mode<MODE_K32B, CfgK32>(wch, le, fn) : pick_mode<MODE_K32, CfgK32>(wch, le, fn);
 }
 // The small-input shape (CfgSmall) exists for the paper's window with the equality marker.
-K1Fn pick_k1_small(bool k63, bool byteidx, int wch, bool le) {
-    if (wch != 3 || le) return nullptr;
-    if (k63) return k1_bulk<MODE_K63, CfgSmall, 3, false>;
+K1Fn pick_k1_small(int k, bool byteidx, int wch, bool le, bool fn) {
+    if (wch != 3 || le || fn || (k >= 33 && k <= 40)) return nullptr;
+    if (k >= 41) return k1_bulk<MODE_K63, CfgSmall, 3, false>;
     return byteidx ? k1_bulk<MODE_K32B, CfgSmall, 3, false> : k1_bulk<MODE_K32, CfgSmall, 3, false>;
 }
 
@@ -357,7 +368,11 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         const int m = 32 - (int)__builtin_ctzll(ctx->p.divisor);     // D = 2^(32-m')
         BulkConst K;
         // top byte t = f >> (k-8): u64 state mulhi(f_hi, 2^(72-k)); u32 state mulhi(f, 2^(40-k))
-        K.mhi = ctx->path == SHRED_PATH_K63 ? (1u << (72 - ctx->k)) : (1u << (40 - ctx->k));
+        K.mhi = ctx->path == SHRED_PATH_K63 ? (ctx->k >= 41 ? (1u << (72 - ctx->k)) : (uint32_t)(ctx->k - 8))
+                                            : (1u << (40 - ctx->k));
+        const uint32_t e = (uint32_t)(16 * ((ctx->p.window + 15) / 16) - ctx->p.window);
+        K.fu = e / 4;
+        K.fsel = 0x3210u + 0x1111u * (e % 4);
         K.m256 = 256u;
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
@@ -551,10 +566,13 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     ctx->dp.pow2 = (p->divisor & (p->divisor - 1)) == 0 ? 1u : 0u;
     ctx->dp.marker = p->marker;
     const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
-    const bool fast_w = p->window == 16 || p->window == 32 || p->window == 48 || p->window == 64;
+    // the hot kernel: any w <= 64 (w % 16 != 0 with the '==' marker: funnel-shifted pops)
+    const bool fast_w = p->window >= 1 && p->window <= 64 &&
+                        (p->window % 16 == 0 || p->marker == SHRED_MARKER_EQ);
     const bool fast = fast_w && pow2 && p->divisor <= (1ull << 32);
-    // u64-state kernel: deg 41..63 (t = mulhi(f_hi, 2^(72-k))); u32-state kernel: deg 9..32
-    if (k >= 41 && k <= 63 && fast) ctx->path = SHRED_PATH_K63;
+    // u64-state kernel: deg 33..63 (t = mulhi(f_hi, 2^(72-k)), or a funnel shift for k <= 40);
+    // u32-state kernel: deg 9..32
+    if (k >= 33 && k <= 63 && fast) ctx->path = SHRED_PATH_K63;
     else if (k >= 9 && k <= 32 && fast) ctx->path = SHRED_PATH_K32;
     else ctx->path = SHRED_PATH_GENERIC;
     if (major != 10) ctx->path = SHRED_PATH_GENERIC;   // the TMA kernels are built for sm_100a only
@@ -610,15 +628,15 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
             return bail(SHRED_ECUDA);
         ctx->encode = (EncodeTiledFn)fn;
         const bool byteidx = SHRED_BYTEIDX && ctx->path == SHRED_PATH_K32 && (k == 16 || k == 24 || k == 32);
-        ctx->k1_fn = pick_k1(ctx->path == SHRED_PATH_K63, byteidx, (int)(p->window / 16),
-                             p->marker == SHRED_MARKER_LE);
+        const int wch = (int)((p->window + 15) / 16);
+        const bool funnel = p->window % 16 != 0;
+        ctx->k1_fn = pick_k1(k, byteidx, wch, p->marker == SHRED_MARKER_LE, funnel);
         if (!ctx->k1_fn ||
             cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM) != cudaSuccess)
             return bail(SHRED_ECUDA);
 #ifndef SHRED_NO_SMALL
-        ctx->k1_small_fn = pick_k1_small(ctx->path == SHRED_PATH_K63, byteidx, (int)(p->window / 16),
-                                         p->marker == SHRED_MARKER_LE);
+        ctx->k1_small_fn = pick_k1_small(k, byteidx, wch, p->marker == SHRED_MARKER_LE, funnel);
 #endif
         if (ctx->k1_small_fn &&
             cudaFuncSetAttribute(ctx->k1_small_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,

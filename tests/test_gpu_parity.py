@@ -115,8 +115,8 @@ def test_launch_shapes_around_small_threshold(pkg, poly, n):
 
 
 def test_generic_path_variants(pkg):
-    for p in (pkg.Params(window=33), pkg.Params(window=1, divisor=256, magic=7),
-              pkg.Params(poly=(1 << 63) | 3, window=24, divisor=1024),
+    for p in (pkg.Params(window=65), pkg.Params(window=1, divisor=256, magic=7, marker=1),
+              pkg.Params(poly=(1 << 63) | 3, window=24, divisor=1024, marker=1),
               pkg.Params(poly=0x11D, window=7, divisor=64, magic=9),
               pkg.Params(divisor=1 << 40, magic=12345)):
         ch = pkg.Chunker(p)
@@ -308,6 +308,22 @@ def test_fast_path_windows_and_le_marker(pkg, poly, path, window, marker):
     check_chunk(ch, synthgen.random_bytes(window + marker, (3 << 20) + 31), offset=5)
 
 
+@pytest.mark.parametrize("poly", [LBFS, 0x104C11DB7, 0x20000005, None])   # K63, K32B, K32, K40
+@pytest.mark.parametrize("window", [1, 2, 7, 15, 17, 31, 33, 47, 49, 63])
+def test_fast_path_any_window(pkg, poly, window):
+    """Windows that are not a multiple of 16 on the hot kernel: the bytes leaving the window are a
+    funnel (PRMT) of two staged 16-byte chunks at offset e = 16 ceil(w/16) - w; every state mode."""
+    if poly is None:
+        poly = _dense_irreducible(37, 37)
+    p = pkg.Params(poly=poly, window=window, divisor=512, magic=window % 512)
+    ch = pkg.Chunker(p)
+    assert ch.path in ("k63", "k32")
+    data = synthgen.random_bytes(100 + window, (2 << 20) + 4 * window + 1)
+    check_chunk(ch, data, offset=window % 16)
+    # the '<=' marker set with such windows runs on the generic path
+    assert pkg.Chunker(pkg.Params(poly=poly, window=window, divisor=512, magic=3, marker=1)).path == "generic"
+
+
 def _dense_irreducible(deg, seed):
     rng = np.random.default_rng(seed)
     while True:
@@ -319,11 +335,12 @@ def _dense_irreducible(deg, seed):
 
 @pytest.mark.parametrize("deg", [8, 9, 12, 16, 24, 31, 32, 33, 40, 41, 48, 57, 62, 63])
 def test_polynomial_degrees(pkg, deg):
-    """Any degree: u32-state fast kernel for 9..32, u64-state for 41..63, generic otherwise
-    (T tables with the (t << k) cancel term); dense random irreducible P, bit-exact."""
+    """Any degree: u32-state fast kernel for 9..32, u64-state for 33..63 (top byte by mulhi for
+    41..63, by a funnel shift for 33..40), generic for 8 (T tables with the (t << k) cancel term);
+    dense random irreducible P, bit-exact."""
     P = _dense_irreducible(deg, deg)
     D = 1 << min(10, deg - 1)
     p = pkg.Params(poly=P, divisor=D, magic=D // 3)
     ch = pkg.Chunker(p)
-    assert ch.path == ("k32" if 9 <= deg <= 32 else "k63" if deg >= 41 else "generic")
+    assert ch.path == ("k32" if 9 <= deg <= 32 else "k63" if deg >= 33 else "generic")
     check_chunk(ch, synthgen.random_bytes(deg, (2 << 20) + 123), offset=deg % 16)
