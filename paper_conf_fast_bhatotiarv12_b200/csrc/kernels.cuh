@@ -9,7 +9,7 @@
 // realised with two 256-entry tables: T (reduces the byte shifted out of the top of the
 // state) and U (removes the byte leaving the window).  See DESIGN.md "Kernels".
 //
-//   k1_bulk<MODE,C,WCH,LE>  TMA-staged hot loop.  The input is viewed as a 2-D [rows][S]
+//   k1_bulk<MODE,C,WCH,LE,FN>  TMA-staged hot loop (FN: w not a multiple of 16, funnel pops).  The input is viewed as a 2-D [rows][S]
 //                   tensor; each consumer thread rolls CH = 2 rows (independent chains) in one
 //                   basic block; rounds of 32 B per row arrive in a 4-stage shared-memory ring
 //                   (SWIZZLE_32B, conflict-free LDS.128) fed by a producer warp.  T/U live in
