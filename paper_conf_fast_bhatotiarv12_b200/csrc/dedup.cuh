@@ -26,6 +26,7 @@ struct DedupTable {
 __global__ void k_dedup_insert(DedupTable T, const uint8_t *__restrict__ digests, const uint64_t *cuts,
                                const uint64_t *n_cuts, uint64_t len, uint64_t max_chunks,
                                uint8_t *new_flags) {
+    pdl_entry();
     const uint64_t ncut = *n_cuts;
     const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nc; i += (uint64_t)gridDim.x * blockDim.x) {

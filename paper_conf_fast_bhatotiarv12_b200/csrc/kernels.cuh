@@ -155,6 +155,14 @@ struct Aux {
     uint64_t sb_fast;           // sb_plan: 1 = every block synced (two-level scan offsets)
 };
 
+// Programmatic dependent launch (shred.cu pdl_launch): wait until the previous kernel of the
+// stream has completed and its writes are visible, then let the next kernel start launching.
+// Both are no-ops for a kernel launched without the attribute.
+__device__ __forceinline__ void pdl_entry() {
+    asm volatile("griddepcontrol.wait;" ::: "memory");
+    asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+}
+
 // ------------------------------------------------------------------------------ PTX helpers
 __device__ __forceinline__ uint32_t smem_u32(const void *p) {
     return static_cast<uint32_t>(__cvta_generic_to_shared(p));
@@ -363,6 +371,7 @@ __device__ __forceinline__ uint32_t roll_slot(const Job &J, const DevParams &P, 
 // Generic-only path: one thread per slot, one group per block of GEN_THREADS slots.
 __global__ void __launch_bounds__(GEN_THREADS)
 k1_generic(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots) {
+    pdl_entry();
     __shared__ uint64_t sT[256], sU[256];
     __shared__ uint32_t ws[33];
     for (int i = threadIdx.x; i < 256; i += blockDim.x) { sT[i] = gt->T[i]; sU[i] = gt->U[i]; }
@@ -592,6 +601,7 @@ template <int MODE, class C, int WCH, bool LE, bool FN = false>
 __global__ void __launch_bounds__(C::NTC + 32, 1)
 k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_img,
         const GenTables *__restrict__ gt, Job J, DevParams P, BulkConst K) {
+    pdl_entry();
     constexpr int CH = C::CH, NTC = C::NTC, ROUND = C::ROUND, CPR = C::CPR;
     extern __shared__ uint8_t smem_raw[];
     // align the dynamic shared base to 1 KiB (the TMA swizzle pattern is address-based)
@@ -791,6 +801,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
 // ------------------------------------------------------------------------------ k_total
 // Sum of the group sums -> aux->total (bounded path: needed on the host before k_scatter).
 __global__ void k_total(const uint64_t *__restrict__ group_sum, uint32_t ngroups, Aux *aux) {
+    pdl_entry();
     uint64_t s = 0;
     for (uint32_t g = threadIdx.x; g < ngroups; g += blockDim.x) s += group_sum[g];
     for (int d = 16; d; d >>= 1) s += __shfl_xor_sync(0xffffffffu, s, d);
@@ -815,6 +826,7 @@ __global__ void __launch_bounds__(SCATTER_THREADS)
 k_scatter(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots,
           uint64_t *__restrict__ dst, uint64_t dst_cap, Aux *aux, int streaming,
           uint64_t *n_direct) {
+    pdl_entry();
     __shared__ uint64_t gbase[MAX_GROUPS];
     __shared__ uint64_t wsum[SCATTER_THREADS / 32 + 1];
     const uint32_t ng = J.map.ngroups;
@@ -876,6 +888,7 @@ k_scatter(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots,
 // After an unbounded piece ending at `end`: emit the previously held cut at out_pos, hold the
 // piece's last candidate if it sits exactly at the stream end, advance out_pos.
 __global__ void k_piece_done(Aux *aux, uint64_t *dst, uint64_t dst_cap, uint64_t end) {
+    pdl_entry();
     if (threadIdx.x != 0 || blockIdx.x != 0) return;
     const uint64_t held = aux->held;
     if (held && aux->out_pos < dst_cap) dst[aux->out_pos] = aux->held_val;
@@ -886,9 +899,13 @@ __global__ void k_piece_done(Aux *aux, uint64_t *dst, uint64_t dst_cap, uint64_t
     aux->held_val = hold_new ? end : 0;
 }
 
-__global__ void k_call_begin(Aux *aux) { aux->out_pos = 0; }
+__global__ void k_call_begin(Aux *aux) {
+    pdl_entry();
+    aux->out_pos = 0;
+}
 
 __global__ void k_call_end(Aux *aux, uint64_t *n_out, uint64_t cap, volatile uint64_t *sticky_flag) {
+    pdl_entry();
     *n_out = aux->out_pos;
     if (aux->out_pos > cap) {
         aux->overflow = 1;
@@ -897,18 +914,24 @@ __global__ void k_call_end(Aux *aux, uint64_t *n_out, uint64_t cap, volatile uin
 }
 
 __global__ void k_stream_reset(Aux *aux) {
+    pdl_entry();
     aux->total = 0; aux->last_cand = 0; aux->out_pos = 0;
     aux->s = 0; aux->held = 0; aux->held_val = 0; aux->dense = 0;
 }
 
-__global__ void k_write_u64(uint64_t *p, uint64_t v) { *p = v; }
+__global__ void k_write_u64(uint64_t *p, uint64_t v) {
+    pdl_entry();
+    *p = v;
+}
 
 // Entry / exit of shred_size_bound_state.
 __global__ void k_state_in(Aux *aux, uint64_t s, uint64_t held) {
+    pdl_entry();
     aux->total = 0; aux->last_cand = 0; aux->out_pos = 0; aux->dense = 0;
     aux->s = s; aux->held = held; aux->held_val = held ? s : 0;
 }
 __global__ void k_state_out(const Aux *aux, uint64_t *state, uint64_t *n_out, uint64_t cap) {
+    pdl_entry();
     state[0] = aux->s; state[1] = aux->held;
     *n_out = aux->out_pos;
 }
@@ -916,6 +939,7 @@ __global__ void k_state_out(const Aux *aux, uint64_t *state, uint64_t *n_out, ui
 // New carry = the last min(keep, old_len + len) bytes of (old carry || src[0..len)).
 __global__ void k_carry(const uint8_t *old_c, uint32_t old_len, const uint8_t *src, uint64_t len,
                         uint8_t *new_c, uint32_t keep) {
+    pdl_entry();
     const uint64_t tot = (uint64_t)old_len + len;
     const uint32_t nl = (uint32_t)(tot < keep ? tot : keep);
     for (uint32_t j = threadIdx.x; j < nl; j += blockDim.x) {
@@ -934,6 +958,7 @@ __device__ __forceinline__ uint64_t splitmix_word(uint64_t seed, uint64_t k) {
     return z ^ (z >> 31);
 }
 __global__ void k_synth_fill(uint8_t *dst, uint64_t len, uint64_t seed, uint64_t offset) {
+    pdl_entry();
     // byte j of dst = byte (offset + j) of the stream; each thread writes 16 bytes
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x * 16ull;
     for (uint64_t j0 = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) * 16ull; j0 < len; j0 += stride) {

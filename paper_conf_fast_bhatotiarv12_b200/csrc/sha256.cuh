@@ -117,6 +117,7 @@ __device__ __forceinline__ void chunk_bounds(const uint64_t *cuts, uint64_t ncut
 
 __global__ void k_hash_hist(const uint64_t *__restrict__ cuts, const uint64_t *n_cuts, uint64_t len,
                             uint64_t max_chunks, uint32_t *hist) {
+    pdl_entry();
     const uint64_t ncut = *n_cuts;
     const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nc; i += (uint64_t)gridDim.x * blockDim.x) {
@@ -128,6 +129,7 @@ __global__ void k_hash_hist(const uint64_t *__restrict__ cuts, const uint64_t *n
 
 // One CTA: exclusive scan of the HB bucket counts (in place) and reset of the work queue.
 __global__ void __launch_bounds__(HB) k_hash_scan(uint32_t *hist, unsigned long long *queue) {
+    pdl_entry();
     __shared__ uint32_t ws[33];
     const uint32_t v = hist[threadIdx.x];
     uint32_t tot;
@@ -138,6 +140,7 @@ __global__ void __launch_bounds__(HB) k_hash_scan(uint32_t *hist, unsigned long 
 
 __global__ void k_hash_scatter(const uint64_t *__restrict__ cuts, const uint64_t *n_cuts, uint64_t len,
                                uint64_t max_chunks, uint32_t *offs, uint32_t *order) {
+    pdl_entry();
     const uint64_t ncut = *n_cuts;
     const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nc; i += (uint64_t)gridDim.x * blockDim.x) {
@@ -164,6 +167,7 @@ __global__ void __launch_bounds__(256)
 k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__restrict__ cuts,
               const uint64_t *n_cuts, uint64_t max_chunks, uint8_t *__restrict__ digests,
               const uint32_t *__restrict__ order, unsigned long long *queue) {
+    pdl_entry();
     const uint64_t ncut = *n_cuts;
     const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
     const int lane = threadIdx.x & 31;

@@ -111,6 +111,9 @@ K1Fn pick_mode(int wch, bool le, bool fn) {
 }
 // The hot-kernel instance for (u64 state: deg 41..63 | deg 33..40; u32 state with a whole-byte
 // top byte | u32 state; ceil(w/16), marker set, w % 16 != 0).
+#ifndef SHRED_PDL
+#define SHRED_PDL 1       // 0: plain stream serialization (A/B)
+#endif
 #ifndef SHRED_BYTEIDX
 #define SHRED_BYTEIDX 1   // deg 16/24/32: PRMT table index (MODE_K32B); 0: IMAD index (MODE_K32)
 #endif
@@ -203,6 +206,23 @@ int cuda_fail(shred_ctx *c, cudaError_t e, const char *what) {
 }
 #define CK(call, what) do { cudaError_t _e = (call); if (_e != cudaSuccess) return cuda_fail(ctx, _e, what); } while (0)
 #define LAUNCHED(what) do { ++ctx->launches; cudaError_t _e = cudaGetLastError(); if (_e != cudaSuccess) return cuda_fail(ctx, _e, what); } while (0)
+
+// Programmatic dependent launch: every kernel of a call's chain is launched with programmatic
+// stream serialization, and each starts with griddepcontrol.wait + launch_dependents
+// (kernels.cuh pdl_entry), so a kernel's launch overlaps the tail of its predecessor instead of
+// paying the full launch gap (small inputs are launch-latency-bound).
+template <typename... KArgs, typename... Args>
+cudaError_t pdl_launch(void (*k)(KArgs...), dim3 g, dim3 b, size_t smem, cudaStream_t st, Args... args) {
+    cudaLaunchConfig_t cfg{};
+    cfg.gridDim = g; cfg.blockDim = b; cfg.dynamicSmemBytes = smem; cfg.stream = st;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[0].val.programmaticStreamSerializationAllowed = SHRED_PDL;
+    cfg.attrs = at; cfg.numAttrs = 1;
+    return cudaLaunchKernelEx(&cfg, k, static_cast<KArgs>(args)...);
+}
+#define PDL(k, g, b, smem, st, ...) do { cudaError_t _pe = pdl_launch(k, g, b, smem, st, __VA_ARGS__); \
+    if (_pe != cudaSuccess) return cuda_fail(ctx, _pe, #k); } while (0)
 
 template <class T>
 int grow(shred_ctx *ctx, T *&ptr, uint64_t &cap, uint64_t need, const char *what) {
@@ -381,11 +401,11 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         int threads = (ctx->path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC) + 32;
         K1Fn fn = ctx->k1_fn;
         if (pl.small) { smem = CfgSmall::SMEM; threads = CfgSmall::NTC + 32; fn = ctx->k1_small_fn; }
-        fn<<<pl.bulk_ctas, threads, smem, st>>>(pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
+        PDL(fn, pl.bulk_ctas, threads, smem, st, pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
         LAUNCHED("k1_bulk");
         if (e1) CK(cudaEventRecord(e1, st), "profile record");
     } else {
-        k1_generic<<<(pl.nslots + GEN_THREADS - 1) / GEN_THREADS, GEN_THREADS, 0, st>>>(pl.J, ctx->dp, ctx->d_gen,
+        PDL(k1_generic, (pl.nslots + GEN_THREADS - 1) / GEN_THREADS, GEN_THREADS, 0, st, pl.J, ctx->dp, ctx->d_gen,
                                                                                        pl.nslots);
         LAUNCHED("k1_generic");
     }
@@ -396,12 +416,12 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
 int launch_scatter(shred_ctx *ctx, Plan &pl, uint64_t *dst, uint64_t dst_cap, Aux *aux, int streaming,
                    uint64_t *n_direct, cudaStream_t st) {
     if (pl.nslots == 0) {
-        k_write_u64<<<1, 1, 0, st>>>(&aux->total, 0);
+        PDL(k_write_u64, 1, 1, 0, st, &aux->total, 0);
         LAUNCHED("k_write_u64");
-        if (n_direct) { k_write_u64<<<1, 1, 0, st>>>(n_direct, 0); LAUNCHED("k_write_u64"); }
+        if (n_direct) { PDL(k_write_u64, 1, 1, 0, st, n_direct, 0); LAUNCHED("k_write_u64"); }
         return SHRED_OK;
     }
-    k_scatter<<<(pl.nslots + SCATTER_THREADS - 1) / SCATTER_THREADS, SCATTER_THREADS, 0, st>>>(
+    PDL(k_scatter, (pl.nslots + SCATTER_THREADS - 1) / SCATTER_THREADS, SCATTER_THREADS, 0, st, 
         pl.J, ctx->dp, ctx->d_gen, pl.nslots, dst, dst_cap, aux, streaming, n_direct);
     LAUNCHED("k_scatter");
     return SHRED_OK;
@@ -432,14 +452,14 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
     uint64_t g = (nb + SB_THREADS - 1) / SB_THREADS;
     if (g > gmax) g = gmax;
     if (nb) {
-        sb_spec_check<<<(unsigned)g, SB_THREADS, 0, st>>>(A);
+        PDL(sb_spec_check, (unsigned)g, SB_THREADS, 0, st, A);
         LAUNCHED("sb_spec_check");
     }
-    sb_plan<<<1, 1024, 0, st>>>(A);
+    PDL(sb_plan, 1, 1024, 0, st, A);
     LAUNCHED("sb_plan");
     uint64_t ge = (nb + 1 + SB_THREADS - 1) / SB_THREADS;
     if (ge > gmax) ge = gmax;
-    sb_emit<<<(unsigned)ge, SB_THREADS, 0, st>>>(A);
+    PDL(sb_emit, (unsigned)ge, SB_THREADS, 0, st, A);
     LAUNCHED("sb_emit");
     if (pl && pl->nslots) {
         uint64_t maxseg = pl->J.map.S;
@@ -447,7 +467,7 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
         if (pl->J.map.tail_seg > maxseg) maxseg = pl->J.map.tail_seg;
         if (maxseg > SBD_WIN) maxseg = SBD_WIN;
         const size_t smem = (size_t)((maxseg + 31) / 32) * 4;
-        sb_dense<<<1, SBD_THREADS, smem, st>>>(pl->J, ctx->dp, ctx->d_gen, pl->nslots, A);
+        PDL(sb_dense, 1, SBD_THREADS, smem, st, pl->J, ctx->dp, ctx->d_gen, pl->nslots, A);
         LAUNCHED("sb_dense");
     }
     return SHRED_OK;
@@ -466,9 +486,9 @@ int run_piece(shred_ctx *ctx, Aux *aux, const uint8_t *src, uint64_t p_begin, co
         if ((rc = launch_scatter(ctx, pl, dst, dst_cap, aux, 1, nullptr, st))) return rc;
         if (final_) {
             // one-shot: nothing held; out_pos += total
-            k_piece_done<<<1, 1, 0, st>>>(aux, dst, dst_cap, ~0ull);
+            PDL(k_piece_done, 1, 1, 0, st, aux, dst, dst_cap, ~0ull);
         } else {
-            k_piece_done<<<1, 1, 0, st>>>(aux, dst, dst_cap, t_end);
+            PDL(k_piece_done, 1, 1, 0, st, aux, dst, dst_cap, t_end);
         }
         LAUNCHED("k_piece_done");
         return SHRED_OK;
@@ -688,10 +708,10 @@ int shred_chunk(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, uint64_t *d_o
         if ((rc = launch_detect(ctx, pl, st))) return rc;
         return launch_scatter(ctx, pl, d_out, cap, aux, 0, n_out, st);
     }
-    k_stream_reset<<<1, 1, 0, st>>>(aux);
+    PDL(k_stream_reset, 1, 1, 0, st, aux);
     LAUNCHED("k_stream_reset");
     if ((rc = run_piece(ctx, aux, d_in, 0, nullptr, 0, 0, len, len, 1, d_out, cap, st))) return rc;
-    k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, nullptr);
+    PDL(k_call_end, 1, 1, 0, st, aux, n_out, cap, nullptr);
     LAUNCHED("k_call_end");
     return SHRED_OK;
 }
@@ -724,11 +744,11 @@ int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, ui
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
     Aux *aux = ctx->d_aux + 0;
-    k_stream_reset<<<1, 1, 0, st>>>(aux);
+    PDL(k_stream_reset, 1, 1, 0, st, aux);
     LAUNCHED("k_stream_reset");
     if ((rc = launch_size_bound(ctx, d_cand, nullptr, n_cand, n_cand, total_len, 1, d_out, cap, aux,
                                 nullptr, st))) return rc;
-    k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, nullptr);
+    PDL(k_call_end, 1, 1, 0, st, aux, n_out, cap, nullptr);
     LAUNCHED("k_call_end");
     return SHRED_OK;
 }
@@ -744,11 +764,11 @@ int shred_size_bound_state(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_ca
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
     Aux *aux = ctx->d_aux + 0;
-    k_state_in<<<1, 1, 0, st>>>(aux, state_in[0], state_in[1] ? 1ull : 0ull);
+    PDL(k_state_in, 1, 1, 0, st, aux, state_in[0], state_in[1] ? 1ull : 0ull);
     LAUNCHED("k_state_in");
     if ((rc = launch_size_bound(ctx, d_cand, nullptr, n_cand, n_cand, end, fin ? 1 : 0, d_out, cap, aux,
                                 nullptr, st))) return rc;
-    k_state_out<<<1, 1, 0, st>>>(aux, d_state_out, n_out, cap);
+    PDL(k_state_out, 1, 1, 0, st, aux, d_state_out, n_out, cap);
     LAUNCHED("k_state_out");
     return SHRED_OK;
 }
@@ -794,7 +814,7 @@ int feed_device_piece(shred_ctx *ctx, const uint8_t *src, uint64_t len, uint64_t
     if (rc) return rc;
     const uint32_t keep = ctx->p.window - 1u;
     uint8_t *nc = ctx->d_carry[ctx->carry_idx ^ 1];
-    k_carry<<<1, 256, 0, st>>>(prefix, ctx->carry_len, src, len, nc, keep);
+    PDL(k_carry, 1, 256, 0, st, prefix, ctx->carry_len, src, len, nc, keep);
     LAUNCHED("k_carry");
     ctx->carry_idx ^= 1;
     const uint64_t tot = (uint64_t)ctx->carry_len + len;
@@ -815,7 +835,7 @@ int shred_feed(shred_ctx *ctx, const void *in, uint64_t len, uint64_t *d_out, ui
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
     Aux *aux = ctx->d_aux + 1;
-    k_call_begin<<<1, 1, 0, st>>>(aux);
+    PDL(k_call_begin, 1, 1, 0, st, aux);
     LAUNCHED("k_call_begin");
     if (len) {
         if (!in) return fail(ctx, SHRED_EINVAL, "in is NULL");
@@ -860,7 +880,7 @@ int shred_feed(shred_ctx *ctx, const void *in, uint64_t len, uint64_t *d_out, ui
             ctx->ring_next = slot_of(npieces);
         }
     }
-    k_call_end<<<1, 1, 0, st>>>(aux, n_out, cap, ctx->d_flag);
+    PDL(k_call_end, 1, 1, 0, st, aux, n_out, cap, ctx->d_flag);
     LAUNCHED("k_call_end");
     return SHRED_OK;
 }
@@ -873,9 +893,9 @@ int shred_flush(shred_ctx *ctx, uint64_t *d_out, uint64_t cap, uint64_t *n_out, 
     cudaStream_t st = (cudaStream_t)stream;
     // Every forced cut strictly inside the stream was emitted by the last feed; a cut held at
     // exactly the stream end is dropped (c = N is never a cut, reading Q11).
-    k_stream_reset<<<1, 1, 0, st>>>(ctx->d_aux + 1);
+    PDL(k_stream_reset, 1, 1, 0, st, ctx->d_aux + 1);
     LAUNCHED("k_stream_reset");
-    k_write_u64<<<1, 1, 0, st>>>(n_out, 0);
+    PDL(k_write_u64, 1, 1, 0, st, n_out, 0);
     LAUNCHED("k_write_u64");
     ctx->pos = 0; ctx->carry_len = 0; ctx->carry_idx = 0;
     return SHRED_OK;
@@ -908,13 +928,13 @@ int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const u
     if (max_chunks > 0xFFFFFFFFull) return fail(ctx, SHRED_EINVAL, "max_chunks must be < 2^32");
     CK(cudaMemsetAsync(ctx->d_hhist, 0, HB * sizeof(uint32_t), st), "hash hist reset");
     const unsigned gs = (unsigned)(ctx->sm_count * 8);
-    k_hash_hist<<<gs, 256, 0, st>>>(d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist);
+    PDL(k_hash_hist, gs, 256, 0, st, d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist);
     LAUNCHED("k_hash_hist");
-    k_hash_scan<<<1, HB, 0, st>>>(ctx->d_hhist, ctx->d_queue);
+    PDL(k_hash_scan, 1, HB, 0, st, ctx->d_hhist, ctx->d_queue);
     LAUNCHED("k_hash_scan");
-    k_hash_scatter<<<gs, 256, 0, st>>>(d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist, ctx->d_order);
+    PDL(k_hash_scatter, gs, 256, 0, st, d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist, ctx->d_order);
     LAUNCHED("k_hash_scatter");
-    k_hash_chunks<<<ctx->sm_count * SHRED_HASH_CTAS_PER_SM, SHRED_HASH_THREADS, 0, st>>>(d_in, len, d_cuts, d_ncuts, max_chunks, d_digests,
+    PDL(k_hash_chunks, ctx->sm_count * SHRED_HASH_CTAS_PER_SM, SHRED_HASH_THREADS, 0, st, d_in, len, d_cuts, d_ncuts, max_chunks, d_digests,
                                                       ctx->d_order, ctx->d_queue);
     LAUNCHED("k_hash_chunks");
     return SHRED_OK;
@@ -954,7 +974,7 @@ int shred_index_insert(shred_ctx *ctx, const uint8_t *d_digests, const uint64_t 
     if (!len || !max_chunks) return SHRED_OK;
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
-    k_dedup_insert<<<ctx->sm_count * 8, 256, 0, st>>>(ctx->index, d_digests, d_cuts, d_ncuts, len, max_chunks,
+    PDL(k_dedup_insert, ctx->sm_count * 8, 256, 0, st, ctx->index, d_digests, d_cuts, d_ncuts, len, max_chunks,
                                                       d_new_flags);
     LAUNCHED("k_dedup_insert");
     return SHRED_OK;

@@ -81,6 +81,7 @@ __device__ __forceinline__ uint64_t sb_tail_count(uint64_t s, const SBArgs &A) {
 // Tiles of SB_THREADS blocks; CTA i takes tiles i, i + gridDim.x, ... (the grid is sized for the
 // capacity bound, the tile count comes from the true count on the device).
 __global__ void __launch_bounds__(SB_THREADS) sb_spec_check(SBArgs A) {
+    pdl_entry();
     if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
@@ -147,6 +148,7 @@ __global__ void __launch_bounds__(SB_THREADS) sb_spec_check(SBArgs A) {
 // One CTA: entries, offsets, totals and the streaming state.  Each thread owns a contiguous
 // range of blocks; one block scan of the range sums gives every block's offset.
 __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
+    pdl_entry();
     __shared__ uint32_t ws[33];
     __shared__ uint64_t wsum[33];
     if (A.aux->dense) return;
@@ -244,6 +246,7 @@ __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
 
 // Every block writes its cuts; thread nb writes the forced cuts after the last candidate.
 __global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
+    pdl_entry();
     if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
@@ -301,6 +304,7 @@ constexpr int SBD_THREADS = 256;
 constexpr uint64_t SBD_WIN = 1ull << 20;              // window ends per bitmap pass (128 KiB)
 __global__ void __launch_bounds__(SBD_THREADS)
 sb_dense(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots, SBArgs A) {
+    pdl_entry();
     Aux *aux = A.aux;
     if (!aux->dense) return;
     extern __shared__ uint32_t bm[];
