@@ -208,6 +208,36 @@ def test_feed_matches_one_shot(pkg, pinned, bounded):
     assert np.array_equal(got2, exp)
 
 
+@pytest.mark.parametrize("window,poly", [(47, LBFS), (33, 0x104C11DB7), (9, 0x20000005)])
+def test_feed_and_shards_funnel_windows(pkg, window, poly):
+    """Windows that are not a multiple of 16 (funnel pops on the hot kernel) through the
+    streaming carry (w-1 bytes across feeds, pinned and device pieces) and through byte-range
+    shards with a w-1 halo: both equal the oracle on the whole stream."""
+    n = (3 << 20) + 4321
+    data = synthgen.random_bytes(40 + window, n)
+    p = pkg.Params(poly=poly, window=window, divisor=1024, magic=window)
+    op = oparams(p)
+    exp = oracle.chunk(data, op)
+    ch = pkg.Chunker(p)
+    assert ch.path in ("k63", "k32")
+    ch.set_ring(2, 1 << 20)
+    sizes = [1, window - 1, 70000, (1 << 20) + 5, 3, n - (1 + window - 1 + 70000 + (1 << 20) + 5 + 3)]
+    assert np.array_equal(_feed_all(ch, data, sizes, pinned=True), exp)
+    assert np.array_equal(_feed_all(ch, data, sizes[::-1], pinned=False), exp)
+    G = 3
+    bounds = [n * g // G for g in range(G + 1)]
+    parts = []
+    for g in range(G):
+        a, b = bounds[g], bounds[g + 1]
+        halo = min(window - 1, a)
+        parts.append(ch.candidates_range(dev(data[a - halo:b]), halo, a, n).cpu().numpy())
+    assert np.array_equal(np.concatenate(parts).astype(np.uint64), oracle.candidates(data, op))
+    chb = pkg.Chunker(pkg.Params(poly=poly, window=window, divisor=1024, magic=window,
+                                 min_size=256, max_size=8192))
+    assert np.array_equal(_feed_all(chb, data, sizes, pinned=True),
+                          oracle.chunk(data, oparams(chb.params)))
+
+
 def test_feed_candidate_at_piece_boundary(pkg):
     """A candidate exactly at a feed end is held, emitted once more data arrives."""
     data = synthgen.periodic(b"\x04\xd5", 4000)
