@@ -111,6 +111,9 @@ K1Fn pick_mode(int wch, bool le, bool fn) {
 }
 // The hot-kernel instance for (u64 state: deg 41..63 | deg 33..40; u32 state with a whole-byte
 // top byte | u32 state; ceil(w/16), marker set, w % 16 != 0).
+#ifndef SHRED_L2PROMO
+#define SHRED_L2PROMO CU_TENSOR_MAP_L2_PROMOTION_L2_128B   // TMA L2 promotion of the row tiles (A/B: r01_ab_variants)
+#endif
 #ifndef SHRED_PDL
 #define SHRED_PDL 1       // 0: plain stream serialization (A/B)
 #endif
@@ -344,7 +347,7 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
                                  CU_TENSOR_MAP_INTERLEAVE_NONE,
                                  ROUND == 64 ? CU_TENSOR_MAP_SWIZZLE_64B
                                              : (ROUND == 32 ? CU_TENSOR_MAP_SWIZZLE_32B : CU_TENSOR_MAP_SWIZZLE_NONE),
-                                 CU_TENSOR_MAP_L2_PROMOTION_L2_256B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+                                 (CUtensorMapL2promotion)SHRED_L2PROMO, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
         if (r != CUDA_SUCCESS) return fail(ctx, SHRED_ECUDA, "cuTensorMapEncodeTiled failed (%d)", (int)r);
     }
     pl.nslots = m.n_head + m.nrows + m.n_tail;
