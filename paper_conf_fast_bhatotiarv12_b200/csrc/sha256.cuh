@@ -31,7 +31,18 @@ __constant__ uint32_t kSha256K[64] = {
 __device__ __forceinline__ uint32_t rotr(uint32_t x, int n) { return __funnelshift_r(x, x, n); }
 
 // One SHA-256 compression of the 16 big-endian words W into H.
-__device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[16]) {
+// The rounds are ALU-pipe bound (rotates, LOP3, IADD3 all issue there, ncu 77 % of peak while
+// active); the FMA pipe is idle.  SHRED_SHA_FMA=1 moves two additions per round off the ALU
+// (x * one + y with a runtime one becomes an IMAD): +7 % on throughput-bound batches (bounded
+// chunks 410-418 -> 448 GB/s) but -8 % when the longest chunk's latency bounds the launch (1 GiB,
+// bounds off: 292 -> 270 GB/s), so it is off (profiles/r01_hash_ab.txt).
+#ifndef SHRED_SHA_FMA
+#define SHRED_SHA_FMA 0
+#endif
+__device__ __forceinline__ uint32_t fma_add(uint32_t x, uint32_t one, uint32_t y) {
+    return SHRED_SHA_FMA ? x * one + y : x + y;
+}
+__device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[16], uint32_t one) {
     uint32_t a = H[0], b = H[1], c = H[2], d = H[3], e = H[4], f = H[5], g = H[6], h = H[7];
 #pragma unroll
     for (int t = 0; t < 64; ++t) {
@@ -42,15 +53,15 @@ __device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[
             const uint32_t w15 = W[(t - 15) & 15], w2 = W[(t - 2) & 15];
             const uint32_t s0 = rotr(w15, 7) ^ rotr(w15, 18) ^ (w15 >> 3);
             const uint32_t s1 = rotr(w2, 17) ^ rotr(w2, 19) ^ (w2 >> 10);
-            w = W[t & 15] = W[t & 15] + s0 + W[(t - 7) & 15] + s1;
+            w = W[t & 15] = fma_add(W[t & 15], one, W[(t - 7) & 15]) + s0 + s1;
         }
         const uint32_t S1 = rotr(e, 6) ^ rotr(e, 11) ^ rotr(e, 25);
         const uint32_t ch = (e & f) ^ (~e & g);
-        const uint32_t t1 = h + S1 + ch + kSha256K[t] + w;
+        const uint32_t hkw = fma_add(h, one, fma_add(w, one, kSha256K[t]));
+        const uint32_t t1 = hkw + S1 + ch;
         const uint32_t S0 = rotr(a, 2) ^ rotr(a, 13) ^ rotr(a, 22);
         const uint32_t mj = (a & b) ^ (a & c) ^ (b & c);
-        const uint32_t t2 = S0 + mj;
-        h = g; g = f; f = e; e = d + t1; d = c; c = b; b = a; a = t1 + t2;
+        h = g; g = f; f = e; e = d + t1; d = c; c = b; b = a; a = t1 + S0 + mj;
     }
     H[0] += a; H[1] += b; H[2] += c; H[3] += d; H[4] += e; H[5] += f; H[6] += g; H[7] += h;
 }
@@ -166,7 +177,7 @@ __device__ __forceinline__ void sha256_store(uint8_t *digests, uint64_t chunk, c
 __global__ void __launch_bounds__(256)
 k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__restrict__ cuts,
               const uint64_t *n_cuts, uint64_t max_chunks, uint8_t *__restrict__ digests,
-              const uint32_t *__restrict__ order, unsigned long long *queue) {
+              const uint32_t *__restrict__ order, unsigned long long *queue, uint32_t one) {
     pdl_entry();
     const uint64_t ncut = *n_cuts;
     const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
@@ -184,9 +195,31 @@ k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__re
             chunk_bounds(cuts, ncut, len, chunk, a, b);
             const uint64_t L = b - a, nblk = (L + 9 + 63) / 64;
             sha256_init(H);
-            for (uint64_t blk = 0; blk < nblk; ++blk) {
+            // full blocks: the 17 aligned words of block blk+1 are loaded before block blk is
+            // compressed (software pipelining: the load latency hides behind ~1.5K cycles of
+            // rounds); the padded tail blocks take the byte path of sha256_block
+            const uint32_t sh = (uint32_t)(a & 3) * 8;
+            const uint32_t *src0 = reinterpret_cast<const uint32_t *>(in + (a & ~3ull));
+            uint64_t nfull = L / 64;                               // complete message blocks
+            if (nfull && (a & ~3ull) + 64 * nfull + 4 > len) --nfull;   // 17th word in bounds
+            uint32_t Rw[17];
+            if (nfull) {
+#pragma unroll
+                for (int k = 0; k < 17; ++k) Rw[k] = __ldg(src0 + k);
+            }
+            for (uint64_t blk = 0; blk < nfull; ++blk) {
+#pragma unroll
+                for (int k = 0; k < 16; ++k) W[k] = __byte_perm(__funnelshift_r(Rw[k], Rw[k + 1], sh), 0, 0x0123);
+                if (blk + 1 < nfull) {
+                    const uint32_t *nx = src0 + 16 * (blk + 1);
+#pragma unroll
+                    for (int k = 0; k < 17; ++k) Rw[k] = __ldg(nx + k);
+                }
+                sha256_compress(H, W, one);
+            }
+            for (uint64_t blk = nfull; blk < nblk; ++blk) {
                 sha256_block(in, len, a, L, blk, W);
-                sha256_compress(H, W);
+                sha256_compress(H, W, one);
             }
             sha256_store(digests, chunk, H);
         }

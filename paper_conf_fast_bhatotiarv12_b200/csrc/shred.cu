@@ -938,7 +938,7 @@ int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const u
     PDL(k_hash_scatter, gs, 256, 0, st, d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist, ctx->d_order);
     LAUNCHED("k_hash_scatter");
     PDL(k_hash_chunks, ctx->sm_count * SHRED_HASH_CTAS_PER_SM, SHRED_HASH_THREADS, 0, st, d_in, len, d_cuts, d_ncuts, max_chunks, d_digests,
-                                                      ctx->d_order, ctx->d_queue);
+                                                      ctx->d_order, ctx->d_queue, 1u);
     LAUNCHED("k_hash_chunks");
     return SHRED_OK;
 }
