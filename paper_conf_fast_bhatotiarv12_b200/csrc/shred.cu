@@ -87,13 +87,16 @@ typedef void (*K1Fn)(const __grid_constant__ CUtensorMap, const uint4 *, const G
 
 template <int MODE, class C>
 K1Fn pick_mode(int wch, bool le, bool fn) {
-    if (fn) {                                // windows that are not a multiple of 16: '==' marker
-        if (le) return nullptr;
-        switch (wch) {
-            case 1: return k1_bulk<MODE, C, 1, false, true>;
-            case 2: return k1_bulk<MODE, C, 2, false, true>;
-            case 3: return k1_bulk<MODE, C, 3, false, true>;
-            case 4: return k1_bulk<MODE, C, 4, false, true>;
+    if (fn) {                                // windows that are not a multiple of 16
+        switch (wch * 2 + (le ? 1 : 0)) {
+            case 2: return k1_bulk<MODE, C, 1, false, true>;
+            case 3: return k1_bulk<MODE, C, 1, true, true>;
+            case 4: return k1_bulk<MODE, C, 2, false, true>;
+            case 5: return k1_bulk<MODE, C, 2, true, true>;
+            case 6: return k1_bulk<MODE, C, 3, false, true>;
+            case 7: return k1_bulk<MODE, C, 3, true, true>;
+            case 8: return k1_bulk<MODE, C, 4, false, true>;
+            case 9: return k1_bulk<MODE, C, 4, true, true>;
             default: return nullptr;
         }
     }
@@ -589,9 +592,8 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     ctx->dp.pow2 = (p->divisor & (p->divisor - 1)) == 0 ? 1u : 0u;
     ctx->dp.marker = p->marker;
     const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
-    // the hot kernel: any w <= 64 (w % 16 != 0 with the '==' marker: funnel-shifted pops)
-    const bool fast_w = p->window >= 1 && p->window <= 64 &&
-                        (p->window % 16 == 0 || p->marker == SHRED_MARKER_EQ);
+    // the hot kernel: any w <= 64 (w % 16 != 0: funnel-shifted pops), either marker set
+    const bool fast_w = p->window >= 1 && p->window <= 64;
     const bool fast = fast_w && pow2 && p->divisor <= (1ull << 32);
     // u64-state kernel: deg 33..63 (t = mulhi(f_hi, 2^(72-k)), or a funnel shift for k <= 40);
     // u32-state kernel: deg 9..32

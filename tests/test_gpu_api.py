@@ -104,7 +104,7 @@ def test_init_validation_and_paths(pkg):
     assert pkg.Chunker(pkg.Params()).path == "k63"
     assert pkg.Chunker(pkg.Params(poly=0x104C11DB7)).path == "k32"
     assert pkg.Chunker(pkg.Params(window=47)).path == "k63"
-    assert pkg.Chunker(pkg.Params(window=47, marker=1)).path == "generic"
+    assert pkg.Chunker(pkg.Params(window=47, marker=1)).path == "k63"
     assert pkg.Chunker(pkg.Params(window=65)).path == "generic"
     ch = pkg.Chunker(pkg.Params(min_size=100))
     assert ch.max_cuts(1001) == 1000 // 100 + 1

@@ -115,12 +115,19 @@ def test_launch_shapes_around_small_threshold(pkg, poly, n):
 
 
 def test_generic_path_variants(pkg):
-    for p in (pkg.Params(window=65), pkg.Params(window=1, divisor=256, magic=7, marker=1),
-              pkg.Params(poly=(1 << 63) | 3, window=24, divisor=1024, marker=1),
+    for p in (pkg.Params(window=65), pkg.Params(window=80, divisor=256, magic=7, marker=1),
+              pkg.Params(poly=0x11D, window=24, divisor=128, magic=5, marker=1),
               pkg.Params(poly=0x11D, window=7, divisor=64, magic=9),
+              pkg.Params(divisor=3000, magic=2999, marker=1),
               pkg.Params(divisor=1 << 40, magic=12345)):
         ch = pkg.Chunker(p)
         assert ch.path == "generic"
+        check_chunk(ch, synthgen.random_bytes(11, 300000))
+    # the '<=' marker with any window <= 64 runs on the hot kernel (funnel-shifted pops)
+    for p in (pkg.Params(window=1, divisor=256, magic=7, marker=1),
+              pkg.Params(poly=(1 << 63) | 3, window=24, divisor=1024, marker=1)):
+        ch = pkg.Chunker(p)
+        assert ch.path == "k63"
         check_chunk(ch, synthgen.random_bytes(11, 300000))
 
 
@@ -208,14 +215,15 @@ def test_feed_matches_one_shot(pkg, pinned, bounded):
     assert np.array_equal(got2, exp)
 
 
-@pytest.mark.parametrize("window,poly", [(47, LBFS), (33, 0x104C11DB7), (9, 0x20000005)])
-def test_feed_and_shards_funnel_windows(pkg, window, poly):
+@pytest.mark.parametrize("window,poly,marker", [(47, LBFS, 0), (33, 0x104C11DB7, 0), (9, 0x20000005, 0),
+                                               (47, LBFS, 1), (31, 0x104C11DB7, 1)])
+def test_feed_and_shards_funnel_windows(pkg, window, poly, marker):
     """Windows that are not a multiple of 16 (funnel pops on the hot kernel) through the
     streaming carry (w-1 bytes across feeds, pinned and device pieces) and through byte-range
     shards with a w-1 halo: both equal the oracle on the whole stream."""
     n = (3 << 20) + 4321
     data = synthgen.random_bytes(40 + window, n)
-    p = pkg.Params(poly=poly, window=window, divisor=1024, magic=window)
+    p = pkg.Params(poly=poly, window=window, divisor=1024, magic=window, marker=marker)
     op = oparams(p)
     exp = oracle.chunk(data, op)
     ch = pkg.Chunker(p)
@@ -233,7 +241,7 @@ def test_feed_and_shards_funnel_windows(pkg, window, poly):
         parts.append(ch.candidates_range(dev(data[a - halo:b]), halo, a, n).cpu().numpy())
     assert np.array_equal(np.concatenate(parts).astype(np.uint64), oracle.candidates(data, op))
     chb = pkg.Chunker(pkg.Params(poly=poly, window=window, divisor=1024, magic=window,
-                                 min_size=256, max_size=8192))
+                                 min_size=256, max_size=8192, marker=marker))
     assert np.array_equal(_feed_all(chb, data, sizes, pinned=True),
                           oracle.chunk(data, oparams(chb.params)))
 
@@ -350,8 +358,10 @@ def test_fast_path_any_window(pkg, poly, window):
     assert ch.path in ("k63", "k32")
     data = synthgen.random_bytes(100 + window, (2 << 20) + 4 * window + 1)
     check_chunk(ch, data, offset=window % 16)
-    # the '<=' marker set with such windows runs on the generic path
-    assert pkg.Chunker(pkg.Params(poly=poly, window=window, divisor=512, magic=3, marker=1)).path == "generic"
+    # the '<=' marker set (L249-L251) with the same funnel windows
+    chl = pkg.Chunker(pkg.Params(poly=poly, window=window, divisor=512, magic=3, marker=1))
+    assert chl.path == ch.path
+    check_chunk(chl, data, offset=(window + 3) % 16)
 
 
 def _dense_irreducible(deg, seed):
@@ -374,3 +384,28 @@ def test_polynomial_degrees(pkg, deg):
     ch = pkg.Chunker(p)
     assert ch.path == ("k32" if 9 <= deg <= 32 else "k63" if deg >= 33 else "generic")
     check_chunk(ch, synthgen.random_bytes(deg, (2 << 20) + 123), offset=deg % 16)
+
+
+@pytest.mark.parametrize("poly", [LBFS, 0x104C11DB7])
+@pytest.mark.parametrize("log2d", [1, 20, 31, 32, 33])
+def test_divisor_range_with_planted_magic(pkg, poly, log2d):
+    """D from 2 up to past the hot kernel's 2^32 limit (the marker test keeps the low log2 D
+    bits at the top of a u32: D = 2^32 is the shift-by-0 edge).  On random data a large D hits
+    nothing, so r is planted: the residue of three real window fingerprints (oracle R2), and the
+    candidate set must be exactly the positions sharing it."""
+    if poly != LBFS and log2d > 32:
+        pytest.skip("deg 32: D <= 2^32")
+    data = synthgen.random_bytes(700 + log2d, (3 << 20) + 77)
+    op = oracle.Params(poly=poly)
+    fps = oracle.window_fps(data, op)
+    D = 1 << log2d
+    for k in (5, fps.size // 2, fps.size - 9):
+        r = int(fps[k]) % D
+        p = pkg.Params(poly=poly, divisor=D, magic=r)
+        ch = pkg.Chunker(p)
+        assert ch.path == ("generic" if log2d > 32 else "k63" if poly == LBFS else "k32")
+        got = check_chunk(ch, data)
+        if log2d >= 20:
+            exp = np.nonzero((fps % np.uint64(D)) == np.uint64(r))[0].astype(np.uint64) + np.uint64(op.window)
+            exp = exp[exp < data.size]
+            assert np.array_equal(got, exp) and got.size >= 1
