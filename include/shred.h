@@ -74,12 +74,13 @@ enum { SHRED_MARKER_EQ = 0, SHRED_MARKER_LE = 1 };
 
 /* Kernel paths the ctx selected for its parameters (shred_path). */
 enum {
-    SHRED_PATH_K63     = 1, /* deg(P) in 33..63 (the paper's reading: 63), D = 2^m <= 2^32,
-                               1 <= w <= 64, either marker set: u64 state, TMA-staged, smem
-                               LDS.64 tables                                                    */
+    SHRED_PATH_K63     = 1, /* deg(P) in 33..63 (the paper's reading: 63), 1 <= w <= 64, and
+                               either D = 2^m <= 2^32 with either marker set, or the '==' marker
+                               with any D = d 2^s, s < 32 (divisibility test on the full state):
+                               u64 state, TMA-staged, smem LDS.64 tables                        */
     SHRED_PATH_K32     = 2, /* deg(P) in 9..32, same w / D / marker conditions: u32 state, LDS.32 */
-    SHRED_PATH_GENERIC = 3  /* any other valid parameters (deg 8, w > 64, D not a power of two
-                               or > 2^32): byte-at-a-time                                       */
+    SHRED_PATH_GENERIC = 3  /* any other valid parameters (deg 8, w > 64, the '<=' marker with D
+                               not a power of two, D with 2^32 | D): byte-at-a-time             */
 };
 
 /* Fill *p with the paper defaults (readings Q1, Q5, Q6, Q15): P = 0xbfe6b8a5bf378d83, w = 48,

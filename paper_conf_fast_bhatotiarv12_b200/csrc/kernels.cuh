@@ -9,7 +9,7 @@
 // realised with two 256-entry tables: T (reduces the byte shifted out of the top of the
 // state) and U (removes the byte leaving the window).  See DESIGN.md "Kernels".
 //
-//   k1_bulk<MODE,C,WCH,LE,FN>  TMA-staged hot loop (FN: w not a multiple of 16, funnel pops).  The input is viewed as a 2-D [rows][S]
+//   k1_bulk<MODE,C,WCH,MK,FN>  TMA-staged hot loop (FN: w not a multiple of 16, funnel pops).  The input is viewed as a 2-D [rows][S]
 //                   tensor; each consumer thread rolls CH = 2 rows (independent chains) in one
 //                   basic block; rounds of 32 B per row arrive in a 4-stage shared-memory ring
 //                   (SWIZZLE_32B, conflict-free LDS.128) fed by a producer warp.  T/U live in
@@ -116,7 +116,7 @@ struct DevParams {              // chunking parameters as the kernels need them
 
 // The marker predicate of the generic path (L247-L251, L447-L451).  The 64-bit modulo is a
 // software division: keep it behind a real branch so power-of-two divisors never pay for it.
-__device__ __noinline__ uint64_t mod_u64(uint64_t f, uint64_t d) { return f % d; }
+static __device__ __noinline__ uint64_t mod_u64(uint64_t f, uint64_t d) { return f % d; }
 __device__ __forceinline__ bool generic_marker(uint64_t f, const DevParams &P) {
     uint64_t v;
     if (P.pow2) v = f & P.dmask;
@@ -367,6 +367,7 @@ __device__ __forceinline__ uint32_t roll_slot(const Job &J, const DevParams &P, 
     return cnt;
 }
 
+#ifndef SHRED_K1_ONLY   // k1_inst.cu (hot-kernel instances) compiles only k1_bulk
 // ------------------------------------------------------------------------------ k1_generic
 // Generic-only path: one thread per slot, one group per block of GEN_THREADS slots.
 __global__ void __launch_bounds__(GEN_THREADS)
@@ -385,6 +386,8 @@ k1_generic(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots
     if (threadIdx.x == 0) J.group_sum[blockIdx.x] = tot;
 }
 
+#endif  // SHRED_K1_ONLY
+
 // ------------------------------------------------------------------------------ k1_bulk
 // Per-lane constants of the hot loop.  The multipliers are runtime values so that ptxas keeps
 // the index math and the marker-test shift on the FMA pipe (IMAD / IMAD.HI) instead of turning
@@ -398,6 +401,12 @@ struct BulkCtx {
     uint32_t tmul;      // 2^(32-m): (f_lo * tmul) keeps the low m bits at the top
     uint32_t rsh;       // r << (32-m)
     uint32_t tsel;      // K32B: PRMT selector 0x55s4 placing byte s = (k-8)/8 of f at bits 8..15
+    // MK_DIV (any D = d 2^s, s < 32): f mod D == r  <=>  D | (f + D - r)  (no overflow: f < 2^63,
+    // D - r <= 2^63)  <=>  rotr64((f + D - r) * d^-1 mod 2^64, s) <= floor((2^64 - 1) / D)
+    uint64_t dc;        // D - r
+    uint64_t dinv;      // d^-1 mod 2^64 (d = the odd part of D)
+    uint64_t dlim;      // floor((2^64 - 1) / D)
+    uint32_t dsh;       // s
 };
 
 // One byte step, u64 state (deg P = k in 41..63; the paper's reading k = 63), f = fh:fl < 2^k:
@@ -442,6 +451,7 @@ template <> struct State<MODE_K63> {
         step63<K>(fl, fh, in, pop, c);
     }
     __device__ __forceinline__ uint32_t low() const { return fl; }
+    __device__ __forceinline__ uint64_t full() const { return ((uint64_t)fh << 32) | fl; }
 };
 template <> struct State<MODE_K40> {
     uint32_t fl = 0, fh = 0;
@@ -449,6 +459,7 @@ template <> struct State<MODE_K40> {
         step63<K, true>(fl, fh, in, pop, c);
     }
     __device__ __forceinline__ uint32_t low() const { return fl; }
+    __device__ __forceinline__ uint64_t full() const { return ((uint64_t)fh << 32) | fl; }
 };
 template <> struct State<MODE_K32> {
     uint32_t f = 0;
@@ -456,6 +467,7 @@ template <> struct State<MODE_K32> {
         step32<K, false>(f, in, pop, c);
     }
     __device__ __forceinline__ uint32_t low() const { return f; }
+    __device__ __forceinline__ uint64_t full() const { return f; }
 };
 template <> struct State<MODE_K32B> {
     uint32_t f = 0;
@@ -463,16 +475,21 @@ template <> struct State<MODE_K32B> {
         step32<K, true>(f, in, pop, c);
     }
     __device__ __forceinline__ uint32_t low() const { return f; }
+    __device__ __forceinline__ uint64_t full() const { return f; }
 };
 
+// Marker kinds of the hot kernel: MK_EQ / MK_LE: D = 2^m <= 2^32, "fp mod D == r" / "<= r"
+// (L447-L451 / L249-L251) on the low word; MK_DIV: "fp mod D == r" for a D that is not a power of
+// two (Q8: the integer remainder of the fingerprint's value), on the full state.
+enum { MK_EQ = 0, MK_LE = 1, MK_DIV = 2 };
 // marker test: (f mod D) == r  <=>  (f_lo << (32-m)) == (r << (32-m))   (D = 2^m <= 2^32)
 __device__ __forceinline__ bool is_marker(uint32_t lo, const BulkCtx &c) { return lo * c.tmul == c.rsh; }
 // m | BIT if marker else m: ISETP + predicated LOP3 (the PTX predication survives ptxas).
 // LE: the "mod D <= r" marker set (L249-L251): (f_lo << (32-m)) <= (r << (32-m)).
-template <uint32_t BIT, bool LE>
+template <uint32_t BIT, int MK>
 __device__ __forceinline__ uint32_t or_if_marker(uint32_t m, uint32_t lo, const BulkCtx &c) {
     const uint32_t x = lo * c.tmul;
-    if (LE)
+    if (MK == MK_LE)
         asm("{\n .reg .pred p;\n setp.le.u32 p, %1, %2;\n @p or.b32 %0, %0, %3;\n}"
             : "+r"(m) : "r"(x), "r"(c.rsh), "n"(BIT));
     else
@@ -481,12 +498,22 @@ __device__ __forceinline__ uint32_t or_if_marker(uint32_t m, uint32_t lo, const 
     return m;
 }
 
+// MK_DIV: divisibility of f + D - r by D = d 2^s (Granlund-Montgomery): multiply by d^-1 mod
+// 2^64, rotate right by s, compare with floor((2^64 - 1) / D).
+template <uint32_t BIT>
+__device__ __forceinline__ uint32_t or_if_div(uint32_t m, uint64_t f, const BulkCtx &c) {
+    const uint64_t q = (f + c.dc) * c.dinv;
+    const uint32_t ql = (uint32_t)q, qh = (uint32_t)(q >> 32);
+    const uint64_t rot = ((uint64_t)__funnelshift_r(qh, ql, c.dsh) << 32) | __funnelshift_r(ql, qh, c.dsh);
+    return rot <= c.dlim ? (m | BIT) : m;
+}
+
 struct SlotOut {
     uint64_t *lst; uint32_t cnt; uint32_t cap;
 };
 
 // Emit the marker hits of one 16-byte chunk: bit j of m = a hit at window end pos + j.
-__device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t min_i, uint64_t c_limit,
+static __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t min_i, uint64_t c_limit,
                                        SlotOut &o) {
     while (m) {
         const int j = __ffs(m) - 1;
@@ -503,9 +530,11 @@ __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t min_i,
 #if SHRED_HITMODE == 0
 #define SHRED_MARK(ch, q) m[ch] |= is_marker(st[ch].low(), c) ? (1u << (4 * J + q)) : 0u;
 #else
-#define SHRED_MARK(ch, q) m[ch] = or_if_marker<(1u << (4 * J + q)), LE>(m[ch], st[ch].low(), c);
+#define SHRED_MARK(ch, q)                                                                   \
+    m[ch] = (MK == MK_DIV) ? or_if_div<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
+                           : or_if_marker<(1u << (4 * J + q)), MK>(m[ch], st[ch].low(), c);
 #endif
-template <int MODE, int CH, bool TEST, int J, bool LE>
+template <int MODE, int CH, bool TEST, int J, int MK>
 __device__ __forceinline__ void word4xN(State<MODE> (&st)[CH], const uint32_t (&in)[CH],
                                         const uint32_t (&pop)[CH], uint32_t (&m)[CH], const BulkCtx &c) {
 #pragma unroll
@@ -537,7 +566,7 @@ __device__ __forceinline__ void word4xN(State<MODE> (&st)[CH], const uint32_t (&
 
 // 16 bytes of CH chains in one basic block (ILP across the chains): d = data chunk,
 // p = the chunk 48 bytes earlier (its bytes leave the window).
-template <int MODE, int CH, bool TEST, bool LE>
+template <int MODE, int CH, bool TEST, int MK>
 __device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d)[CH], const uint4 (&p)[CH],
                                           const BulkCtx &c, uint32_t (&m)[CH]) {
     uint32_t in[CH], po[CH];
@@ -545,20 +574,22 @@ __device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d
     for (int ch = 0; ch < CH; ++ch) m[ch] = 0;
 #pragma unroll
     for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].x; po[ch] = p[ch].x; }
-    word4xN<MODE, CH, TEST, 0, LE>(st, in, po, m, c);
+    word4xN<MODE, CH, TEST, 0, MK>(st, in, po, m, c);
 #pragma unroll
     for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].y; po[ch] = p[ch].y; }
-    word4xN<MODE, CH, TEST, 1, LE>(st, in, po, m, c);
+    word4xN<MODE, CH, TEST, 1, MK>(st, in, po, m, c);
 #pragma unroll
     for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].z; po[ch] = p[ch].z; }
-    word4xN<MODE, CH, TEST, 2, LE>(st, in, po, m, c);
+    word4xN<MODE, CH, TEST, 2, MK>(st, in, po, m, c);
 #pragma unroll
     for (int ch = 0; ch < CH; ++ch) { in[ch] = d[ch].w; po[ch] = p[ch].w; }
-    word4xN<MODE, CH, TEST, 3, LE>(st, in, po, m, c);
+    word4xN<MODE, CH, TEST, 3, MK>(st, in, po, m, c);
 }
 
 struct BulkConst {
     uint32_t mhi, m256, tmul, rsh, tsel;
+    uint64_t dc, dinv, dlim;   // MK_DIV constants (BulkCtx)
+    uint32_t dsh;
     uint32_t fu, fsel;  // FN windows (w % 16 != 0): e = 16*ceil(w/16) - w = 4*fu + v, fsel = PRMT
                         // selector of bytes v..v+3 (0x3210 + 0x1111 v)
 };
@@ -596,8 +627,8 @@ __device__ __forceinline__ void pops16(const uint4 (&lo)[CH], const uint4 (&hi)[
 // SWIZZLE_32B for 32-byte rounds, no swizzle for 16-byte rounds).  The window is fixed at
 // w = 48 = 3 chunks of 16 B: the byte leaving the window at chunk q is the same byte slot of
 // chunk q-3, kept in a 4-slot register ring per chain (slot = chunk index mod 4).  WCH = w/16
-// (w in {16, 32, 48, 64}) generalises the pop distance; LE selects the "mod D <= r" marker set.
-template <int MODE, class C, int WCH, bool LE, bool FN = false>
+// (w in {16, 32, 48, 64}) generalises the pop distance; MK selects the marker kind.
+template <int MODE, class C, int WCH, int MK, bool FN = false>
 __global__ void __launch_bounds__(C::NTC + 32, 1)
 k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_img,
         const GenTables *__restrict__ gt, Job J, DevParams P, BulkConst K) {
@@ -694,6 +725,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         c.laneU = 128u + (uint32_t)lane * 4u;
     }
     c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh; c.tsel = K.tsel;
+    c.dc = K.dc; c.dinv = K.dinv; c.dlim = K.dlim; c.dsh = K.dsh;
 
     bool act[CH];
     uint64_t pos0[CH];
@@ -735,7 +767,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                 hi[ch] = (q + 1 >= WCH) ? R[ch][q + 1 - WCH] : Z;
             }
             pops16<FN, CH>(lo, hi, p, K);
-            chunk16xN<MODE, CH, false, LE>(st, d, p, c, m);
+            chunk16xN<MODE, CH, false, MK>(st, d, p, c, m);
         }
     }
 
@@ -773,7 +805,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                     }
                     pops16<FN, CH>(lo, hi, p, K);
                 }
-                chunk16xN<MODE, CH, true, LE>(st, d, p, c, m);
+                chunk16xN<MODE, CH, true, MK>(st, d, p, c, m);
 #pragma unroll
                 for (int ch = 0; ch < CH; ++ch) {
                     R[ch][cq] = D[ch][u];
@@ -798,6 +830,13 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     if (tid == 0) J.group_sum[1 + blockIdx.x] = base;
 }
 
+// A hot-kernel instance; pick_k1 / pick_k1_small (k1_inst.cu) map parameters to instances.
+typedef void (*K1Fn)(const __grid_constant__ CUtensorMap, const uint4 *, const GenTables *, Job,
+                     DevParams, BulkConst);
+K1Fn pick_k1(int k, bool byteidx, int wch, int mk, bool fn);
+K1Fn pick_k1_small(int k, bool byteidx, int wch, int mk, bool fn);
+
+#ifndef SHRED_K1_ONLY
 // ------------------------------------------------------------------------------ k_total
 // Sum of the group sums -> aux->total (bounded path: needed on the host before k_scatter).
 __global__ void k_total(const uint64_t *__restrict__ group_sum, uint32_t ngroups, Aux *aux) {
@@ -986,5 +1025,6 @@ __global__ void k_synth_fill(uint8_t *dst, uint64_t len, uint64_t seed, uint64_t
         }
     }
 }
+#endif  // SHRED_K1_ONLY
 
 }  // namespace shred

@@ -82,38 +82,6 @@ void byte_times_xpow(uint64_t P, int k, uint64_t e, uint64_t out[256]) {
     }
 }
 
-typedef void (*K1Fn)(const __grid_constant__ CUtensorMap, const uint4 *, const GenTables *, Job,
-                     DevParams, BulkConst);
-
-template <int MODE, class C>
-K1Fn pick_mode(int wch, bool le, bool fn) {
-    if (fn) {                                // windows that are not a multiple of 16
-        switch (wch * 2 + (le ? 1 : 0)) {
-            case 2: return k1_bulk<MODE, C, 1, false, true>;
-            case 3: return k1_bulk<MODE, C, 1, true, true>;
-            case 4: return k1_bulk<MODE, C, 2, false, true>;
-            case 5: return k1_bulk<MODE, C, 2, true, true>;
-            case 6: return k1_bulk<MODE, C, 3, false, true>;
-            case 7: return k1_bulk<MODE, C, 3, true, true>;
-            case 8: return k1_bulk<MODE, C, 4, false, true>;
-            case 9: return k1_bulk<MODE, C, 4, true, true>;
-            default: return nullptr;
-        }
-    }
-    switch (wch * 2 + (le ? 1 : 0)) {
-        case 2: return k1_bulk<MODE, C, 1, false>;
-        case 3: return k1_bulk<MODE, C, 1, true>;
-        case 4: return k1_bulk<MODE, C, 2, false>;
-        case 5: return k1_bulk<MODE, C, 2, true>;
-        case 6: return k1_bulk<MODE, C, 3, false>;
-        case 7: return k1_bulk<MODE, C, 3, true>;
-        case 8: return k1_bulk<MODE, C, 4, false>;
-        case 9: return k1_bulk<MODE, C, 4, true>;
-        default: return nullptr;
-    }
-}
-// The hot-kernel instance for (u64 state: deg 41..63 | deg 33..40; u32 state with a whole-byte
-// top byte | u32 state; ceil(w/16), marker set, w % 16 != 0).
 #ifndef SHRED_L2PROMO
 #define SHRED_L2PROMO CU_TENSOR_MAP_L2_PROMOTION_L2_128B   // TMA L2 promotion of the row tiles (A/B: r01_ab_variants)
 #endif
@@ -123,18 +91,6 @@ K1Fn pick_mode(int wch, bool le, bool fn) {
 #ifndef SHRED_BYTEIDX
 #define SHRED_BYTEIDX 1   // deg 16/24/32: PRMT table index (MODE_K32B); 0: IMAD index (MODE_K32)
 #endif
-K1Fn pick_k1(int k, bool byteidx, int wch, bool le, bool fn) {
-    if (k >= 41) return pick_mode<MODE_K63, CfgK63>(wch, le, fn);
-    if (k >= 33) return pick_mode<MODE_K40, CfgK63>(wch, le, fn);
-    return byteidx ? pick_mode<MODE_K32B, CfgK32>(wch, le, fn) : pick_mode<MODE_K32, CfgK32>(wch, le, fn);
-}
-// The small-input shape (CfgSmall) exists for the paper's window with the equality marker.
-K1Fn pick_k1_small(int k, bool byteidx, int wch, bool le, bool fn) {
-    if (wch != 3 || le || fn || (k >= 33 && k <= 40)) return nullptr;
-    if (k >= 41) return k1_bulk<MODE_K63, CfgSmall, 3, false>;
-    return byteidx ? k1_bulk<MODE_K32B, CfgSmall, 3, false> : k1_bulk<MODE_K32, CfgSmall, 3, false>;
-}
-
 typedef CUresult (*EncodeTiledFn)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *,
                                   const cuuint64_t *, const cuuint64_t *, const cuuint32_t *,
                                   const cuuint32_t *, CUtensorMapInterleave, CUtensorMapSwizzle,
@@ -151,6 +107,7 @@ struct shred_ctx {
     int device = 0;
     int path = 0;
     int k = 0;
+    int mk = MK_EQ;                      // marker kind of the hot kernel (kernels.cuh MK_*)
     DevParams dp{};
     uint4 *d_tab_img = nullptr;          // 64 KiB replicated T|U image (fast paths)
     GenTables *d_gen = nullptr;          // plain T/U (generic path, recompute)
@@ -391,7 +348,7 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
             ctx->prof_bytes += (pl.J.map.t_end - pl.J.map.head_start);
             CK(cudaEventRecord(e0, st), "profile record");
         }
-        const int m = 32 - (int)__builtin_ctzll(ctx->p.divisor);     // D = 2^(32-m')
+        const int m = ctx->mk == MK_DIV ? 0 : 32 - (int)__builtin_ctzll(ctx->p.divisor);   // D = 2^(32-m)
         BulkConst K;
         // top byte t = f >> (k-8): u64 state mulhi(f_hi, 2^(72-k)); u32 state mulhi(f, 2^(40-k))
         K.mhi = ctx->path == SHRED_PATH_K63 ? (ctx->k >= 41 ? (1u << (72 - ctx->k)) : (uint32_t)(ctx->k - 8))
@@ -402,6 +359,14 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         K.m256 = 256u;
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
+        {   // MK_DIV: D = d 2^s; d^-1 mod 2^64 by Newton's iteration (d odd: d*d = 1 mod 8)
+            const uint64_t D = ctx->p.divisor;
+            const uint32_t sh = (uint32_t)__builtin_ctzll(D);
+            const uint64_t d = D >> sh;
+            uint64_t inv = d;
+            for (int it = 0; it < 5; ++it) inv *= 2u - d * inv;
+            K.dc = D - ctx->p.magic; K.dinv = inv; K.dlim = ~0ull / D; K.dsh = sh;
+        }
         K.tsel = 0x5504u | ((uint32_t)((ctx->k - 8) / 8) << 4);         // byte (k-8)/8 -> bits 8..15
         int smem = ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM;
         int threads = (ctx->path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC) + 32;
@@ -592,9 +557,14 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     ctx->dp.pow2 = (p->divisor & (p->divisor - 1)) == 0 ? 1u : 0u;
     ctx->dp.marker = p->marker;
     const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
-    // the hot kernel: any w <= 64 (w % 16 != 0: funnel-shifted pops), either marker set
+    // the hot kernel: any w <= 64 (w % 16 != 0: funnel-shifted pops); D = 2^m <= 2^32 with either
+    // marker set on the low word, or the '==' marker with any D = d 2^s (s < 32) by the
+    // divisibility test on the full state (MK_DIV)
     const bool fast_w = p->window >= 1 && p->window <= 64;
-    const bool fast = fast_w && pow2 && p->divisor <= (1ull << 32);
+    if (pow2 && p->divisor <= (1ull << 32)) ctx->mk = p->marker == SHRED_MARKER_LE ? MK_LE : MK_EQ;
+    else if (p->marker == SHRED_MARKER_EQ && __builtin_ctzll(p->divisor) < 32) ctx->mk = MK_DIV;
+    else ctx->mk = -1;
+    const bool fast = fast_w && ctx->mk >= 0;
     // u64-state kernel: deg 33..63 (t = mulhi(f_hi, 2^(72-k)), or a funnel shift for k <= 40);
     // u32-state kernel: deg 9..32
     if (k >= 33 && k <= 63 && fast) ctx->path = SHRED_PATH_K63;
@@ -655,13 +625,13 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         const bool byteidx = SHRED_BYTEIDX && ctx->path == SHRED_PATH_K32 && (k == 16 || k == 24 || k == 32);
         const int wch = (int)((p->window + 15) / 16);
         const bool funnel = p->window % 16 != 0;
-        ctx->k1_fn = pick_k1(k, byteidx, wch, p->marker == SHRED_MARKER_LE, funnel);
+        ctx->k1_fn = pick_k1(k, byteidx, wch, ctx->mk, funnel);
         if (!ctx->k1_fn ||
             cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM) != cudaSuccess)
             return bail(SHRED_ECUDA);
 #ifndef SHRED_NO_SMALL
-        ctx->k1_small_fn = pick_k1_small(k, byteidx, wch, p->marker == SHRED_MARKER_LE, funnel);
+        ctx->k1_small_fn = pick_k1_small(k, byteidx, wch, ctx->mk, funnel);
 #endif
         if (ctx->k1_small_fn &&
             cudaFuncSetAttribute(ctx->k1_small_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,

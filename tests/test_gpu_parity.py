@@ -323,15 +323,46 @@ def test_bounded_adversarial_stream(pkg):
 
 # ------------------------------------------------------------------ variants (f4)
 def test_marker_le_and_non_pow2_divisor(pkg):
-    """The "value mod p <= constant" marker set (L249-L251) and divisors that are not powers of
-    two run on the generic path, bit-exact vs the oracle; bounded mode on top."""
+    """Divisors that are not powers of two (Q8: the integer remainder of the fingerprint's value):
+    the '==' marker runs on the hot kernel (divisibility test on the full state), the
+    "value mod p <= constant" set (L249-L251) on the generic path; bit-exact vs the oracle,
+    bounded mode on top."""
     data = synthgen.random_bytes(31, (2 << 20) + 77)
-    for p in (pkg.Params(divisor=10000, magic=1234),
-              pkg.Params(divisor=12345, magic=3, marker=1), pkg.Params(divisor=3, magic=0),
-              pkg.Params(divisor=5000, magic=4, marker=1, min_size=1000, max_size=20000)):
+    for p, path in ((pkg.Params(divisor=10000, magic=1234), "k63"),
+                    (pkg.Params(divisor=12345, magic=3, marker=1), "generic"),
+                    (pkg.Params(divisor=3, magic=0), "k63"),
+                    (pkg.Params(divisor=3000, magic=2999, min_size=1000, max_size=20000), "k63"),
+                    (pkg.Params(divisor=5000, magic=4, marker=1, min_size=1000, max_size=20000), "generic")):
         ch = pkg.Chunker(p)
-        assert ch.path == "generic"
+        assert ch.path == path
         check_chunk(ch, data)
+
+
+@pytest.mark.parametrize("poly", [LBFS, 0x104C11DB7, 0x20000005, None])   # K63, K32B, K32, K40
+@pytest.mark.parametrize("D", [3, 7, 10000, 3 << 20, 3 << 31, (1 << 40) + 1, 12345678901, (1 << 32) - 1])
+def test_non_pow2_divisor_hot_kernel(pkg, poly, D):
+    """'==' marker with D = d 2^s (d odd > 1, s < 32) on the hot kernel: f mod D == r iff
+    rotr64((f + D - r) d^-1, s) <= floor((2^64-1)/D).  Large D hit nothing on random data, so r is
+    planted from real window fingerprints (oracle R2); a funnel window (w = 47) and a feed too."""
+    if poly is None:
+        poly = _dense_irreducible(37, 37)
+    k = oracle.degree(poly)
+    if D > (1 << k):
+        pytest.skip("D <= 2^deg")
+    data = synthgen.random_bytes(int(D % 1000) + k, (3 << 20) + 333)
+    fps = oracle.window_fps(data, oracle.Params(poly=poly))
+    for w, r in ((48, int(fps[fps.size // 3]) % D), (47, 1 % D)):
+        p = pkg.Params(poly=poly, window=w, divisor=D, magic=r)
+        ch = pkg.Chunker(p)
+        assert ch.path == ("k63" if k >= 33 else "k32")
+        got = check_chunk(ch, data, offset=w % 16)
+        if w == 48:
+            assert got.size >= 1
+    # streaming with the carry across pinned pieces
+    ch = pkg.Chunker(pkg.Params(poly=poly, divisor=D, magic=int(fps[7]) % D))
+    exp = oracle.chunk(data, oparams(ch.params))
+    n = data.size
+    assert np.array_equal(_feed_all(ch, data, [n // 3, 47, n - n // 3 - 47], True), exp)
 
 
 @pytest.mark.parametrize("poly,path", [(LBFS, "k63"), (0x104C11DB7, "k32")])
