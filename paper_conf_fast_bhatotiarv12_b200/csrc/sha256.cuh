@@ -31,16 +31,18 @@ __constant__ uint32_t kSha256K[64] = {
 __device__ __forceinline__ uint32_t rotr(uint32_t x, int n) { return __funnelshift_r(x, x, n); }
 
 // One SHA-256 compression of the 16 big-endian words W into H.
-// The rounds are ALU-pipe bound (rotates, LOP3, IADD3 all issue there, ncu 77 % of peak while
-// active); the FMA pipe is idle.  SHRED_SHA_FMA=1 moves two additions per round off the ALU
-// (x * one + y with a runtime one becomes an IMAD): +7 % on throughput-bound batches (bounded
-// chunks 410-418 -> 448 GB/s) but -8 % when the longest chunk's latency bounds the launch (1 GiB,
-// bounds off: 292 -> 270 GB/s), so it is off (profiles/r01_hash_ab.txt).
+// The rounds are bound by the ALU pipe of the warp's SM sub-partition (rotates, LOP3 and IADD3
+// all issue there: ~21.5 ALU instructions per round at 2 cycles each), and the warps hashing the
+// longest chunks set the launch time.  SHRED_SHA_FMA=2 (default) turns every addition into an
+// IMAD (x * one + y with a runtime one) on the otherwise idle FMA pipe, leaving ~16 rotate/logic
+// ops per round on the ALU: 1 GiB, bounds off 294 -> 396 GB/s, bounded chunks 400 -> 500 GB/s.
+// 1 = only two additions per round moved (292 -> 270); 0 = all on the ALU
+// (profiles/r01_hash_ab.txt).
 #ifndef SHRED_SHA_FMA
-#define SHRED_SHA_FMA 0
+#define SHRED_SHA_FMA 2
 #endif
 __device__ __forceinline__ uint32_t fma_add(uint32_t x, uint32_t one, uint32_t y) {
-    return SHRED_SHA_FMA ? x * one + y : x + y;
+    return SHRED_SHA_FMA == 1 ? x * one + y : x + y;
 }
 __device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[16], uint32_t one) {
     uint32_t a = H[0], b = H[1], c = H[2], d = H[3], e = H[4], f = H[5], g = H[6], h = H[7];
@@ -53,15 +55,23 @@ __device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[
             const uint32_t w15 = W[(t - 15) & 15], w2 = W[(t - 2) & 15];
             const uint32_t s0 = rotr(w15, 7) ^ rotr(w15, 18) ^ (w15 >> 3);
             const uint32_t s1 = rotr(w2, 17) ^ rotr(w2, 19) ^ (w2 >> 10);
-            w = W[t & 15] = fma_add(W[t & 15], one, W[(t - 7) & 15]) + s0 + s1;
+            if (SHRED_SHA_FMA == 2)
+                w = W[t & 15] = s1 * one + (s0 * one + (W[t & 15] * one + W[(t - 7) & 15]));
+            else
+                w = W[t & 15] = fma_add(W[t & 15], one, W[(t - 7) & 15]) + s0 + s1;
         }
         const uint32_t S1 = rotr(e, 6) ^ rotr(e, 11) ^ rotr(e, 25);
-        const uint32_t ch = (e & f) ^ (~e & g);
-        const uint32_t hkw = fma_add(h, one, fma_add(w, one, kSha256K[t]));
-        const uint32_t t1 = hkw + S1 + ch;
         const uint32_t S0 = rotr(a, 2) ^ rotr(a, 13) ^ rotr(a, 22);
+        const uint32_t ch = (e & f) ^ (~e & g);
         const uint32_t mj = (a & b) ^ (a & c) ^ (b & c);
-        h = g; g = f; f = e; e = d + t1; d = c; c = b; b = a; a = t1 + S0 + mj;
+        if (SHRED_SHA_FMA == 2) {          // every addition an IMAD (x * one + y): ALU keeps the logic
+            const uint32_t t1 = (ch * one + (S1 * one + (w * one + (h * one + kSha256K[t]))));
+            h = g; g = f; f = e; e = d * one + t1; d = c; c = b; b = a; a = mj * one + (S0 * one + t1);
+        } else {
+            const uint32_t hkw = fma_add(h, one, fma_add(w, one, kSha256K[t]));
+            const uint32_t t1 = hkw + S1 + ch;
+            h = g; g = f; f = e; e = d + t1; d = c; c = b; b = a; a = t1 + S0 + mj;
+        }
     }
     H[0] += a; H[1] += b; H[2] += c; H[3] += d; H[4] += e; H[5] += f; H[6] += g; H[7] += h;
 }
