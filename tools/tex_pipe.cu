@@ -12,6 +12,8 @@
 //   mode 4: T LDS.64 + U as two 16-entry halves (U = Ulo[o & 15] ^ Uhi[o >> 4], one 128-B line
 //           each) by tex1Dfetch
 //   mode 5: T LDS.64 only (half the lookups: the ceiling if U were free)
+//   mode 6/7/8: T LDS.64; U by tex1Dfetch for 3/4/6 of every 16 bytes, by LDS.64 for the rest
+//           (the two data pipes in parallel)
 // Output: one JSON line per mode with the input-byte rate each mix would allow.
 //
 // Build/run (GPU box): nvcc -O3 -gencode arch=compute_100a,code=sm_100a -o /tmp/tex_pipe
@@ -52,6 +54,14 @@ __global__ void __launch_bounds__(512, 1) mix(uint32_t *out, int iters, cudaText
             } else if (MODE == 3) {
                 const uint2 u = __ldg(gU + o);
                 c = u.x; e = u.y;
+            } else if (MODE >= 6) {
+                constexpr int NT = MODE == 6 ? 3 : MODE == 7 ? 4 : 6;
+                if (j % 16 < NT) {
+                    const uint2 u = tex1Dfetch<uint2>(tex, (int)o);
+                    c = u.x; e = u.y;
+                } else {
+                    asm volatile("ld.shared.v2.u32 {%0,%1}, [%2];" : "=r"(c), "=r"(e) : "r"(laneU + o * 256));
+                }
             } else if (MODE == 4) {
                 const uint2 u0 = tex1Dfetch<uint2>(texh, (int)(o & 15u));
                 const uint2 u1 = tex1Dfetch<uint2>(texh, (int)(16u + (o >> 4)));
@@ -121,5 +131,8 @@ int main() {
     run<3>(p.multiProcessorCount, clk, tex, texh, dU);
     run<4>(p.multiProcessorCount, clk, tex, texh, dU);
     run<5>(p.multiProcessorCount, clk, tex, texh, dU);
+    run<6>(p.multiProcessorCount, clk, tex, texh, dU);
+    run<7>(p.multiProcessorCount, clk, tex, texh, dU);
+    run<8>(p.multiProcessorCount, clk, tex, texh, dU);
     return 0;
 }
