@@ -299,11 +299,16 @@ class Chunker:
             raise ShredError(f"capacity {cap} < {n} cuts")
         return out[:n]
 
-    def flush(self) -> torch.Tensor:
-        out = self._out(1)
+    def flush(self, cap: int = 64) -> torch.Tensor:
+        """End the stream; returns the cuts it emits (the feeds have already emitted every cut
+        strictly inside the stream that they could decide, so this is normally empty)."""
+        out = self._out(cap)
         rc = lib().shred_flush(self._ctx, out.data_ptr(), out.numel(), self._n.data_ptr(), _stream(None))
         self._check(rc, "shred_flush")
-        return out[:int(self._n.item())]
+        n = int(self._n.item())
+        if n > cap:
+            raise ShredError(f"capacity {cap} < {n} cuts")
+        return out[:n]
 
     def reset(self) -> None:
         self._check(lib().shred_reset(self._ctx), "shred_reset")
