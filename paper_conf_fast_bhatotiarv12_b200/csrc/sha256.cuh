@@ -44,6 +44,8 @@ __device__ __forceinline__ uint32_t rotr(uint32_t x, int n) { return __funnelshi
 __device__ __forceinline__ uint32_t fma_add(uint32_t x, uint32_t one, uint32_t y) {
     return SHRED_SHA_FMA == 1 ? x * one + y : x + y;
 }
+
+template <int SHA_FMA = SHRED_SHA_FMA>
 __device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[16], uint32_t one) {
     uint32_t a = H[0], b = H[1], c = H[2], d = H[3], e = H[4], f = H[5], g = H[6], h = H[7];
 #pragma unroll
@@ -55,7 +57,7 @@ __device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[
             const uint32_t w15 = W[(t - 15) & 15], w2 = W[(t - 2) & 15];
             const uint32_t s0 = rotr(w15, 7) ^ rotr(w15, 18) ^ (w15 >> 3);
             const uint32_t s1 = rotr(w2, 17) ^ rotr(w2, 19) ^ (w2 >> 10);
-            if (SHRED_SHA_FMA == 2)
+            if (SHA_FMA == 2)
                 w = W[t & 15] = s1 * one + (s0 * one + (W[t & 15] * one + W[(t - 7) & 15]));
             else
                 w = W[t & 15] = fma_add(W[t & 15], one, W[(t - 7) & 15]) + s0 + s1;
@@ -64,7 +66,7 @@ __device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[
         const uint32_t S0 = rotr(a, 2) ^ rotr(a, 13) ^ rotr(a, 22);
         const uint32_t ch = (e & f) ^ (~e & g);
         const uint32_t mj = (a & b) ^ (a & c) ^ (b & c);
-        if (SHRED_SHA_FMA == 2) {          // every addition an IMAD (x * one + y): ALU keeps the logic
+        if (SHA_FMA == 2) {                // every addition an IMAD (x * one + y): ALU keeps the logic
             const uint32_t t1 = (ch * one + (S1 * one + (w * one + (h * one + kSha256K[t]))));
             h = g; g = f; f = e; e = d * one + t1; d = c; c = b; b = a; a = mj * one + (S0 * one + t1);
         } else {
