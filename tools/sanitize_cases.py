@@ -20,7 +20,7 @@ def check(ch, data, off=0):
     x.copy_(torch.from_numpy(data))
     got = ch.chunk(x).cpu().numpy().astype(np.uint64)
     p = ch.params
-    exp = oracle.chunk(data, oracle.Params(p.poly, p.window, p.divisor, p.magic, p.min_size, p.max_size))
+    exp = oracle.chunk(data, oracle.Params(p.poly, p.window, p.divisor, p.magic, p.min_size, p.max_size, p.marker))
     assert np.array_equal(got, exp), (p, data.size)
 
 
@@ -34,6 +34,20 @@ def main():
     check(pkg.Chunker(pkg.Params(min_size=2048, max_size=65536)), data)
     check(pkg.Chunker(pkg.Params()), synthgen.periodic(b"\x04\xd5", 300000))
     check(pkg.Chunker(pkg.Params(min_size=3)), synthgen.periodic(b"\x04\xd5", 100000))
+    check(pkg.Chunker(pkg.Params(divisor=10000, magic=1234)), data, 5)          # MK_DIV
+    check(pkg.Chunker(pkg.Params(window=47, divisor=4096, magic=9, marker=1)), data[:300000], 2)   # funnel, '<='
+    check(pkg.Chunker(pkg.Params(window=65)), data[:100000])                       # generic
+    # f2 / f3: SHA-256 of every chunk (hashlib oracle) and the dedup index
+    chh = pkg.Chunker(pkg.Params())
+    x = torch.from_numpy(data).cuda()
+    cuts = chh.chunk(x)
+    dig = chh.hash_chunks(x, cuts).cpu().numpy()
+    assert np.array_equal(dig, oracle.chunk_digests(data, cuts.cpu().numpy().astype(np.uint64)))
+    chh.index_reset(1 << 12)
+    n_c = torch.tensor([cuts.numel()], dtype=torch.int64, device="cuda")
+    chh.index_insert_async(torch.from_numpy(dig.reshape(-1)).cuda(), cuts, n_c, data.size)
+    torch.cuda.synchronize()
+    assert chh.index_stats()["chunks"] == dig.shape[0]
     ch = pkg.Chunker(pkg.Params(divisor=1024, min_size=256, max_size=4096))
     ch.set_ring(2, 1 << 18)
     outs = []
