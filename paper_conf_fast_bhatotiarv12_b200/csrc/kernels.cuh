@@ -240,6 +240,26 @@ __device__ __forceinline__ uint32_t job_byte(const Job &J, uint64_t pos) {
     return 0u;
 }
 
+// Sequential reader of a job's bytes: 16-byte aligned vector loads (generic address space: the
+// source is global memory or a shared-memory staging buffer), one load per 16 positions instead
+// of a byte load per position (every lane of a warp reads its own segment, so each byte load
+// touched 32 lines); byte loads for the carried prefix and for the block that reaches `lim`.
+struct ByteStream {
+    const uint8_t *lim;                 // end of the bytes this reader may touch
+    const uint8_t *blk = nullptr;       // the 16-byte block held in v
+    uint4 v;
+    __device__ __forceinline__ uint32_t get(const Job &J, uint64_t pos) {
+        if (pos < J.p_begin) return job_byte(J, pos);
+        const uint8_t *a = J.src + (pos - J.p_begin);
+        const uint8_t *b = reinterpret_cast<const uint8_t *>(reinterpret_cast<uintptr_t>(a) & ~(uintptr_t)15);
+        if (b + 16 > lim) return *a;
+        if (b != blk) { blk = b; v = *reinterpret_cast<const uint4 *>(b); }
+        const uint32_t k = (uint32_t)(reinterpret_cast<uintptr_t>(a) & 15u);
+        const uint32_t w = (k & 8u) ? ((k & 4u) ? v.w : v.z) : ((k & 4u) ? v.y : v.x);
+        return __byte_perm(w, 0u, 0x4440u | (k & 3u));
+    }
+};
+
 // Roll the exact fingerprint over window ends [seg_start, seg_end) from a zero state
 // w-1 bytes earlier (or the first available byte), calling emit(c) for every candidate.
 // Plain byte-at-a-time form: f <- ((f << 8) mod x^k) ^ b ^ T[top byte] ^ U[B[pos-w]].
@@ -250,11 +270,13 @@ __device__ __forceinline__ void roll_generic(const Job &J, const DevParams &P, c
     const uint64_t warm = (uint64_t)P.w - 1u;
     uint64_t p = (seg_start >= lo + warm) ? seg_start - warm : lo;
     uint64_t f = 0;
+    const uint8_t *lim = seg_end > J.p_begin ? J.src + (seg_end - J.p_begin) : J.src;
+    ByteStream in{lim}, out{lim};
     for (uint64_t pos = p; pos < seg_end; ++pos) {
-        uint32_t b = job_byte(J, pos);
+        uint32_t b = in.get(J, pos);
         uint32_t t = (uint32_t)(f >> (P.k - 8u)) & 0xFFu;
         f = ((f << 8) & P.kmask) ^ (uint64_t)b ^ tab.T(t);
-        if (pos >= p + P.w) f ^= tab.U(job_byte(J, pos - P.w));
+        if (pos >= p + P.w) f ^= tab.U(out.get(J, pos - P.w));
         if (pos >= seg_start && pos >= J.min_i && generic_marker(f, P) && pos + 1 < J.c_limit)
             emit(pos + 1);
     }
