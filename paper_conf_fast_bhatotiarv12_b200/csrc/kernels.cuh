@@ -263,7 +263,10 @@ struct ByteStream {
 // Roll the exact fingerprint over window ends [seg_start, seg_end) from a zero state
 // w-1 bytes earlier (or the first available byte), calling emit(c) for every candidate.
 // Plain byte-at-a-time form: f <- ((f << 8) mod x^k) ^ b ^ T[top byte] ^ U[B[pos-w]].
-template <class Tab, class Emit>
+// VEC: bytes through ByteStream (long segments in global memory); else one load per byte (the
+// edge CTA's short segments staged in shared memory, where the per-byte latency chain matters:
+// 1 MiB call 14.3 -> 18.1 us with ByteStream there).
+template <class Tab, class Emit, bool VEC = true>
 __device__ __forceinline__ void roll_generic(const Job &J, const DevParams &P, const Tab &tab,
                                              uint64_t seg_start, uint64_t seg_end, Emit emit) {
     const uint64_t lo = J.p_begin - J.prefix_len;
@@ -273,10 +276,10 @@ __device__ __forceinline__ void roll_generic(const Job &J, const DevParams &P, c
     const uint8_t *lim = seg_end > J.p_begin ? J.src + (seg_end - J.p_begin) : J.src;
     ByteStream in{lim}, out{lim};
     for (uint64_t pos = p; pos < seg_end; ++pos) {
-        uint32_t b = in.get(J, pos);
+        uint32_t b = VEC ? in.get(J, pos) : job_byte(J, pos);
         uint32_t t = (uint32_t)(f >> (P.k - 8u)) & 0xFFu;
         f = ((f << 8) & P.kmask) ^ (uint64_t)b ^ tab.T(t);
-        if (pos >= p + P.w) f ^= tab.U(out.get(J, pos - P.w));
+        if (pos >= p + P.w) f ^= tab.U(VEC ? out.get(J, pos - P.w) : job_byte(J, pos - P.w));
         if (pos >= seg_start && pos >= J.min_i && generic_marker(f, P) && pos + 1 < J.c_limit)
             emit(pos + 1);
     }
@@ -375,17 +378,18 @@ __device__ __forceinline__ Job stage_job(const Job &J, uint64_t from, uint64_t t
 }
 
 // Roll one generic slot into its list; returns the true count.
-template <class Tab>
+template <class Tab, bool VEC = true>
 __device__ __forceinline__ uint32_t roll_slot(const Job &J, const DevParams &P, const Tab &tab,
                                               uint32_t slot) {
     uint64_t a, b;
     slot_range(J.map, slot, a, b);
     uint32_t cnt = 0;
     uint64_t *lst = J.scratch + (uint64_t)slot * J.cap;
-    roll_generic(J, P, tab, a, b, [&](uint64_t c) {
+    auto emit = [&](uint64_t c) {
         if (cnt < J.cap) lst[cnt] = c;
         ++cnt;
-    });
+    };
+    roll_generic<Tab, decltype(emit), VEC>(J, P, tab, a, b, emit);
     return cnt;
 }
 
@@ -687,8 +691,11 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         if (tid >= NTC) return;
         SmemGenTab tab{sT, sU};
         const uint32_t tail0 = J.map.n_head + J.map.nrows;
-        const uint32_t ch = (uint32_t)tid < J.map.n_head ? roll_slot(JH, P, tab, tid) : 0u;
-        const uint32_t ct = (uint32_t)tid < J.map.n_tail ? roll_slot(JT, P, tab, tail0 + tid) : 0u;
+        // staged segments (shared memory): byte loads; unstaged (too long to stage): vector loads
+        const uint32_t ch = (uint32_t)tid < J.map.n_head
+                                ? (sh ? roll_slot<SmemGenTab, false>(JH, P, tab, tid) : roll_slot(JH, P, tab, tid)) : 0u;
+        const uint32_t ct = (uint32_t)tid < J.map.n_tail
+                                ? (stl ? roll_slot<SmemGenTab, false>(JT, P, tab, tail0 + tid) : roll_slot(JT, P, tab, tail0 + tid)) : 0u;
         uint32_t th, tt;
         const uint32_t oh = block_exscan(ch, NTC, 1, ws, &th);
         const uint32_t ot = block_exscan(ct, NTC, 1, ws, &tt);
