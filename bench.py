@@ -124,6 +124,17 @@ def oracle_rate(sample: np.ndarray, threads: int):
     return sample.size / dt / 1e9, dt, c.size
 
 
+def cpu_model() -> str:
+    try:
+        with open("/proc/cpuinfo") as f:
+            for ln in f:
+                if ln.startswith("model name"):
+                    return ln.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
+
+
 def cpu_baseline(host: np.ndarray, budget_s: float = 12.0):
     """Oracle (R2, multithreaded over this process's cores) on a bounded prefix sample."""
     import oracle
@@ -134,9 +145,12 @@ def cpu_baseline(host: np.ndarray, budget_s: float = 12.0):
     n = int(min(host.size, max(16 << 20, rate * 1e9 * budget_s)))
     n -= n % 4096
     rate, dt, nc = oracle_rate(host[:n], cores)
+    rate1, dt1, _ = oracle_rate(host[: 16 << 20], 1)          # also on 1 core
     return {"value": round(rate, 4), "unit": "GB/s", "cores": cores, "kind": "oracle",
             "sample": f"first {n / 2**20:.0f} MiB of the configs[1] base file, R2 direct per-window "
-                      f"reduction (48 table lookups/window), {cores} threads, {dt:.1f} s, {nc} candidates"}
+                      f"reduction (48 table lookups/window), {cores} threads, {dt:.1f} s, {nc} candidates",
+            "value_1core": round(rate1, 4), "sample_1core": f"first 16 MiB, 1 thread, {dt1:.1f} s",
+            "cpu_model": cpu_model()}
 
 
 # ------------------------------------------------------------------------------- reference arm
