@@ -199,6 +199,15 @@ uint64_t shred_launch_count(const shred_ctx *ctx);
    their number and the input bytes they covered (algorithmic bytes = 1 per input byte), then
    clears the record.  enable = 0 stops recording. */
 int shred_profile(shred_ctx *ctx, int enable);
+
+/* Test hook (no device needed): the slot map planning would use for window ends [t_begin, t_end)
+   of a job whose bytes start at stream position p_begin at address src_addr, for kernel path
+   `path` (SHRED_PATH_*), with (small_ok) or without the small-input launch shape, on sm_count SMs.
+   out[16] = {bulk, small, head_start, head_seg, n_head, b0, S, nrows, tail_start, tail_seg,
+   n_tail, bulk CTAs, slot groups, rows per CTA, per-slot list capacity for `divisor`, threads per
+   edge CTA}.  SHRED_EINVAL on inconsistent arguments. */
+int shred_debug_plan(int path, int small_ok, int sm_count, uint64_t src_addr, uint64_t p_begin,
+                     uint64_t t_begin, uint64_t t_end, uint64_t divisor, uint64_t out[16]);
 int shred_profile_read(shred_ctx *ctx, double *ms, uint64_t *launches, uint64_t *bytes);
 
 #ifdef __cplusplus

@@ -224,6 +224,85 @@ struct Plan {
     CUtensorMap tmap;
 };
 
+// The pure part of planning (no device state; shred_debug_plan exposes it to CPU tests): the
+// slot map of window ends [t_begin, t_end) of a job whose bytes start at stream position p_begin
+// at address src_addr.  Fast paths: an aligned bulk region [b0, b0 + nrows*S) of rows for
+// k1_bulk, head segments [t_begin, b0) and tail segments for its edge CTA (at most NTC each:
+// one thread per segment).  Otherwise generic segments only.  Returns the row length S.
+struct MapShape { bool fast; bool k63; bool small_ok; int sm_count; };
+uint64_t plan_map(const MapShape &sh, uint64_t src_addr, uint64_t p_begin, uint64_t t_begin,
+                  uint64_t t_end, SlotMap &m, bool &bulk, bool &small) {
+    m = SlotMap{};
+    m.t_end = t_end;
+    const uint64_t len = t_end > t_begin ? t_end - t_begin : 0;
+    const uint64_t GS = 64;                    // head/tail segment (edge CTA)
+    uint64_t ROWS_CTA = sh.k63 ? CfgK63::ROWS : CfgK32::ROWS;
+    uint64_t NTC = sh.k63 ? CfgK63::NTC : CfgK32::NTC;
+    bulk = false;
+    small = false;
+    uint64_t S = 0, nrows = 0, b0 = t_end;
+    if (sh.fast && len >= 4096) {
+        // bulk region: aligned start b0 >= max(t_begin, p_begin + 64), rows of S bytes
+        uint64_t lo = t_begin > p_begin + 64 ? t_begin : p_begin + 64;
+        const uint64_t a = src_addr + (lo - p_begin);
+        b0 = lo + ((16u - (a & 15u)) & 15u);
+        if (b0 + 256 < t_end) {
+            const uint64_t blen = t_end - b0;
+            // one wave: (SMs - 1) bulk CTAs of ROWS_CTA rows + the edge CTA
+            const uint64_t sms = (uint64_t)(sh.sm_count > 1 ? sh.sm_count - 1 : 1);
+            uint64_t target = sms * ROWS_CTA;
+            if (sh.small_ok && blen <= target * 32) {
+                // rows of < 64 B with the big shape: use the small one, two CTAs per SM
+                // (tools/size_latency.py: faster up to ~4 MiB, slower from ~16 MiB)
+                small = true;
+                ROWS_CTA = CfgSmall::ROWS; NTC = CfgSmall::NTC;
+                target = 2 * sms * ROWS_CTA;
+            }
+            S = (blen + target - 1) / target;
+            S = (S + 63) / 64 * 64;                // an even number of ROUND-byte rounds
+            if (S < 64) S = 64;                    // small inputs: more rows, latency-bound anyway
+            nrows = blen / S;
+            if (nrows > 0 && nrows < (1ull << 31) && S < (1ull << 39) && (b0 - t_begin) <= GS * NTC)
+                bulk = true;
+        }
+    }
+    if (!bulk) {
+        small = false;
+        // generic only: segments of about len / (sm_count * 4 * 256) bytes, >= 256
+        uint64_t seg = 256;
+        const uint64_t want = (uint64_t)sh.sm_count * 4 * GEN_THREADS;
+        if (len / want > seg) seg = (len / want + 63) / 64 * 64;
+        m.head_start = t_begin; m.head_seg = seg;
+        m.n_head = (uint32_t)((len + seg - 1) / seg);
+        m.nrows = 0; m.b0 = t_end; m.S = 0;
+        m.tail_start = t_end; m.tail_seg = seg; m.n_tail = 0;
+        m.nc = 0;
+        m.ngroups = (m.n_head + GEN_THREADS - 1) / GEN_THREADS;
+        return 0;
+    }
+    m.head_start = t_begin; m.head_seg = GS;
+    m.n_head = (uint32_t)((b0 - t_begin + GS - 1) / GS);
+    m.b0 = b0; m.S = S; m.nrows = (uint32_t)nrows;
+    m.tail_start = b0 + nrows * S;
+    const uint64_t tl = t_end - m.tail_start;
+    uint64_t ts = (tl + NTC - 1) / NTC;
+    ts = ts < GS ? GS : (ts + 15) / 16 * 16;
+    m.tail_seg = ts;
+    m.n_tail = (uint32_t)((tl + ts - 1) / ts);
+    m.nc = (uint32_t)((nrows + ROWS_CTA - 1) / ROWS_CTA);
+    m.rows_cta = (uint32_t)ROWS_CTA;
+    m.ngroups = m.nc + 2;
+    return S;
+}
+
+// Per-slot list capacity: twice the expected count of the longest segment + slack.
+uint32_t slot_cap(const SlotMap &m, bool bulk, uint64_t divisor) {
+    uint64_t maxseg = bulk ? m.S : m.head_seg;
+    if (bulk && m.tail_seg > maxseg) maxseg = m.tail_seg;
+    uint64_t cap = 2 * maxseg / divisor + 16;
+    return (uint32_t)(cap > 256 ? 256 : cap);
+}
+
 // Plan candidate detection for window ends [t_begin, t_end) of a job whose bytes start at
 // stream position p_begin (src) with `prefix_len` carried bytes before it.
 int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, const uint8_t *prefix,
@@ -234,76 +313,20 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
     J.min_i = (uint64_t)ctx->p.window - 1u;
     J.c_limit = c_limit;
     SlotMap &m = J.map;
-    m.t_end = t_end;
-    const uint64_t len = t_end > t_begin ? t_end - t_begin : 0;
-    const uint64_t GS = 64;                    // head/tail segment (edge CTA)
-
-    // bulk region: aligned start b0 >= max(t_begin, p_begin + 64), rows of S bytes
-    const bool k63 = ctx->path == SHRED_PATH_K63;
-    uint64_t ROWS_CTA = k63 ? CfgK63::ROWS : CfgK32::ROWS;
-    uint64_t NTC = k63 ? CfgK63::NTC : CfgK32::NTC;
-    const uint64_t ROUND = k63 ? CfgK63::ROUND : CfgK32::ROUND;
-    static_assert(CfgK63::ROUND == CfgSmall::ROUND && CfgK32::ROUND == CfgSmall::ROUND, "round");
-    pl.bulk = false;
-    pl.small = false;
-    uint64_t S = 0, nrows = 0, b0 = t_end;
-    if ((ctx->path == SHRED_PATH_K63 || ctx->path == SHRED_PATH_K32) && len >= 4096) {
-        uint64_t lo = t_begin > p_begin + 64 ? t_begin : p_begin + 64;
-        const uintptr_t a = (uintptr_t)(src + (lo - p_begin));
-        b0 = lo + ((16u - (a & 15u)) & 15u);
-        if (b0 + 256 < t_end) {
-            const uint64_t blen = t_end - b0;
-            // one wave: (SMs - 1) bulk CTAs of ROWS_CTA rows + the edge CTA
-            const uint64_t sms = (uint64_t)(ctx->sm_count > 1 ? ctx->sm_count - 1 : 1);
-            uint64_t target = sms * ROWS_CTA;
-            if (ctx->k1_small_fn && blen <= target * 32) {
-                // rows of < 64 B with the big shape: use the small one, two CTAs per SM
-                // (tools/size_latency.py: faster up to ~4 MiB, slower from ~16 MiB)
-                pl.small = true;
-                ROWS_CTA = CfgSmall::ROWS; NTC = CfgSmall::NTC;
-                target = 2 * sms * ROWS_CTA;
-            }
-            S = (blen + target - 1) / target;
-            S = (S + 63) / 64 * 64;                // an even number of ROUND-byte rounds
-            if (S < 64) S = 64;                    // small inputs: more rows, latency-bound anyway
-            nrows = blen / S;
-            if (nrows > 0 && nrows < (1ull << 31) && S < (1ull << 39) && (b0 - t_begin) <= GS * NTC)
-                pl.bulk = true;
-        }
-    }
-    if (!pl.bulk) {
-        pl.small = false;
-        // generic only: segments of about len / (sm_count * 4 * 256) bytes, >= 256
-        uint64_t seg = 256;
-        const uint64_t want = (uint64_t)ctx->sm_count * 4 * GEN_THREADS;
-        if (len / want > seg) seg = (len / want + 63) / 64 * 64;
-        m.head_start = t_begin; m.head_seg = seg;
-        m.n_head = (uint32_t)((len + seg - 1) / seg);
-        m.nrows = 0; m.b0 = t_end; m.S = 0;
-        m.tail_start = t_end; m.tail_seg = seg; m.n_tail = 0;
-        m.nc = 0;
-        m.ngroups = (m.n_head + GEN_THREADS - 1) / GEN_THREADS;
-    } else {
-        m.head_start = t_begin; m.head_seg = GS;
-        m.n_head = (uint32_t)((b0 - t_begin + GS - 1) / GS);
-        m.b0 = b0; m.S = S; m.nrows = (uint32_t)nrows;
-        m.tail_start = b0 + nrows * S;
-        const uint64_t tl = t_end - m.tail_start;
-        uint64_t ts = (tl + NTC - 1) / NTC;
-        ts = ts < GS ? GS : (ts + 15) / 16 * 16;
-        m.tail_seg = ts;
-        m.n_tail = (uint32_t)((tl + ts - 1) / ts);
-        m.nc = (uint32_t)((nrows + ROWS_CTA - 1) / ROWS_CTA);
-        m.rows_cta = (uint32_t)ROWS_CTA;
-        m.ngroups = m.nc + 2;
+    const MapShape sh{ctx->path == SHRED_PATH_K63 || ctx->path == SHRED_PATH_K32, ctx->path == SHRED_PATH_K63,
+                      ctx->k1_small_fn != nullptr, ctx->sm_count};
+    const uint64_t S = plan_map(sh, (uint64_t)(uintptr_t)src, p_begin, t_begin, t_end, m, pl.bulk, pl.small);
+    if (pl.bulk) {
+        const uint64_t ROUND = CfgK63::ROUND;
+        static_assert(CfgK63::ROUND == CfgSmall::ROUND && CfgK32::ROUND == CfgSmall::ROUND, "round");
         pl.bulk_ctas = m.nc + 1;               // + the edge CTA (head + tail, group sums 0, nc+1)
         // 2-D tensor map [nrows][S] over the bulk bytes
-        cuuint64_t gdim[2] = {(cuuint64_t)S, (cuuint64_t)nrows};
+        cuuint64_t gdim[2] = {(cuuint64_t)S, (cuuint64_t)m.nrows};
         cuuint64_t gstride[1] = {(cuuint64_t)S};
         cuuint32_t box[2] = {(cuuint32_t)ROUND, (cuuint32_t)BOX_ROWS};
         cuuint32_t estr[2] = {1, 1};
         CUresult r = ctx->encode(&pl.tmap, CU_TENSOR_MAP_DATA_TYPE_UINT8, 2,
-                                 (void *)(src + (b0 - p_begin)), gdim, gstride, box, estr,
+                                 (void *)(src + (m.b0 - p_begin)), gdim, gstride, box, estr,
                                  CU_TENSOR_MAP_INTERLEAVE_NONE,
                                  ROUND == 64 ? CU_TENSOR_MAP_SWIZZLE_64B
                                              : (ROUND == 32 ? CU_TENSOR_MAP_SWIZZLE_32B : CU_TENSOR_MAP_SWIZZLE_NONE),
@@ -312,17 +335,12 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
     }
     pl.nslots = m.n_head + m.nrows + m.n_tail;
     if (m.ngroups > (uint32_t)MAX_GROUPS) return fail(ctx, SHRED_EINVAL, "too many slot groups (%u)", m.ngroups);
-    // per-slot list capacity: twice the expected count of the longest segment + slack
-    uint64_t maxseg = pl.bulk ? S : m.head_seg;
-    if (pl.bulk && m.tail_seg > maxseg) maxseg = m.tail_seg;
-    uint64_t cap = 2 * maxseg / ctx->p.divisor + 16;
-    if (cap > 256) cap = 256;
-    J.cap = (uint32_t)cap;
+    J.cap = slot_cap(m, pl.bulk, ctx->p.divisor);
     int rc;
     if ((rc = grow(ctx, ctx->d_counts, ctx->counts_cap, (uint64_t)pl.nslots + 1, "counts"))) return rc;
     if ((rc = grow(ctx, ctx->d_local, ctx->local_cap, (uint64_t)pl.nslots + 1, "local offsets"))) return rc;
     if ((rc = grow(ctx, ctx->d_groups, ctx->groups_cap, (uint64_t)m.ngroups + 1, "group sums"))) return rc;
-    if ((rc = grow(ctx, ctx->d_scratch, ctx->scratch_cap, (uint64_t)pl.nslots * cap + 1, "scratch"))) return rc;
+    if ((rc = grow(ctx, ctx->d_scratch, ctx->scratch_cap, (uint64_t)pl.nslots * J.cap + 1, "scratch"))) return rc;
     J.counts = ctx->d_counts;
     J.local_off = ctx->d_local;
     J.group_sum = ctx->d_groups;
@@ -961,6 +979,22 @@ int shred_index_stats(shred_ctx *ctx, uint64_t stats[4]) {
     DevGuard g(ctx->device);
     CK(cudaDeviceSynchronize(), "index stats sync");
     CK(cudaMemcpy(stats, ctx->index.stats, 32, cudaMemcpyDeviceToHost), "index stats");
+    return SHRED_OK;
+}
+
+int shred_debug_plan(int path, int small_ok, int sm_count, uint64_t src_addr, uint64_t p_begin,
+                     uint64_t t_begin, uint64_t t_end, uint64_t divisor, uint64_t out[16]) {
+    if (!out || t_end < t_begin || t_begin < p_begin || sm_count < 1 || divisor < 2) return SHRED_EINVAL;
+    const MapShape sh{path == SHRED_PATH_K63 || path == SHRED_PATH_K32, path == SHRED_PATH_K63, small_ok != 0,
+                      sm_count};
+    SlotMap m;
+    bool bulk = false, small = false;
+    plan_map(sh, src_addr, p_begin, t_begin, t_end, m, bulk, small);
+    const uint64_t v[16] = {bulk, small, m.head_start, m.head_seg, m.n_head, m.b0, m.S, m.nrows,
+                            m.tail_start, m.tail_seg, m.n_tail, m.nc, m.ngroups, m.rows_cta,
+                            slot_cap(m, bulk, divisor), small ? (uint64_t)CfgSmall::NTC
+                                                              : (uint64_t)(path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC)};
+    for (int i = 0; i < 16; ++i) out[i] = v[i];
     return SHRED_OK;
 }
 
