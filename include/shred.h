@@ -200,6 +200,12 @@ uint64_t shred_launch_count(const shred_ctx *ctx);
    clears the record.  enable = 0 stops recording. */
 int shred_profile(shred_ctx *ctx, int enable);
 
+/* Validate *p as shred_init does (no device needed) and report the kernel path an sm_100a
+   device runs it on (SHRED_PATH_*) and the hot kernel's marker kind (0: '==' on the low word,
+   D = 2^m <= 2^32; 1: '<=' on the low word; 2: '==' by the divisibility test, D = d 2^s with
+   s < 32; -1: generic).  Either out pointer may be NULL.  SHRED_EINVAL for invalid parameters. */
+int shred_check_params(const shred_params *p, int *path_out, int *marker_kind_out);
+
 /* Test hook (no device needed): the slot map planning would use for window ends [t_begin, t_end)
    of a job whose bytes start at stream position p_begin at address src_addr, for kernel path
    `path` (SHRED_PATH_*), with (small_ok) or without the small-input launch shape, on sm_count SMs.

@@ -207,11 +207,29 @@ int validate(const shred_params *p, shred_ctx *ctx) {
     if (p->window < 1 || p->window > 4096) return fail(ctx, SHRED_EINVAL, "window %u not in 1..4096", p->window);
     if (p->marker > SHRED_MARKER_LE) return fail(ctx, SHRED_EINVAL, "marker must be SHRED_MARKER_EQ or SHRED_MARKER_LE");
     if (p->divisor < 2) return fail(ctx, SHRED_EINVAL, "divisor must be >= 2");
-    if (k < 63 && p->divisor > (1ull << k)) return fail(ctx, SHRED_EINVAL, "divisor exceeds 2^deg(poly)");
+    if (p->divisor > (1ull << k)) return fail(ctx, SHRED_EINVAL, "divisor exceeds 2^deg(poly)");
     if (p->magic >= p->divisor) return fail(ctx, SHRED_EINVAL, "magic must be < divisor");
     if (p->max_size && p->max_size < (p->min_size > 1 ? p->min_size : 1))
         return fail(ctx, SHRED_EINVAL, "max_size must be >= max(min_size, 1)");
     return SHRED_OK;
+}
+
+// Kernel path and marker kind for valid parameters on an sm_100a device.  The hot kernel takes
+// any w <= 64 (w % 16 != 0: funnel-shifted pops), and D = 2^m <= 2^32 with either marker set on
+// the low word, or the '==' marker with any D = d 2^s (s < 32) by the divisibility test on the
+// full state (MK_DIV).  u64 state: deg 33..63 (top byte by mulhi, or a funnel shift for k <= 40);
+// u32 state: deg 9..32.  Everything else: the generic loop.
+int select_path(const shred_params *p, int *mk) {
+    const int k = deg64(p->poly);
+    const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
+    const bool fast_w = p->window >= 1 && p->window <= 64;
+    if (pow2 && p->divisor <= (1ull << 32)) *mk = p->marker == SHRED_MARKER_LE ? MK_LE : MK_EQ;
+    else if (p->marker == SHRED_MARKER_EQ && __builtin_ctzll(p->divisor) < 32) *mk = MK_DIV;
+    else *mk = -1;
+    const bool fast = fast_w && *mk >= 0;
+    if (k >= 33 && k <= 63 && fast) return SHRED_PATH_K63;
+    if (k >= 9 && k <= 32 && fast) return SHRED_PATH_K32;
+    return SHRED_PATH_GENERIC;
 }
 
 // ---------------------------------------------------------------------------- job planning
@@ -574,20 +592,7 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     ctx->dp.divisor = p->divisor;
     ctx->dp.pow2 = (p->divisor & (p->divisor - 1)) == 0 ? 1u : 0u;
     ctx->dp.marker = p->marker;
-    const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
-    // the hot kernel: any w <= 64 (w % 16 != 0: funnel-shifted pops); D = 2^m <= 2^32 with either
-    // marker set on the low word, or the '==' marker with any D = d 2^s (s < 32) by the
-    // divisibility test on the full state (MK_DIV)
-    const bool fast_w = p->window >= 1 && p->window <= 64;
-    if (pow2 && p->divisor <= (1ull << 32)) ctx->mk = p->marker == SHRED_MARKER_LE ? MK_LE : MK_EQ;
-    else if (p->marker == SHRED_MARKER_EQ && __builtin_ctzll(p->divisor) < 32) ctx->mk = MK_DIV;
-    else ctx->mk = -1;
-    const bool fast = fast_w && ctx->mk >= 0;
-    // u64-state kernel: deg 33..63 (t = mulhi(f_hi, 2^(72-k)), or a funnel shift for k <= 40);
-    // u32-state kernel: deg 9..32
-    if (k >= 33 && k <= 63 && fast) ctx->path = SHRED_PATH_K63;
-    else if (k >= 9 && k <= 32 && fast) ctx->path = SHRED_PATH_K32;
-    else ctx->path = SHRED_PATH_GENERIC;
+    ctx->path = select_path(p, &ctx->mk);
     if (major != 10) ctx->path = SHRED_PATH_GENERIC;   // the TMA kernels are built for sm_100a only
 
     // ---- tables (PAPER.md: shift one byte in, one byte out)
@@ -979,6 +984,16 @@ int shred_index_stats(shred_ctx *ctx, uint64_t stats[4]) {
     DevGuard g(ctx->device);
     CK(cudaDeviceSynchronize(), "index stats sync");
     CK(cudaMemcpy(stats, ctx->index.stats, 32, cudaMemcpyDeviceToHost), "index stats");
+    return SHRED_OK;
+}
+
+int shred_check_params(const shred_params *p, int *path_out, int *marker_kind_out) {
+    const int rc = validate(p, nullptr);
+    if (rc) return rc;
+    int mk = -1;
+    const int path = select_path(p, &mk);
+    if (path_out) *path_out = path;
+    if (marker_kind_out) *marker_kind_out = mk;
     return SHRED_OK;
 }
 
