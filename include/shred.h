@@ -80,8 +80,8 @@ enum {
                                either D = 2^m <= 2^32 with either marker set, or the '==' marker
                                with any D = d 2^s, s < 32 (divisibility test on the full state):
                                u64 state, TMA-staged, smem LDS.64 tables                        */
-    SHRED_PATH_K32     = 2, /* deg(P) in 9..32, same w / D / marker conditions: u32 state, LDS.32 */
-    SHRED_PATH_GENERIC = 3  /* any other valid parameters (deg 8, w > 64, the '<=' marker with D
+    SHRED_PATH_K32     = 2, /* deg(P) in 8..32, same w / D / marker conditions: u32 state, LDS.32 */
+    SHRED_PATH_GENERIC = 3  /* any other valid parameters (w > 64, the '<=' marker with D
                                not a power of two, D with 2^32 | D): byte-at-a-time             */
 };
 

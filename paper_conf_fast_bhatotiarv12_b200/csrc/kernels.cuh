@@ -41,7 +41,7 @@
 namespace shred {
 
 // K63: u64 state, deg 41..63; K40: u64 state, deg 33..40; K32: u32 state, deg 9..32;
-// K32B: u32 state, deg 16/24/32 (whole-byte top byte)
+// K32B: u32 state, deg 8/16/24/32 (whole-byte top byte)
 enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3, MODE_K32B = 4, MODE_K40 = 5 };
 
 constexpr int STAGES      = 4;                 // TMA ring depth

@@ -89,7 +89,7 @@ void byte_times_xpow(uint64_t P, int k, uint64_t e, uint64_t out[256]) {
 #define SHRED_PDL 1       // 0: plain stream serialization (A/B)
 #endif
 #ifndef SHRED_BYTEIDX
-#define SHRED_BYTEIDX 1   // deg 16/24/32: PRMT table index (MODE_K32B); 0: IMAD index (MODE_K32)
+#define SHRED_BYTEIDX 1   // deg 8/16/24/32: PRMT table index (MODE_K32B); 0: IMAD index (MODE_K32)
 #endif
 typedef CUresult (*EncodeTiledFn)(CUtensorMap *, CUtensorMapDataType, cuuint32_t, void *,
                                   const cuuint64_t *, const cuuint64_t *, const cuuint32_t *,
@@ -218,7 +218,8 @@ int validate(const shred_params *p, shred_ctx *ctx) {
 // any w <= 64 (w % 16 != 0: funnel-shifted pops), and D = 2^m <= 2^32 with either marker set on
 // the low word, or the '==' marker with any D = d 2^s (s < 32) by the divisibility test on the
 // full state (MK_DIV).  u64 state: deg 33..63 (top byte by mulhi, or a funnel shift for k <= 40);
-// u32 state: deg 9..32.  Everything else: the generic loop.
+// u32 state: deg 9..32, and 8 (its top byte is the whole state: the PRMT byte index of
+// MODE_K32B).  Everything else: the generic loop.
 int select_path(const shred_params *p, int *mk) {
     const int k = deg64(p->poly);
     const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
@@ -228,7 +229,7 @@ int select_path(const shred_params *p, int *mk) {
     else *mk = -1;
     const bool fast = fast_w && *mk >= 0;
     if (k >= 33 && k <= 63 && fast) return SHRED_PATH_K63;
-    if (k >= 9 && k <= 32 && fast) return SHRED_PATH_K32;
+    if ((k >= 9 || (k == 8 && SHRED_BYTEIDX)) && k <= 32 && fast) return SHRED_PATH_K32;
     return SHRED_PATH_GENERIC;
 }
 
@@ -388,7 +389,7 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         BulkConst K;
         // top byte t = f >> (k-8): u64 state mulhi(f_hi, 2^(72-k)); u32 state mulhi(f, 2^(40-k))
         K.mhi = ctx->path == SHRED_PATH_K63 ? (ctx->k >= 41 ? (1u << (72 - ctx->k)) : (uint32_t)(ctx->k - 8))
-                                            : (1u << (40 - ctx->k));
+                                            : (ctx->k >= 9 ? (1u << (40 - ctx->k)) : 0u);   // deg 8: byte index
         const uint32_t e = (uint32_t)(16 * ((ctx->p.window + 15) / 16) - ctx->p.window);
         K.fu = e / 4;
         K.fsel = 0x3210u + 0x1111u * (e % 4);
@@ -645,7 +646,7 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fn, cudaEnableDefault, &q) != cudaSuccess || !fn)
             return bail(SHRED_ECUDA);
         ctx->encode = (EncodeTiledFn)fn;
-        const bool byteidx = SHRED_BYTEIDX && ctx->path == SHRED_PATH_K32 && (k == 16 || k == 24 || k == 32);
+        const bool byteidx = SHRED_BYTEIDX && ctx->path == SHRED_PATH_K32 && (k == 8 || k == 16 || k == 24 || k == 32);
         const int wch = (int)((p->window + 15) / 16);
         const bool funnel = p->window % 16 != 0;
         ctx->k1_fn = pick_k1(k, byteidx, wch, ctx->mk, funnel);

@@ -116,8 +116,7 @@ def test_launch_shapes_around_small_threshold(pkg, poly, n):
 
 def test_generic_path_variants(pkg):
     for p in (pkg.Params(window=65), pkg.Params(window=80, divisor=256, magic=7, marker=1),
-              pkg.Params(poly=0x11D, window=24, divisor=128, magic=5, marker=1),
-              pkg.Params(poly=0x11D, window=7, divisor=64, magic=9),
+              pkg.Params(poly=0x11D, window=70, divisor=128, magic=5, marker=1),
               pkg.Params(divisor=3000, magic=2999, marker=1),
               pkg.Params(divisor=1 << 40, magic=12345)):
         ch = pkg.Chunker(p)
@@ -406,14 +405,14 @@ def _dense_irreducible(deg, seed):
 
 @pytest.mark.parametrize("deg", [8, 9, 12, 16, 24, 31, 32, 33, 40, 41, 48, 57, 62, 63])
 def test_polynomial_degrees(pkg, deg):
-    """Any degree: u32-state fast kernel for 9..32, u64-state for 33..63 (top byte by mulhi for
-    41..63, by a funnel shift for 33..40), generic for 8 (T tables with the (t << k) cancel term);
-    dense random irreducible P, bit-exact."""
+    """Any degree: u32-state fast kernel for 8..32 (8, 16, 24, 32: the top byte is a whole byte,
+    PRMT index), u64-state for 33..63 (top byte by mulhi for 41..63, by a funnel shift for
+    33..40); T tables with the (t << k) cancel term; dense random irreducible P, bit-exact."""
     P = _dense_irreducible(deg, deg)
     D = 1 << min(10, deg - 1)
     p = pkg.Params(poly=P, divisor=D, magic=D // 3)
     ch = pkg.Chunker(p)
-    assert ch.path == ("k32" if 9 <= deg <= 32 else "k63" if deg >= 33 else "generic")
+    assert ch.path == ("k32" if deg <= 32 else "k63")
     check_chunk(ch, synthgen.random_bytes(deg, (2 << 20) + 123), offset=deg % 16)
 
 
@@ -440,3 +439,22 @@ def test_divisor_range_with_planted_magic(pkg, poly, log2d):
             exp = np.nonzero((fps % np.uint64(D)) == np.uint64(r))[0].astype(np.uint64) + np.uint64(op.window)
             exp = exp[exp < data.size]
             assert np.array_equal(got, exp) and got.size >= 1
+
+
+@pytest.mark.parametrize("window", [1, 7, 16, 47, 48, 64])
+@pytest.mark.parametrize("marker", [0, 1])
+def test_degree8_fast_path(pkg, window, marker):
+    """deg P = 8: the whole state is the top byte, so the u32 kernel's PRMT byte index applies
+    (f <- ((f << 8) | b) ^ T[f] ^ U[o], T carrying the t << 8 cancel term); D <= 2^8.  Sizes on
+    both launch shapes (1 MiB: small; 6 MiB: big), an unaligned base, and the streaming carry."""
+    P = 0x11D
+    for D, r in ((256, 0x78 if not marker else 9), (64, 5), (2, 1 if not marker else 0)):
+        p = pkg.Params(poly=P, window=window, divisor=D, magic=r, marker=marker)
+        ch = pkg.Chunker(p)
+        assert ch.path == "k32"
+        data = synthgen.random_bytes(800 + window + D, (1 << 20) + 77 if D != 256 else (6 << 20) + 5)
+        check_chunk(ch, data, offset=window % 16)
+    ch = pkg.Chunker(pkg.Params(poly=P, window=window, divisor=256, magic=3, marker=marker))
+    data = synthgen.random_bytes(900 + window, (2 << 20) + 11)
+    n = data.size
+    assert np.array_equal(_feed_all(ch, data, [n // 2, 1, n - n // 2 - 1], True), oracle.chunk(data, oparams(ch.params)))

@@ -76,7 +76,7 @@ def test_parameter_ranges(check):
     (dict(divisor=1 << 32, magic=7), K63, MK_EQ), (dict(divisor=1 << 33, magic=7), GENERIC, MK_NONE),
     (dict(divisor=3 << 32, magic=7), GENERIC, MK_NONE), (dict(divisor=10000, magic=7, marker=1), GENERIC, MK_NONE),
     (dict(poly=0x104C11DB7), K32, MK_EQ), (dict(poly=0x104C11DB7, divisor=10000, magic=3), K32, MK_DIV),
-    (dict(poly=0x11D, divisor=64, magic=1), GENERIC, MK_EQ),                     # degree 8
+    (dict(poly=0x11D, divisor=64, magic=1), K32, MK_EQ),                         # degree 8: byte index
     (dict(poly=(1 << 40) | 0x39, divisor=1024, magic=5), K63, MK_EQ),            # degree 40: u64 state
 ])
 def test_path_table(check, kw, path, mk):
