@@ -76,13 +76,11 @@ enum { SHRED_MARKER_EQ = 0, SHRED_MARKER_LE = 1 };
 
 /* Kernel paths the ctx selected for its parameters (shred_path). */
 enum {
-    SHRED_PATH_K63     = 1, /* deg(P) in 33..63 (the paper's reading: 63), 1 <= w <= 64, and
-                               either D = 2^m <= 2^32 with either marker set, or the '==' marker
-                               with any D = d 2^s, s < 32 (divisibility test on the full state):
-                               u64 state, TMA-staged, smem LDS.64 tables                        */
+    SHRED_PATH_K63     = 1, /* deg(P) in 33..63 (the paper's reading: 63), 1 <= w <= 64, any
+                               valid D and marker set (marker kinds below): u64 state,
+                               TMA-staged, smem LDS.64 tables                                   */
     SHRED_PATH_K32     = 2, /* deg(P) in 8..32, same w / D / marker conditions: u32 state, LDS.32 */
-    SHRED_PATH_GENERIC = 3  /* any other valid parameters (w > 64, the '<=' marker with D
-                               not a power of two, D with 2^32 | D): byte-at-a-time             */
+    SHRED_PATH_GENERIC = 3  /* any other valid parameters (w > 64): byte-at-a-time             */
 };
 
 /* Fill *p with the paper defaults (readings Q1, Q5, Q6, Q15): P = 0xbfe6b8a5bf378d83, w = 48,
@@ -203,7 +201,9 @@ int shred_profile(shred_ctx *ctx, int enable);
 /* Validate *p as shred_init does (no device needed) and report the kernel path an sm_100a
    device runs it on (SHRED_PATH_*) and the hot kernel's marker kind (0: '==' on the low word,
    D = 2^m <= 2^32; 1: '<=' on the low word; 2: '==' by the divisibility test, D = d 2^s with
-   s < 32; -1: generic).  Either out pointer may be NULL.  SHRED_EINVAL for invalid parameters. */
+   s < 32; 3: either marker set on the remainder f - floor(f / D) D, the quotient by a 64-bit
+   multiply-high, for every other D).  Either out pointer may be NULL.  SHRED_EINVAL for invalid
+   parameters. */
 int shred_check_params(const shred_params *p, int *path_out, int *marker_kind_out);
 
 /* Test hook (no device needed): the slot map planning would use for window ends [t_begin, t_end)

@@ -39,6 +39,7 @@ K1Fn pick_mode(int wch, int mk, bool fn) {
         case MK_EQ: return pick_w<MODE, C, MK_EQ>(wch, fn);
         case MK_LE: return pick_w<MODE, C, MK_LE>(wch, fn);
         case MK_DIV: return pick_w<MODE, C, MK_DIV>(wch, fn);
+        case MK_REM: return pick_w<MODE, C, MK_REM>(wch, fn);
         default: return nullptr;
     }
 }

@@ -433,6 +433,12 @@ struct BulkCtx {
     uint64_t dinv;      // d^-1 mod 2^64 (d = the odd part of D)
     uint64_t dlim;      // floor((2^64 - 1) / D)
     uint32_t dsh;       // s
+    // MK_REM (any other D, either marker set): rem = f - q D with q = floor(f / D) =
+    // mulhi64(f, rm) >> rsh2 (Granlund-Montgomery, exact for f < 2^63: rm = ceil(2^(63+l) / D),
+    // l = ceil(log2 D), rsh2 = l - 1); marker iff (rem - rlo) mod 2^64 <= rspan
+    // ('==': rlo = r, rspan = 0; '<=': rlo = 0, rspan = r).
+    uint64_t rm, rd, rlo, rspan;
+    uint32_t rsh2;
 };
 
 // One byte step, u64 state (deg P = k in 41..63; the paper's reading k = 63), f = fh:fl < 2^k:
@@ -507,7 +513,9 @@ template <> struct State<MODE_K32B> {
 // Marker kinds of the hot kernel: MK_EQ / MK_LE: D = 2^m <= 2^32, "fp mod D == r" / "<= r"
 // (L447-L451 / L249-L251) on the low word; MK_DIV: "fp mod D == r" for a D that is not a power of
 // two (Q8: the integer remainder of the fingerprint's value), on the full state.
-enum { MK_EQ = 0, MK_LE = 1, MK_DIV = 2 };
+// MK_REM: either marker set for any D the other kinds do not take ('<=' with D not a power of two,
+// D with 2^32 | D): the remainder itself by a multiply-high division.
+enum { MK_EQ = 0, MK_LE = 1, MK_DIV = 2, MK_REM = 3 };
 // marker test: (f mod D) == r  <=>  (f_lo << (32-m)) == (r << (32-m))   (D = 2^m <= 2^32)
 __device__ __forceinline__ bool is_marker(uint32_t lo, const BulkCtx &c) { return lo * c.tmul == c.rsh; }
 // m | BIT if marker else m: ISETP + predicated LOP3 (the PTX predication survives ptxas).
@@ -534,6 +542,14 @@ __device__ __forceinline__ uint32_t or_if_div(uint32_t m, uint64_t f, const Bulk
     return rot <= c.dlim ? (m | BIT) : m;
 }
 
+// MK_REM: f mod D by q = mulhi64(f, rm) >> rsh2, rem = f - q D; one window test (rem - rlo) <= rspan.
+template <uint32_t BIT>
+__device__ __forceinline__ uint32_t or_if_rem(uint32_t m, uint64_t f, const BulkCtx &c) {
+    const uint64_t q = __umul64hi(f, c.rm) >> c.rsh2;
+    const uint64_t x = f - q * c.rd - c.rlo;
+    return x <= c.rspan ? (m | BIT) : m;
+}
+
 struct SlotOut {
     uint64_t *lst; uint32_t cnt; uint32_t cap;
 };
@@ -558,6 +574,7 @@ static __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t
 #else
 #define SHRED_MARK(ch, q)                                                                   \
     m[ch] = (MK == MK_DIV) ? or_if_div<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
+          : (MK == MK_REM) ? or_if_rem<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
                            : or_if_marker<(1u << (4 * J + q)), MK>(m[ch], st[ch].low(), c);
 #endif
 template <int MODE, int CH, bool TEST, int J, int MK>
@@ -616,6 +633,8 @@ struct BulkConst {
     uint32_t mhi, m256, tmul, rsh, tsel;
     uint64_t dc, dinv, dlim;   // MK_DIV constants (BulkCtx)
     uint32_t dsh;
+    uint64_t rm, rd, rlo, rspan;   // MK_REM constants (BulkCtx)
+    uint32_t rsh2;
     uint32_t fu, fsel;  // FN windows (w % 16 != 0): e = 16*ceil(w/16) - w = 4*fu + v, fsel = PRMT
                         // selector of bytes v..v+3 (0x3210 + 0x1111 v)
 };
@@ -755,6 +774,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     }
     c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh; c.tsel = K.tsel;
     c.dc = K.dc; c.dinv = K.dinv; c.dlim = K.dlim; c.dsh = K.dsh;
+    c.rm = K.rm; c.rd = K.rd; c.rlo = K.rlo; c.rspan = K.rspan; c.rsh2 = K.rsh2;
 
     bool act[CH];
     uint64_t pos0[CH];

@@ -216,17 +216,17 @@ int validate(const shred_params *p, shred_ctx *ctx) {
 
 // Kernel path and marker kind for valid parameters on an sm_100a device.  The hot kernel takes
 // any w <= 64 (w % 16 != 0: funnel-shifted pops), and D = 2^m <= 2^32 with either marker set on
-// the low word, or the '==' marker with any D = d 2^s (s < 32) by the divisibility test on the
-// full state (MK_DIV).  u64 state: deg 33..63 (top byte by mulhi, or a funnel shift for k <= 40);
+// the low word, the '==' marker with any D = d 2^s (s < 32) by the divisibility test on the
+// full state (MK_DIV), and every other D by the remainder itself (MK_REM).  u64 state: deg 33..63 (top byte by mulhi, or a funnel shift for k <= 40);
 // u32 state: deg 9..32, and 8 (its top byte is the whole state: the PRMT byte index of
-// MODE_K32B).  Everything else: the generic loop.
+// MODE_K32B).  Windows > 64: the generic loop.
 int select_path(const shred_params *p, int *mk) {
     const int k = deg64(p->poly);
     const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
     const bool fast_w = p->window >= 1 && p->window <= 64;
     if (pow2 && p->divisor <= (1ull << 32)) *mk = p->marker == SHRED_MARKER_LE ? MK_LE : MK_EQ;
     else if (p->marker == SHRED_MARKER_EQ && __builtin_ctzll(p->divisor) < 32) *mk = MK_DIV;
-    else *mk = -1;
+    else *mk = MK_REM;
     const bool fast = fast_w && *mk >= 0;
     if (k >= 33 && k <= 63 && fast) return SHRED_PATH_K63;
     if ((k >= 9 || (k == 8 && SHRED_BYTEIDX)) && k <= 32 && fast) return SHRED_PATH_K32;
@@ -385,7 +385,7 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
             ctx->prof_bytes += (pl.J.map.t_end - pl.J.map.head_start);
             CK(cudaEventRecord(e0, st), "profile record");
         }
-        const int m = ctx->mk == MK_DIV ? 0 : 32 - (int)__builtin_ctzll(ctx->p.divisor);   // D = 2^(32-m)
+        const int m = ctx->mk >= MK_DIV ? 0 : 32 - (int)__builtin_ctzll(ctx->p.divisor);   // D = 2^(32-m)
         BulkConst K;
         // top byte t = f >> (k-8): u64 state mulhi(f_hi, 2^(72-k)); u32 state mulhi(f, 2^(40-k))
         K.mhi = ctx->path == SHRED_PATH_K63 ? (ctx->k >= 41 ? (1u << (72 - ctx->k)) : (uint32_t)(ctx->k - 8))
@@ -403,6 +403,13 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
             uint64_t inv = d;
             for (int it = 0; it < 5; ++it) inv *= 2u - d * inv;
             K.dc = D - ctx->p.magic; K.dinv = inv; K.dlim = ~0ull / D; K.dsh = sh;
+            // MK_REM: l = ceil(log2 D) in 1..63; rm = ceil(2^(63+l) / D) < 2^64 (D > 2^(l-1), or
+            // D = 2^l and rm = 2^63); q = mulhi(f, rm) >> (l-1) = floor(f / D) for every f < 2^63
+            const int l = 64 - __builtin_clzll(D - 1);
+            const unsigned __int128 num = (unsigned __int128)1 << (63 + l);
+            K.rm = (uint64_t)((num + D - 1) / D); K.rd = D; K.rsh2 = (uint32_t)(l - 1);
+            K.rlo = ctx->p.marker == SHRED_MARKER_LE ? 0 : ctx->p.magic;
+            K.rspan = ctx->p.marker == SHRED_MARKER_LE ? ctx->p.magic : 0;
         }
         K.tsel = 0x5504u | ((uint32_t)((ctx->k - 8) / 8) << 4);         // byte (k-8)/8 -> bits 8..15
         int smem = ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM;

@@ -101,8 +101,8 @@ def test_init_validation_and_paths(pkg):
     with pytest.raises(pkg.ShredError):
         pkg.Chunker(pkg.Params(marker=2))
     assert pkg.Chunker(pkg.Params(divisor=3000)).path == 'k63'
-    assert pkg.Chunker(pkg.Params(divisor=3000, magic=5, marker=1)).path == 'generic'
-    assert pkg.Chunker(pkg.Params(divisor=3 << 32)).path == 'generic'
+    assert pkg.Chunker(pkg.Params(divisor=3000, magic=5, marker=1)).path == 'k63'   # MK_REM
+    assert pkg.Chunker(pkg.Params(divisor=3 << 32)).path == 'k63'                   # MK_REM
     assert pkg.Chunker(pkg.Params()).path == "k63"
     assert pkg.Chunker(pkg.Params(poly=0x104C11DB7)).path == "k32"
     assert pkg.Chunker(pkg.Params(window=47)).path == "k63"

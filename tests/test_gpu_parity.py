@@ -117,8 +117,8 @@ def test_launch_shapes_around_small_threshold(pkg, poly, n):
 def test_generic_path_variants(pkg):
     for p in (pkg.Params(window=65), pkg.Params(window=80, divisor=256, magic=7, marker=1),
               pkg.Params(poly=0x11D, window=70, divisor=128, magic=5, marker=1),
-              pkg.Params(divisor=3000, magic=2999, marker=1),
-              pkg.Params(divisor=1 << 40, magic=12345)):
+              pkg.Params(window=100, divisor=3000, magic=2999, marker=1),
+              pkg.Params(window=65, divisor=1 << 40, magic=12345)):
         ch = pkg.Chunker(p)
         assert ch.path == "generic"
         check_chunk(ch, synthgen.random_bytes(11, 300000))
@@ -324,14 +324,14 @@ def test_bounded_adversarial_stream(pkg):
 def test_marker_le_and_non_pow2_divisor(pkg):
     """Divisors that are not powers of two (Q8: the integer remainder of the fingerprint's value):
     the '==' marker runs on the hot kernel (divisibility test on the full state), the
-    "value mod p <= constant" set (L249-L251) on the generic path; bit-exact vs the oracle,
-    bounded mode on top."""
+    "value mod p <= constant" set (L249-L251) too (the remainder by a multiply-high quotient);
+    bit-exact vs the oracle, bounded mode on top."""
     data = synthgen.random_bytes(31, (2 << 20) + 77)
     for p, path in ((pkg.Params(divisor=10000, magic=1234), "k63"),
-                    (pkg.Params(divisor=12345, magic=3, marker=1), "generic"),
+                    (pkg.Params(divisor=12345, magic=3, marker=1), "k63"),
                     (pkg.Params(divisor=3, magic=0), "k63"),
                     (pkg.Params(divisor=3000, magic=2999, min_size=1000, max_size=20000), "k63"),
-                    (pkg.Params(divisor=5000, magic=4, marker=1, min_size=1000, max_size=20000), "generic")):
+                    (pkg.Params(divisor=5000, magic=4, marker=1, min_size=1000, max_size=20000), "k63")):
         ch = pkg.Chunker(p)
         assert ch.path == path
         check_chunk(ch, data)
@@ -433,7 +433,7 @@ def test_divisor_range_with_planted_magic(pkg, poly, log2d):
         r = int(fps[k]) % D
         p = pkg.Params(poly=poly, divisor=D, magic=r)
         ch = pkg.Chunker(p)
-        assert ch.path == ("generic" if log2d > 32 else "k63" if poly == LBFS else "k32")
+        assert ch.path == ("k63" if poly == LBFS else "k32")
         got = check_chunk(ch, data)
         if log2d >= 20:
             exp = np.nonzero((fps % np.uint64(D)) == np.uint64(r))[0].astype(np.uint64) + np.uint64(op.window)
@@ -458,3 +458,40 @@ def test_degree8_fast_path(pkg, window, marker):
     data = synthgen.random_bytes(900 + window, (2 << 20) + 11)
     n = data.size
     assert np.array_equal(_feed_all(ch, data, [n // 2, 1, n - n // 2 - 1], True), oracle.chunk(data, oparams(ch.params)))
+
+
+@pytest.mark.parametrize("poly", [LBFS, 0x104C11DB7, 0x20000005, None, 0x11D])   # K63, K32B, K32, K40, deg 8
+@pytest.mark.parametrize("D", [3, 255, 10000, 3 << 20, (1 << 32) - 1, 1 << 33, 3 << 32, (1 << 40) + 1,
+                               12345678901, (1 << 62) + 12345, 1 << 63])
+def test_remainder_marker_hot_kernel(pkg, poly, D):
+    """MK_REM: the '<=' set (L249-L251) with any D, and '==' where 2^32 | D, on the hot kernel:
+    rem = f - q D with q = mulhi64(f, ceil(2^(63+l) / D)) >> (l-1), l = ceil(log2 D) (exact for
+    f < 2^63).  r is planted from real window fingerprints (oracle R2): for '<=' the smallest
+    residue of the first 4096 windows (about one hit per 4096 B), for '==' one residue; a funnel
+    window (w = 47) and a streaming feed too."""
+    if poly is None:
+        poly = (1 << 40) | 0x39
+    deg = poly.bit_length() - 1
+    if not oracle.is_irreducible(poly):
+        pytest.skip("not irreducible")
+    if D > (1 << deg):
+        pytest.skip("D > 2^deg")
+    data = synthgen.random_bytes(900 + (D % 97), (3 << 20) + 41)
+    for w in (48, 47):
+        op = oracle.Params(poly=poly, window=w)
+        fps = oracle.window_fps(data, op)
+        res = fps[:4096] % np.uint64(D)
+        cases = [(1, int(res.min()))]
+        if D % (1 << 32) == 0 or (D & (D - 1)) != 0:
+            cases.append((0, int(fps[fps.size // 3]) % D))
+        for marker, r in cases:
+            p = pkg.Params(poly=poly, window=w, divisor=D, magic=r, marker=marker)
+            ch = pkg.Chunker(p)
+            assert ch.path == ("k63" if deg >= 33 else "k32")
+            got = check_chunk(ch, data, offset=w % 16)
+            hit = (fps % np.uint64(D)) <= np.uint64(r) if marker else (fps % np.uint64(D)) == np.uint64(r)
+            exp = np.nonzero(hit)[0].astype(np.uint64) + np.uint64(w)
+            assert np.array_equal(got, exp[exp < data.size]) and got.size >= 1
+    ch = pkg.Chunker(pkg.Params(poly=poly, window=47, divisor=D, magic=r, marker=marker))
+    n = data.size
+    assert np.array_equal(_feed_all(ch, data, [n // 3, 5, n - n // 3 - 5], True), oracle.chunk(data, oparams(ch.params)))

@@ -15,7 +15,7 @@ import pytest
 import oracle
 
 K63, K32, GENERIC = 1, 2, 3
-MK_EQ, MK_LE, MK_DIV, MK_NONE = 0, 1, 2, -1
+MK_EQ, MK_LE, MK_DIV, MK_REM = 0, 1, 2, 3
 LBFS = 0xBFE6B8A5BF378D83
 
 
@@ -73,8 +73,10 @@ def test_parameter_ranges(check):
     (dict(window=47), K63, MK_EQ), (dict(window=64), K63, MK_EQ), (dict(window=1), K63, MK_EQ),
     (dict(window=65), GENERIC, MK_EQ), (dict(window=47, marker=1, magic=1), K63, MK_LE),
     (dict(divisor=10000, magic=7), K63, MK_DIV), (dict(divisor=3 << 31, magic=7), K63, MK_DIV),
-    (dict(divisor=1 << 32, magic=7), K63, MK_EQ), (dict(divisor=1 << 33, magic=7), GENERIC, MK_NONE),
-    (dict(divisor=3 << 32, magic=7), GENERIC, MK_NONE), (dict(divisor=10000, magic=7, marker=1), GENERIC, MK_NONE),
+    (dict(divisor=1 << 32, magic=7), K63, MK_EQ), (dict(divisor=1 << 33, magic=7), K63, MK_REM),
+    (dict(divisor=3 << 32, magic=7), K63, MK_REM), (dict(divisor=10000, magic=7, marker=1), K63, MK_REM),
+    (dict(divisor=1 << 40, magic=7, marker=1), K63, MK_REM), (dict(window=65, divisor=10000, magic=7, marker=1), GENERIC, MK_REM),
+    (dict(poly=0x104C11DB7, divisor=1000, magic=999, marker=1), K32, MK_REM),
     (dict(poly=0x104C11DB7), K32, MK_EQ), (dict(poly=0x104C11DB7, divisor=10000, magic=3), K32, MK_DIV),
     (dict(poly=0x11D, divisor=64, magic=1), K32, MK_EQ),                         # degree 8: byte index
     (dict(poly=(1 << 40) | 0x39, divisor=1024, magic=5), K63, MK_EQ),            # degree 40: u64 state

@@ -12,7 +12,12 @@ cases = {"paper (k63 eq pow2)": pkg.Params(), "k32": pkg.Params(poly=0x104C11DB7
          "w=64": pkg.Params(window=64), "D=10000": pkg.Params(divisor=10000, magic=7),
          "deg 40": pkg.Params(poly=0x10000000039), "w=47": pkg.Params(window=47),
          "w=31 k32": pkg.Params(poly=0x104C11DB7, window=31), "w=5": pkg.Params(window=5),
-         "w=65": pkg.Params(window=65), "w=47 le": pkg.Params(window=47, divisor=8192, magic=1, marker=1)}
+         "w=65": pkg.Params(window=65), "w=47 le": pkg.Params(window=47, divisor=8192, magic=1, marker=1),
+         "deg 8": pkg.Params(poly=0x11D, divisor=256, magic=7),
+         "D=10000 le": pkg.Params(divisor=10000, magic=1, marker=1),
+         "D=2^40 le": pkg.Params(divisor=1 << 40, magic=1 << 27, marker=1),
+         "D=3*2^32 eq": pkg.Params(divisor=3 << 32, magic=12345),
+         "k32 D=1000 le": pkg.Params(poly=0x104C11DB7, divisor=1000, magic=0, marker=1)}
 out = torch.empty(n // 256, dtype=torch.int64, device="cuda"); nn = torch.zeros(1, dtype=torch.int64, device="cuda")
 for name, p in cases.items():
     try:
