@@ -550,6 +550,17 @@ __device__ __forceinline__ uint32_t or_if_rem(uint32_t m, uint64_t f, const Bulk
     return x <= c.rspan ? (m | BIT) : m;
 }
 
+// MK_REM, u32 state (deg <= 32, f < 2^32, so D <= 2^32 and MK_REM has D < 2^32, l <= 32): the
+// same quotient from two 32x32 -> 64 products, h = (f rm) >> 32 = f rm_hi + hi32(f rm_lo) and
+// q = hi32(h) >> (l - 1); rem < 2^32, so the rest runs in 32 bits.
+template <uint32_t BIT>
+__device__ __forceinline__ uint32_t or_if_rem32(uint32_t m, uint32_t f, const BulkCtx &c) {
+    const uint64_t h = (uint64_t)f * (uint32_t)(c.rm >> 32) + __umulhi(f, (uint32_t)c.rm);
+    const uint32_t q = (uint32_t)(h >> 32) >> c.rsh2;
+    const uint32_t x = f - q * (uint32_t)c.rd - (uint32_t)c.rlo;
+    return x <= (uint32_t)c.rspan ? (m | BIT) : m;
+}
+
 struct SlotOut {
     uint64_t *lst; uint32_t cnt; uint32_t cap;
 };
@@ -574,6 +585,8 @@ static __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t
 #else
 #define SHRED_MARK(ch, q)                                                                   \
     m[ch] = (MK == MK_DIV) ? or_if_div<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
+          : (MK == MK_REM && (MODE == MODE_K32 || MODE == MODE_K32B))                            \
+                ? or_if_rem32<(1u << (4 * J + q))>(m[ch], st[ch].low(), c)                            \
           : (MK == MK_REM) ? or_if_rem<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
                            : or_if_marker<(1u << (4 * J + q)), MK>(m[ch], st[ch].low(), c);
 #endif
