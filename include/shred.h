@@ -55,7 +55,8 @@ typedef struct shred_params {
     uint64_t divisor;   /* D, 2 <= D <= 2^deg.  Default 8192 ("13 bits", L447).  Any other D is
                            the integer remainder of the fingerprint's value (reading Q8).  Fast
                            paths: D = 2^m <= 2^32 (either marker), or D = d 2^s with s < 32 and
-                           the '==' marker (divisibility test); other D run the generic path.   */
+                           the '==' marker (divisibility test); every other D by the remainder
+                           itself (a multiply-high quotient).                                   */
     uint64_t magic;     /* r < D.  Default 0x78 (reading Q6).                                  */
     uint64_t min_size;  /* 0 = off (paper default)                                  */
     uint64_t max_size;  /* 0 = off (= inf).  Else max_size >= max(min_size, 1)                 */
