@@ -1,5 +1,6 @@
-"""Small cases of every kernel path, for compute-sanitizer (memcheck / racecheck / synccheck).
-Checks results against the oracle too, so a silent corruption under the tool is caught."""
+"""Small cases of every kernel path, for compute-sanitizer (memcheck / racecheck / synccheck;
+tools/sanitize.sh).  Test infrastructure (kept under tests/ because it calls the oracle): checks
+results against the oracle too, so a silent corruption under the tool is caught."""
 import os
 import sys
 
@@ -37,6 +38,10 @@ def main():
     check(pkg.Chunker(pkg.Params(divisor=10000, magic=1234)), data, 5)          # MK_DIV
     check(pkg.Chunker(pkg.Params(window=47, divisor=4096, magic=9, marker=1)), data[:300000], 2)   # funnel, '<='
     check(pkg.Chunker(pkg.Params(window=65)), data[:100000])                       # generic
+    check(pkg.Chunker(pkg.Params(divisor=12345, magic=3, marker=1)), data[:400000], 7)   # MK_REM, u64
+    check(pkg.Chunker(pkg.Params(divisor=3 << 32, magic=77)), data[:300000], 1)          # MK_REM '=='
+    check(pkg.Chunker(pkg.Params(poly=0x104C11DB7, divisor=1000, magic=2, marker=1)), data[:300000])  # MK_REM, u32
+    check(pkg.Chunker(pkg.Params(poly=0x11D, window=20, divisor=256, magic=9)), data[:300000], 4)      # degree 8
     # f2 / f3: SHA-256 of every chunk (hashlib oracle) and the dedup index
     chh = pkg.Chunker(pkg.Params())
     x = torch.from_numpy(data).cuda()
