@@ -440,6 +440,18 @@ def main():
             v32 = timed(c32, base)
             line["k32_variant"] = {"value": round(v32, 2), "unit": "GB/s", "hbm_frac": round(v32 / hbm, 4),
                                    "params": "P=0x104C11DB7 (deg 32, irreducible), other params as paper"}
+            # content sensitivity. Text-like bytes (words from a fixed
+            # 1,000-word list; skewed outgoing bytes for the U lookups), 64 MiB generated on the
+            # host and tiled to 256 MiB on the device; paper params on the same ctx.
+            import synthgen
+            tl = torch.from_numpy(synthgen.text_like(7, 64 << 20)).to(dev).repeat(4)
+            vt = timed(ch, tl)
+            vr = timed(ch, base[: 256 << 20])
+            line["text_like_256mib"] = {"value": round(vt, 2), "unit": "GB/s", "hbm_frac": round(vt / hbm, 4),
+                                        "random_256mib": round(vr, 2),
+                                        "note": "words from a 1,000-word list (64 MiB tiled x4), paper params; "
+                                                "random_256mib: the first 256 MiB of the random file, same call"}
+            del tl
             # configs[0]: 1 MiB per call, launch-latency bound -> report microseconds per call
             small = base[: 1 << 20]
             o_s = torch.empty(4096, dtype=torch.int64, device=dev)

@@ -88,6 +88,9 @@ void byte_times_xpow(uint64_t P, int k, uint64_t e, uint64_t out[256]) {
 #ifndef SHRED_PDL
 #define SHRED_PDL 1       // 0: plain stream serialization (A/B)
 #endif
+#ifndef SHRED_EDGE_GS
+#define SHRED_EDGE_GS 16  // edge-CTA head/tail segment: each is a chain of w-1 + GS dependent steps
+#endif
 #ifndef SHRED_BYTEIDX
 #define SHRED_BYTEIDX 1   // deg 8/16/24/32: PRMT table index (MODE_K32B); 0: IMAD index (MODE_K32)
 #endif
@@ -254,7 +257,7 @@ uint64_t plan_map(const MapShape &sh, uint64_t src_addr, uint64_t p_begin, uint6
     m = SlotMap{};
     m.t_end = t_end;
     const uint64_t len = t_end > t_begin ? t_end - t_begin : 0;
-    const uint64_t GS = 64;                    // head/tail segment (edge CTA)
+    const uint64_t GS = SHRED_EDGE_GS;         // head/tail segment (edge CTA)
     uint64_t ROWS_CTA = sh.k63 ? CfgK63::ROWS : CfgK32::ROWS;
     uint64_t NTC = sh.k63 ? CfgK63::NTC : CfgK32::NTC;
     bulk = false;
