@@ -52,9 +52,10 @@ constexpr int GEN_THREADS = 256;
 // Launch shape of the hot kernel: CH rows (independent fingerprint chains) per consumer
 // thread, NTC consumer threads (+ 1 producer warp) per CTA, one CTA per SM.  A pipeline round
 // brings ROUND = 64/CH bytes of every row; 4 chunks of 16 B per row per loop iteration.
-template <int CH_, int NTC_>
+template <int CH_, int NTC_, bool DW_ = false>
 struct BulkCfg {
     static constexpr int CH = CH_, NTC = NTC_;
+    static constexpr bool DIRECT_WARM = DW_;              // row start state by positional tables
     static constexpr int ROWS = NTC * CH;                 // rows per bulk CTA
     static constexpr int ROUND = 64 / CH;                 // bytes per row per round
     static constexpr int CPR = ROUND / 16;                // 16-byte chunks per row per round
@@ -80,7 +81,14 @@ using CfgK63 = BulkCfg<SHRED_K63_CH, SHRED_K63_NT>;
 using CfgK32 = BulkCfg<SHRED_K32_CH, SHRED_K32_NT>;
 // Small inputs (< ~5 MB): 128 consumers x 2 rows per CTA (two CTAs per SM fit), so the short
 // rows still spread over every SM (1 MiB: 65 CTAs instead of 17; 19.8 -> 16.7 us per call).
-using CfgSmall = BulkCfg<2, 128>;
+// Its rows are 64 B, as long as the 64-byte warm-up.  DIRECT_WARM (off) computes the row start
+// state directly (w independent positional-table loads) instead of by 64 dependent steps: parity
+// green but slower (1 MiB 13.1 -> 13.5 us per call; the uncoalesced gathers cost more than the
+// chain, which is not the critical path of a small call).
+#ifndef SHRED_DIRECT_WARM
+#define SHRED_DIRECT_WARM 0   // A/B: measured slower (profiles/r01_ab_variants.txt)
+#endif
+using CfgSmall = BulkCfg<2, 128, SHRED_DIRECT_WARM != 0>;
 
 // Slot id -> range of window-end positions.  Slots are numbered in stream order:
 // [0, n_head) generic head segments, then the bulk rows, then generic tail segments.
@@ -479,6 +487,7 @@ template <int MODE>
 struct State;
 template <> struct State<MODE_K63> {
     uint32_t fl = 0, fh = 0;
+    __device__ __forceinline__ void set(uint64_t v) { fl = (uint32_t)v; fh = (uint32_t)(v >> 32); }
     template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
         step63<K>(fl, fh, in, pop, c);
     }
@@ -487,6 +496,7 @@ template <> struct State<MODE_K63> {
 };
 template <> struct State<MODE_K40> {
     uint32_t fl = 0, fh = 0;
+    __device__ __forceinline__ void set(uint64_t v) { fl = (uint32_t)v; fh = (uint32_t)(v >> 32); }
     template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
         step63<K, true>(fl, fh, in, pop, c);
     }
@@ -495,6 +505,7 @@ template <> struct State<MODE_K40> {
 };
 template <> struct State<MODE_K32> {
     uint32_t f = 0;
+    __device__ __forceinline__ void set(uint64_t v) { f = (uint32_t)v; }
     template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
         step32<K, false>(f, in, pop, c);
     }
@@ -503,6 +514,7 @@ template <> struct State<MODE_K32> {
 };
 template <> struct State<MODE_K32B> {
     uint32_t f = 0;
+    __device__ __forceinline__ void set(uint64_t v) { f = (uint32_t)v; }
     template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
         step32<K, true>(f, in, pop, c);
     }
@@ -648,6 +660,8 @@ struct BulkConst {
     uint32_t dsh;
     uint64_t rm, rd, rlo, rspan;   // MK_REM constants (BulkCtx)
     uint32_t rsh2;
+    const uint64_t *pos;       // DIRECT_WARM: C_j[b] = b x^{8j} mod P at pos[256 j + b], j < w
+    uint32_t w;                // window bytes (DIRECT_WARM)
     uint32_t fu, fsel;  // FN windows (w % 16 != 0): e = 16*ceil(w/16) - w = 4*fu + v, fsel = PRMT
                         // selector of bytes v..v+3 (0x3210 + 0x1111 v)
 };
@@ -802,7 +816,6 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         o[ch].lst = J.scratch + (uint64_t)(J.map.n_head + row) * J.cap;
         o[ch].cnt = 0; o[ch].cap = J.cap;
     }
-    mbar_wait(tabbar, 0);                             // T|U image resident
     {
         // warm-up: the 64 bytes before each row (b0 >= p_begin + 64 keeps them inside src)
         const uint4 Z = make_uint4(0, 0, 0, 0);
@@ -816,9 +829,30 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                 for (int q = 0; q < 4; ++q) R[ch][q] = __ldg(h + q);
             }
         }
+        if (C::DIRECT_WARM) {
+            // The state at the row start is the fingerprint of the w bytes before it (the rolled
+            // warm-up pushes 64 bytes and pops all but the last w): XOR of C_j[B[pos0-1-j]] over
+            // j < w, independent loads (no T|U lookups: the table TMA is still in flight).
+#pragma unroll
+            for (int ch = 0; ch < CH; ++ch) {
+                uint64_t f = 0;
+#pragma unroll
+                for (int j = 0; j < 64; ++j) {
+                    if ((uint32_t)j < K.w) {
+                        const int i = 63 - j;             // byte pos0-1-j = byte i of R[ch][0..3]
+                        const uint4 v = R[ch][i >> 4];
+                        const uint32_t wd = ((i >> 2) & 3) == 0 ? v.x : ((i >> 2) & 3) == 1 ? v.y
+                                          : ((i >> 2) & 3) == 2 ? v.z : v.w;
+                        f ^= __ldg(K.pos + 256 * j + ((wd >> (8 * (i & 3))) & 0xFFu));
+                    }
+                }
+                st[ch].set(f);
+            }
+        }
+        mbar_wait(tabbar, 0);                         // T|U image resident
         uint32_t m[CH];
 #pragma unroll
-        for (int q = 0; q < 4; ++q) {
+        for (int q = 0; q < (C::DIRECT_WARM ? 0 : 4); ++q) {
             uint4 d[CH], p[CH];
 #pragma unroll
             uint4 lo[CH], hi[CH];

@@ -114,6 +114,7 @@ struct shred_ctx {
     DevParams dp{};
     uint4 *d_tab_img = nullptr;          // 64 KiB replicated T|U image (fast paths)
     GenTables *d_gen = nullptr;          // plain T/U (generic path, recompute)
+    uint64_t *d_pos = nullptr;           // positional tables C_j[b] = b x^{8j} mod P, j < w (small shape)
     EncodeTiledFn encode = nullptr;
     K1Fn k1_fn = nullptr;                // the hot-kernel instance for these parameters
     K1Fn k1_small_fn = nullptr;          // the same with the small-input shape (or null)
@@ -415,6 +416,7 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
             K.rspan = ctx->p.marker == SHRED_MARKER_LE ? ctx->p.magic : 0;
         }
         K.tsel = 0x5504u | ((uint32_t)((ctx->k - 8) / 8) << 4);         // byte (k-8)/8 -> bits 8..15
+        K.pos = ctx->d_pos; K.w = ctx->p.window;
         int smem = ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM;
         int threads = (ctx->path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC) + 32;
         K1Fn fn = ctx->k1_fn;
@@ -671,6 +673,15 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
             cudaFuncSetAttribute(ctx->k1_small_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  CfgSmall::SMEM) != cudaSuccess)
             return bail(SHRED_ECUDA);
+        if (ctx->k1_small_fn && CfgSmall::DIRECT_WARM) {
+            // the small shape's row start states: C_j[b] = b x^{8j} mod P (direct definition of
+            // the window fingerprint), j < w <= 64: w x 2 KiB
+            std::vector<uint64_t> pos(256 * (size_t)p->window);
+            for (uint32_t j = 0; j < p->window; ++j) byte_times_xpow(p->poly, k, 8ull * j, &pos[256 * (size_t)j]);
+            if (cudaMalloc(&ctx->d_pos, pos.size() * 8) != cudaSuccess) { cudaGetLastError(); return bail(SHRED_ENOMEM); }
+            if (cudaMemcpy(ctx->d_pos, pos.data(), pos.size() * 8, cudaMemcpyHostToDevice) != cudaSuccess)
+                return bail(SHRED_ECUDA);
+        }
     }
     if (cudaFuncSetAttribute(sb_dense, cudaFuncAttributeMaxDynamicSharedMemorySize,
                              (int)(SBD_WIN / 8)) != cudaSuccess)
@@ -692,7 +703,7 @@ void shred_destroy(shred_ctx *ctx) {
     for (auto &e : ctx->prof_ev) cudaEventDestroy(e);
     for (auto p : ctx->ring) cudaFree(p);
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
-    cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_counts); cudaFree(ctx->d_local); cudaFree(ctx->d_groups);
+    cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_pos); cudaFree(ctx->d_counts); cudaFree(ctx->d_local); cudaFree(ctx->d_groups);
     cudaFree(ctx->d_scratch); cudaFree(ctx->d_cand); cudaFree(ctx->d_sb); cudaFree(ctx->d_aux);
     cudaFree(ctx->d_carry[0]); cudaFree(ctx->d_carry[1]); cudaFree(ctx->d_queue); cudaFree(ctx->d_hhist); cudaFree(ctx->d_order);
     cudaFree(ctx->index.tag); cudaFree(ctx->index.key); cudaFree(ctx->index.ready); cudaFree(ctx->index.stats);
