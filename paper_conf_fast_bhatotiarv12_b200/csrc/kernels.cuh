@@ -59,10 +59,11 @@ struct BulkCfg {
     static constexpr int ROWS = NTC * CH;                 // rows per bulk CTA
     static constexpr int ROUND = 64 / CH;                 // bytes per row per round
     static constexpr int CPR = ROUND / 16;                // 16-byte chunks per row per round
+    static constexpr int BOX = ROWS < BOX_ROWS ? ROWS : BOX_ROWS;   // rows per TMA box
     static constexpr int STAGE = ROWS * ROUND;            // bytes per TMA stage
     static constexpr int BAR_OFF = TAB_BYTES + STAGES * STAGE;
     static constexpr int SMEM = BAR_OFF + 2048;           // + barriers/scan scratch + 1 KiB align
-    static_assert(ROWS % BOX_ROWS == 0 && (CH == 1 || CH == 2 || CH == 4) && NTC % 32 == 0 &&
+    static_assert(ROWS % BOX == 0 && STAGE % 1024 == 0 && (CH == 1 || CH == 2 || CH == 4) && NTC % 32 == 0 &&
                   NTC + 32 <= 1024, "shape");
 };
 #ifndef SHRED_K63_CH
@@ -88,7 +89,10 @@ using CfgK32 = BulkCfg<SHRED_K32_CH, SHRED_K32_NT>;
 #ifndef SHRED_DIRECT_WARM
 #define SHRED_DIRECT_WARM 0   // A/B: measured slower (profiles/r01_ab_variants.txt)
 #endif
-using CfgSmall = BulkCfg<2, 128, SHRED_DIRECT_WARM != 0>;
+#ifndef SHRED_SMALL_NT
+#define SHRED_SMALL_NT 128    // 128 consumers x 2 rows; 64 (128-row CTAs, 129 CTAs for 1 MiB): slower (r01_ab_variants)
+#endif
+using CfgSmall = BulkCfg<2, SHRED_SMALL_NT, SHRED_DIRECT_WARM != 0>;
 
 // Slot id -> range of window-end positions.  Slots are numbered in stream order:
 // [0, n_head) generic head segments, then the bulk rows, then generic tail segments.
@@ -780,8 +784,8 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                 mbar_expect_tx(bars + 8 * s, C::STAGE);
                 const uint32_t dst = stages + s * C::STAGE;
 #pragma unroll
-                for (int q = 0; q < C::ROWS / BOX_ROWS; ++q)
-                    tma_load_2d(dst + q * BOX_ROWS * ROUND, &tmap, (int)(r * ROUND), (int)(row0 + q * BOX_ROWS),
+                for (int q = 0; q < C::ROWS / C::BOX; ++q)
+                    tma_load_2d(dst + q * C::BOX * ROUND, &tmap, (int)(r * ROUND), (int)(row0 + q * C::BOX),
                                 bars + 8 * s);
             }
         }

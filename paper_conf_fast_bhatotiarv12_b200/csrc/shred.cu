@@ -346,7 +346,8 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
         // 2-D tensor map [nrows][S] over the bulk bytes
         cuuint64_t gdim[2] = {(cuuint64_t)S, (cuuint64_t)m.nrows};
         cuuint64_t gstride[1] = {(cuuint64_t)S};
-        cuuint32_t box[2] = {(cuuint32_t)ROUND, (cuuint32_t)BOX_ROWS};
+        cuuint32_t box[2] = {(cuuint32_t)ROUND, (cuuint32_t)(pl.small ? CfgSmall::BOX : CfgK63::BOX)};
+        static_assert(CfgK63::BOX == CfgK32::BOX, "box");
         cuuint32_t estr[2] = {1, 1};
         CUresult r = ctx->encode(&pl.tmap, CU_TENSOR_MAP_DATA_TYPE_UINT8, 2,
                                  (void *)(src + (m.b0 - p_begin)), gdim, gstride, box, estr,
