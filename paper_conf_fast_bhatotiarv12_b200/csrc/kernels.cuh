@@ -174,6 +174,14 @@ __device__ __forceinline__ void pdl_entry() {
     asm volatile("griddepcontrol.wait;" ::: "memory");
     asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
 }
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+__device__ __forceinline__ void pdl_trigger() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
+// k1_bulk: the ctx's constant tables (written once at shred_init) are staged and the mbarriers
+// initialised before griddepcontrol.wait, so that prologue overlaps the previous kernel of the
+// stream; everything that reads the input or writes the job's scratch comes after the wait.
+#ifndef SHRED_PDL_EARLY
+#define SHRED_PDL_EARLY 1
+#endif
 
 // ------------------------------------------------------------------------------ PTX helpers
 __device__ __forceinline__ uint32_t smem_u32(const void *p) {
@@ -708,7 +716,7 @@ template <int MODE, class C, int WCH, int MK, bool FN = false>
 __global__ void __launch_bounds__(C::NTC + 32, 1)
 k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_img,
         const GenTables *__restrict__ gt, Job J, DevParams P, BulkConst K) {
-    pdl_entry();
+    if (SHRED_PDL_EARLY) pdl_trigger(); else pdl_entry();
     constexpr int CH = C::CH, NTC = C::NTC, ROUND = C::ROUND, CPR = C::CPR;
     extern __shared__ uint8_t smem_raw[];
     // align the dynamic shared base to 1 KiB (the TMA swizzle pattern is address-based)
@@ -723,6 +731,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         uint64_t *sT = reinterpret_cast<uint64_t *>(smem + TAB_BYTES);
         uint64_t *sU = sT + 256;
         for (int i = tid; i < 256; i += blockDim.x) { sT[i] = gt->T[i]; sU[i] = gt->U[i]; }
+        if (SHRED_PDL_EARLY) pdl_wait();
         // Stage the head and tail byte ranges (with their w-1 warm-up bytes) in the idle stage
         // ring, so the byte loop reads shared memory instead of one dependent global load per
         // byte (that latency chain set a ~16 us floor on every call).
@@ -771,6 +780,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
             bulk_g2s(sbase + q * (TAB_BYTES / 4), reinterpret_cast<const uint8_t *>(tab_img) + q * (TAB_BYTES / 4),
                      TAB_BYTES / 4, tabbar);
     }
+    if (SHRED_PDL_EARLY) pdl_wait();
     __syncthreads();
 
     const uint32_t row0 = blockIdx.x * C::ROWS;
