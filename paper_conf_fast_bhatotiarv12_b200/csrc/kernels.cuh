@@ -44,7 +44,10 @@ namespace shred {
 // K32B: u32 state, deg 8/16/24/32 (whole-byte top byte)
 enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3, MODE_K32B = 4, MODE_K40 = 5 };
 
-constexpr int STAGES      = 4;                 // TMA ring depth
+#ifndef SHRED_STAGES
+#define SHRED_STAGES 2   // A/B (profiles/r01_ab_variants.txt): 2 stages 1,879 GB/s > 3: 1,861 > 4: 1,854
+#endif
+constexpr int STAGES      = SHRED_STAGES;      // TMA ring depth (5 does not fit beside the 64 KiB table)
 constexpr int BOX_ROWS    = 256;               // rows per TMA box (hardware max 256)
 constexpr int TAB_BYTES   = 65536;             // replicated T|U image (256 rows x 256 B)
 constexpr int GEN_THREADS = 256;
