@@ -667,6 +667,9 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
             cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM) != cudaSuccess)
             return bail(SHRED_ECUDA);
+#ifdef SHRED_CARVEOUT   // A/B only: force the L1/SMEM split of the hot kernel (percent of max smem)
+        cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributePreferredSharedMemoryCarveout, SHRED_CARVEOUT);
+#endif
 #ifndef SHRED_NO_SMALL
         ctx->k1_small_fn = pick_k1_small(k, byteidx, wch, ctx->mk, funnel);
 #endif
