@@ -55,12 +55,16 @@ constexpr int GEN_THREADS = 256;
 // Launch shape of the hot kernel: CH rows (independent fingerprint chains) per consumer
 // thread, NTC consumer threads (+ 1 producer warp) per CTA, one CTA per SM.  A pipeline round
 // brings ROUND = 64/CH bytes of every row; 4 chunks of 16 B per row per loop iteration.
+#ifndef SHRED_ROUND
+#define SHRED_ROUND 0   // 0: 64/CH bytes per row per TMA round; A/B: 16 (smaller stages)
+#endif
 template <int CH_, int NTC_, bool DW_ = false>
 struct BulkCfg {
     static constexpr int CH = CH_, NTC = NTC_;
     static constexpr bool DIRECT_WARM = DW_;              // row start state by positional tables
     static constexpr int ROWS = NTC * CH;                 // rows per bulk CTA
-    static constexpr int ROUND = 64 / CH;                 // bytes per row per round
+    static constexpr int ROUND = SHRED_ROUND ? SHRED_ROUND : 64 / CH;   // bytes per row per round
+    static constexpr int RPI = 64 / ROUND;                // rounds per 64-byte loop iteration
     static constexpr int CPR = ROUND / 16;                // 16-byte chunks per row per round
     static constexpr int BOX = ROWS < BOX_ROWS ? ROWS : BOX_ROWS;   // rows per TMA box
     static constexpr int STAGE = ROWS * ROUND;            // bytes per TMA stage
@@ -888,9 +892,9 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     // low bits as tid): SWIZZLE_64B: ^ (row >> 1) & 3, SWIZZLE_32B: ^ (row >> 2) & 1, 16 B: none
     const uint32_t swz = (ROUND == 64) ? (((uint32_t)tid >> 1) & 3u)
                        : (ROUND == 32) ? (((uint32_t)tid >> 2) & 1u) : 0u;
-    for (uint32_t r = 0; r < nrounds; r += CH) {
+    for (uint32_t r = 0; r < nrounds; r += C::RPI) {
 #pragma unroll
-        for (int qr = 0; qr < CH; ++qr) {             // round r + qr: chunks qr*CPR .. +CPR-1
+        for (int qr = 0; qr < C::RPI; ++qr) {             // round r + qr: chunks qr*CPR .. +CPR-1
             const uint32_t s = (r + qr) % STAGES;
             mbar_wait(bars + 8 * s, ((r + qr) / STAGES) & 1u);
             const uint32_t sb = stages + s * C::STAGE;
