@@ -135,22 +135,59 @@ def cpu_model() -> str:
     return "unknown"
 
 
-def cpu_baseline(host: np.ndarray, budget_s: float = 12.0):
-    """Oracle (R2, multithreaded over this process's cores) on a bounded prefix sample."""
+def cpu_measurements(runs: int = 3, budget_s: float = 4.0) -> dict:
+    """The host-core baselines, measured in a FRESH process with no CUDA context (bench.py
+    --cpu-only, started before the parent touches the GPU): the oracle (R2, all cores) on a
+    bounded prefix of the configs[1] base file, median of `runs`, and the paper's §5.1
+    multithreaded rolling chunker on the whole file.  Round 1 measured the oracle in-process
+    after the CUDA work and got half the rate of the same code in a fresh process."""
     import oracle
+    import synthgen
     oracle.build()
-    cores = len(os.sched_getaffinity(0))
-    cal = host[: 8 << 20]
-    rate, dt, _ = oracle_rate(cal, cores)
+    cores = sorted(os.sched_getaffinity(0))
+    nc = len(cores)
+    host = synthgen.random_bytes_fast(2, GiB)             # = the device's synth_fill(seed 2)
+    rate, _, _ = oracle_rate(host[: 8 << 20], nc)          # calibration (also warms the tables)
     n = int(min(host.size, max(16 << 20, rate * 1e9 * budget_s)))
     n -= n % 4096
-    rate, dt, nc = oracle_rate(host[:n], cores)
-    rate1, dt1, _ = oracle_rate(host[: 16 << 20], 1)          # SURVEY §8(d) d3: also on 1 core
-    return {"value": round(rate, 4), "unit": "GB/s", "cores": cores, "kind": "oracle",
-            "sample": f"first {n / 2**20:.0f} MiB of the configs[1] base file, R2 direct per-window "
-                      f"reduction (48 table lookups/window), {cores} threads, {dt:.1f} s, {nc} candidates",
-            "value_1core": round(rate1, 4), "sample_1core": f"first 16 MiB, 1 thread, {dt1:.1f} s",
-            "cpu_model": cpu_model()}
+    rates, ncand = [], 0
+    for _ in range(runs):
+        r, dt, ncand = oracle_rate(host[:n], nc)
+        rates.append(r)
+    rate1, dt1, _ = oracle_rate(host[: 8 << 20], 1)
+    out = {"cpu_baseline": {
+        "value": round(float(np.median(rates)), 4), "unit": "GB/s", "cores": nc, "kind": "oracle",
+        "sample": f"first {n / 2**20:.0f} MiB of the configs[1] base file (SplitMix64 seed 2), R2 direct "
+                  f"per-window reduction (48 table lookups/window), {nc} threads, median of {runs} runs "
+                  f"({', '.join(f'{r:.4f}' for r in rates)} GB/s), fresh process without a CUDA context",
+        "runs": [round(r, 4) for r in rates], "affinity": f"cpus {cores[0]}-{cores[-1]} ({nc})",
+        "value_1core": round(rate1, 4), "sample_1core": f"first 8 MiB, 1 thread, {dt1:.1f} s",
+        "cpu_model": cpu_model()}}
+    try:
+        import cpu_baseline as cb
+        cb.build()
+        cb.chunk(host[: 64 << 20], threads=nc)
+        cr, cnt = [], 0
+        for _ in range(runs):
+            t0 = time.perf_counter()
+            cnt = int(cb.chunk(host, threads=nc).size)
+            cr.append(host.size / (time.perf_counter() - t0) / 1e9)
+        out["cpu_chunker"] = {"value": round(float(np.median(cr)), 3), "unit": "GB/s", "cores": nc,
+                              "runs": [round(r, 3) for r in cr], "count": cnt,
+                              "kind": "multithreaded rolling chunker (PAPER.md §5.1 SPMD, gcc -O3 -march=x86-64-v3)",
+                              "sample": f"the whole 1 GiB base file, median of {runs} runs, fresh process"}
+    except Exception as e:
+        out["cpu_chunker"] = {"error": repr(e)}
+    return out
+
+
+def cpu_measurements_subprocess() -> dict:
+    import subprocess
+    r = subprocess.run([sys.executable, os.path.abspath(__file__), "--cpu-only"], capture_output=True, text=True)
+    for ln in reversed(r.stdout.splitlines()):
+        if ln.startswith("{"):
+            return json.loads(ln)
+    return {"cpu_baseline": {"error": (r.stderr or r.stdout)[-400:]}}
 
 
 # ------------------------------------------------------------------------------- reference arm
@@ -201,14 +238,20 @@ def main():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--no-extra", action="store_true", help="skip the bounded / k32 side measurements")
+    ap.add_argument("--cpu-only", action="store_true", help=argparse.SUPPRESS)   # internal: fresh-process CPU leg
     ap.add_argument("--variant", default="paper", choices=["paper", "k32"],
                     help="profiling aid: k32 = P 0x104C11DB7 on the main path (not the headline)")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
 
     rank, world, local = env_int("RANK", 0), env_int("WORLD_SIZE", 1), env_int("LOCAL_RANK", 0)
+    if args.cpu_only:
+        print(json.dumps(cpu_measurements()), flush=True)
+        return
     if args.impl == "reference":
         return run_reference(args, rank, world)
+    # host-core baselines first, in a fresh process, before this process creates a CUDA context
+    cpu = cpu_measurements_subprocess() if (not args.no_cpu and rank == 0 and world == 1) else None
 
     import torch
     import torch.distributed as dist
@@ -301,11 +344,12 @@ def main():
     k_avg_ms = k_ms / max(1, k_n)
     k_bytes_per_launch = k_bytes / max(1, k_n)
     achieved = k_bytes_per_launch / (k_avg_ms * 1e-3) / 1e9 if k_n else None
-    traffic = None
+    traffic, traffic_src = None, None
     try:
         with open(os.path.join(ROOT, "profiles", "k1_traffic.json")) as f:
             tr = json.load(f)
         traffic = tr.get("dram_bytes_per_launch")
+        traffic_src = tr.get("source")
     except Exception:
         pass
     roofline = {"bound": "hbm", "achieved": round(achieved, 1) if achieved else None, "peak": hbm,
@@ -313,6 +357,7 @@ def main():
                 "kernel": f"k1_bulk<{ch.path.upper()}>", "launches": k_n, "avg_launch_ms": round(k_avg_ms, 4),
                 "algorithmic_bytes_per_launch": int(k_bytes_per_launch),
                 "share_of_step": round(k_ms / ms, 4) if ms else None, "peak_source": hbm_src,
+                "traffic_source": traffic_src,
                 "note": "algorithmic bytes = 1 B read per input byte (+8 B per candidate, ~0.001 B/B); "
                         "the kernel is bound by the shared-memory lookup datapath below HBM (DESIGN.md)"}
     # the unit that actually binds: 128 B/clk/SM of shared-memory datapath; per input byte the K63
@@ -383,6 +428,13 @@ def main():
         s1.record(stream)
         torch.cuda.synchronize()
         ems = s0.elapsed_time(s1)
+        # the last e2e step's offsets (base + edited, copied back to pinned host) == the
+        # device-resident path's, element by element (world 1: both chunk the same two files)
+        match = None
+        if world == 1:
+            na_, nb_ = int(n0.item()), int(n1.item())
+            match = bool(a == na_ and b == nb_ and torch.equal(res_h[:a], out0[:na_].cpu())
+                         and torch.equal(res_h[a:a + b], out1[:nb_].cpu()))
         et = coll_dev(torch.tensor([ems], dtype=torch.float64, device=dev))
         if world > 1:
             dist.all_reduce(et, op=dist.ReduceOp.MAX)
@@ -415,7 +467,7 @@ def main():
                        "d2h_bytes_per_step": d2h[0], "ms_per_step": round(ems / args.steps, 3),
                        "api": "shred_feed(pinned host, 2 x 256 MiB device slots) + shred_flush + D2H of cuts",
                        "h2d_peak_gbs": round(h2d_peak, 2), "frac_of_h2d_peak": round(ev / world / h2d_peak, 4),
-                       "cuts_match_device_path": (a == int(n0.item()) if world == 1 else None)}
+                       "cuts_match_device_path": match}
         del tmp
 
     # ---- side measurements (not the headline): bounded mode and the k32 instantiation
@@ -527,23 +579,15 @@ def main():
         except Exception as e:  # side numbers must never break the headline line
             line["extra_error"] = repr(e)
 
-    # ---- CPU baselines on this box's host cores (rank 0, N = 1 only): the oracle, and the
-    # multithreaded rolling chunker of the paper's §5.1 design (cpu_baseline/)
-    if not args.no_cpu and rank == 0 and world == 1:
-        line["cpu_baseline"] = cpu_baseline(host_base)
-        try:
-            import cpu_baseline as cb
-            cb.build()
-            cores = len(os.sched_getaffinity(0))
-            cb.chunk(host_base[: 64 << 20], threads=cores)
-            t0 = time.perf_counter()
-            cc = cb.chunk(host_base, threads=cores)
-            dt = time.perf_counter() - t0
-            line["cpu_chunker"] = {"value": round(host_base.size / dt / 1e9, 3), "unit": "GB/s", "cores": cores,
-                                   "kind": "multithreaded rolling chunker (PAPER.md §5.1 SPMD, gcc -O3 -march=x86-64-v3)",
-                                   "sample": "the whole 1 GiB base file", "matches_gpu_count": int(cc.size) == n_cand}
-        except Exception as e:
-            line["cpu_chunker"] = {"error": repr(e)}
+    # ---- CPU baselines on this box's host cores (rank 0, N = 1 only; measured above in a fresh
+    # process before the CUDA work): the oracle, and the paper's §5.1 multithreaded chunker
+    if cpu is not None:
+        line["cpu_baseline"] = cpu.get("cpu_baseline")
+        if "cpu_chunker" in cpu:
+            cc = dict(cpu["cpu_chunker"])
+            if "count" in cc:
+                cc["matches_gpu_count"] = cc.pop("count") == n_cand
+            line["cpu_chunker"] = cc
 
     if rank == 0:
         print(json.dumps(line), flush=True)

@@ -166,6 +166,66 @@ def candidates(data, p: Params = Params(), method: int = 2, threads: int | None 
         cap = int(n)
 
 
+def candidates_stream(seed: int, n: int, p: Params = Params(), slice_bytes: int = 1 << 30,
+                      threads: int | None = None):
+    """Candidates of the first n bytes of the synthetic stream ``seed`` (synthgen), computed
+    slice by slice so that GiB-scale configs fit in host memory (R2 over
+    host slices with a w-1 byte overlap, the partition-with-overlap of PAPER.md L282-L287).
+
+    Yields (a, b, cands) for consecutive slices: cands = every candidate c with a < c <= b
+    (a = 0 for the first slice, whose lower end is the stream start), ascending, absolute.
+    Slice [a, b) is evaluated on the stream bytes [a - (w-1), b + 1): its full windows end at
+    i in [a, b - 1] (c = i + 1 in [a + 1, b]; c = b + 1 is excluded by c < N of the slice, and
+    it is the next slice's first candidate position).  The last slice ends at N = n, where
+    c < n (reading Q11).  Pinned against :func:`candidates` on whole streams in
+    tests/test_oracle.py::test_candidates_stream_equals_whole."""
+    import synthgen
+    import threading
+    k = p.window - 1
+    bounds = list(range(0, n, slice_bytes)) + [n]
+
+    def load(j):
+        a, b = bounds[j], bounds[j + 1]
+        lo, hi = max(0, a - k), min(n, b + 1)
+        return synthgen.random_bytes_fast(seed, hi - lo, lo), lo
+
+    nxt = [None]
+
+    def prefetch(j):
+        nxt[0] = load(j)
+
+    t = None
+    cur = load(0) if len(bounds) > 1 else None
+    for j in range(len(bounds) - 1):
+        if j + 2 < len(bounds):
+            t = threading.Thread(target=prefetch, args=(j + 1,))
+            t.start()
+        data, lo = cur
+        a, b = bounds[j], bounds[j + 1]
+        c = candidates(data, p, 2, threads) + np.uint64(lo)
+        yield a, b, c[(c > np.uint64(a)) & (c <= np.uint64(b))]
+        if t is not None:
+            t.join()
+            t = None
+            cur = nxt[0]
+
+
+def bucket_digests(cuts: np.ndarray, n: int, bucket: int = 1 << 30) -> list[list]:
+    """[count, sha256 hex] of the ascending offsets c with j*bucket < c <= (j+1)*bucket, for
+    every bucket j covering [1, n): a compact exact record of a GiB-scale cut list (the
+    little-endian u64 bytes of each bucket are hashed), so full-size results can be compared
+    element by element against oracle values stored by tools/oracle_fullsize.py."""
+    import hashlib
+    c = np.ascontiguousarray(cuts, dtype="<u8")
+    nb = max(1, (n - 1 + bucket - 1) // bucket)
+    idx = np.searchsorted(c, np.arange(0, nb + 1, dtype=np.uint64) * np.uint64(bucket), side="right")
+    out = []
+    for j in range(nb):
+        part = c[idx[j]:idx[j + 1]]
+        out.append([int(part.size), hashlib.sha256(part.tobytes()).hexdigest()])
+    return out
+
+
 def size_bound(cands: np.ndarray, n: int, min_size: int, max_size: int) -> np.ndarray:
     """The min/max rule over ascending candidates (L259-L269, Q12-Q15); max_size 0 = inf."""
     c = np.ascontiguousarray(cands, dtype=np.uint64)

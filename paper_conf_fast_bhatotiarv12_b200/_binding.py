@@ -212,9 +212,20 @@ class Chunker:
             c = n
         raise ShredError(f"capacity {c} < {n} candidates")
 
+    def _rule_cap(self, n_cand: int, span: int) -> int:
+        """Cuts the size rule can emit over `span` bytes from `n_cand` candidates: the accepted
+        candidates, the forced cuts (one per max_size bytes) and a held cut; with min_size > 0
+        also at most span // min_size + 1 (ADVICE r01: bounded by the range, not by its
+        absolute end offset)."""
+        p = self.params
+        cap = n_cand + (span // p.max_size + 1 if p.max_size else 0) + 2
+        if p.min_size:
+            cap = min(cap, span // p.min_size + 2)
+        return max(1, cap)
+
     def size_bound(self, cands: torch.Tensor, total_len: int, cap: int | None = None) -> torch.Tensor:
         assert cands.is_cuda and cands.dtype == torch.int64 and cands.is_contiguous()
-        cap = self.max_cuts(total_len) if cap is None else cap
+        cap = self._rule_cap(cands.numel(), total_len) if cap is None else cap
         out = self._out(cap)
         rc = lib().shred_size_bound(self._ctx, cands.data_ptr(), cands.numel(), total_len,
                                     out.data_ptr(), out.numel(), self._n.data_ptr(), _stream(None))
@@ -230,7 +241,7 @@ class Chunker:
         assert cands.dtype == torch.int64 and cands.is_contiguous()
         dev = torch.device("cuda", self.device)
         c = cands if cands.is_cuda else cands.to(dev)
-        cap = self.max_cuts(end + 2) + 2 if cap is None else cap
+        cap = self._rule_cap(c.numel(), end - s) if cap is None else cap
         out = self._out(cap)
         st = torch.zeros(2, dtype=torch.int64, device=dev)
         sin = (ctypes.c_uint64 * 2)(s, int(held))

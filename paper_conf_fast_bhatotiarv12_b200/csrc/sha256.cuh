@@ -87,11 +87,14 @@ __device__ __forceinline__ void sha256_init(uint32_t (&H)[8]) {
 __device__ __forceinline__ void sha256_block(const uint8_t *__restrict__ in, uint64_t in_len, uint64_t a,
                                              uint64_t L, uint64_t blk, uint32_t (&W)[16]) {
     const uint64_t m0 = blk * 64;                     // message offset of the block
-    const uint64_t p = a + m0;                        // stream position
-    const uint64_t wa = p & ~3ull;                    // aligned word start
-    if (m0 + 64 <= L && wa + 68 <= in_len) {          // full block, 17 aligned words in bounds
-        const uint32_t *src = reinterpret_cast<const uint32_t *>(in + wa);
-        const uint32_t sh = (uint32_t)(p & 3) * 8;
+    // word alignment of the ABSOLUTE address (in itself may be unaligned, e.g. a slice x[1:]);
+    // an aligned word that holds a byte of [in, in + in_len) lies inside the same allocation
+    const uintptr_t pa = reinterpret_cast<uintptr_t>(in) + a + m0;
+    const uintptr_t wa = pa & ~(uintptr_t)3;
+    const uintptr_t lim = (reinterpret_cast<uintptr_t>(in) + in_len + 3) & ~(uintptr_t)3;
+    if (m0 + 64 <= L && wa + 68 <= lim) {             // full block, 17 aligned words in bounds
+        const uint32_t *src = reinterpret_cast<const uint32_t *>(wa);
+        const uint32_t sh = (uint32_t)(pa & 3) * 8;
         uint32_t prev = __ldg(src);
 #pragma unroll
         for (int k = 0; k < 16; ++k) {
@@ -210,10 +213,13 @@ k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__re
             // full blocks: the 17 aligned words of block blk+1 are loaded before block blk is
             // compressed (software pipelining: the load latency hides behind ~1.5K cycles of
             // rounds); the padded tail blocks take the byte path of sha256_block
-            const uint32_t sh = (uint32_t)(a & 3) * 8;
-            const uint32_t *src0 = reinterpret_cast<const uint32_t *>(in + (a & ~3ull));
+            // word loads aligned on the ABSOLUTE address (in may be unaligned: ADVICE r01)
+            const uintptr_t pa = reinterpret_cast<uintptr_t>(in) + a;
+            const uintptr_t lim = (reinterpret_cast<uintptr_t>(in) + len + 3) & ~(uintptr_t)3;
+            const uint32_t sh = (uint32_t)(pa & 3) * 8;
+            const uint32_t *src0 = reinterpret_cast<const uint32_t *>(pa & ~(uintptr_t)3);
             uint64_t nfull = L / 64;                               // complete message blocks
-            if (nfull && (a & ~3ull) + 64 * nfull + 4 > len) --nfull;   // 17th word in bounds
+            if (nfull && (pa & ~(uintptr_t)3) + 64 * nfull + 4 > lim) --nfull;   // 17th word in bounds
             uint32_t Rw[17];
             if (nfull) {
 #pragma unroll

@@ -151,6 +151,12 @@ struct shred_ctx {
     uint64_t launches = 0;
     std::string last_error;
 
+    // stream order of the ctx's shared scratch / aux / ring (StreamOrder): the end of the last
+    // call is recorded on its stream; a call on another stream first waits on it
+    cudaEvent_t ev_done = nullptr;
+    cudaStream_t last_st = nullptr;
+    bool last_valid = false;
+
     // hot-kernel profiling (shred_profile)
     bool prof = false;
     std::vector<cudaEvent_t> prof_ev;    // pool, pairs
@@ -318,13 +324,27 @@ uint64_t plan_map(const MapShape &sh, uint64_t src_addr, uint64_t p_begin, uint6
     return S;
 }
 
-// Per-slot list capacity: twice the expected count of the longest segment + slack.
-uint32_t slot_cap(const SlotMap &m, bool bulk, uint64_t divisor) {
+// Per-slot list capacity: twice the expected count of the longest segment + slack.  The hit
+// rate is 1/D for the '==' marker and (r+1)/D for the '<=' set (sizing '<=' lists
+// by 1/D overflowed every list for a large r, sending unbounded calls to the re-roll and
+// bounded calls to the one-CTA sb_dense walk).  At most SLOT_CAP_MAX entries per slot, and the
+// lists of all slots stay within SCRATCH_BUDGET bytes; beyond that the input is dense and the
+// overflow paths (exact) take over.
+constexpr uint64_t SLOT_CAP_MAX = 4096;
+constexpr uint64_t SCRATCH_BUDGET = 4ull << 30;
+uint32_t slot_cap(const SlotMap &m, bool bulk, uint64_t divisor, uint64_t hits_per_d, uint64_t nslots) {
     uint64_t maxseg = bulk ? m.S : m.head_seg;
     if (bulk && m.tail_seg > maxseg) maxseg = m.tail_seg;
-    uint64_t cap = 2 * maxseg / divisor + 16;
-    return (uint32_t)(cap > 256 ? 256 : cap);
+    const long double exp = (long double)maxseg * (long double)hits_per_d / (long double)divisor;
+    long double capf = 2.0L * exp + 16.0L;
+    if (capf > (long double)SLOT_CAP_MAX) capf = (long double)SLOT_CAP_MAX;
+    uint64_t cap = (uint64_t)capf;
+    if (nslots && cap * 8 * nslots > SCRATCH_BUDGET) cap = SCRATCH_BUDGET / 8 / nslots;
+    if (cap < 16) cap = 16;
+    return (uint32_t)cap;
 }
+// candidate hits per D positions for the ctx's marker set: 1 ('=='), r + 1 ('<=')
+uint64_t hits_per_d(const shred_params &p) { return p.marker == SHRED_MARKER_LE ? p.magic + 1 : 1; }
 
 // Plan candidate detection for window ends [t_begin, t_end) of a job whose bytes start at
 // stream position p_begin (src) with `prefix_len` carried bytes before it.
@@ -359,7 +379,8 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
     }
     pl.nslots = m.n_head + m.nrows + m.n_tail;
     if (m.ngroups > (uint32_t)MAX_GROUPS) return fail(ctx, SHRED_EINVAL, "too many slot groups (%u)", m.ngroups);
-    J.cap = slot_cap(m, pl.bulk, ctx->p.divisor);
+    pl.nslots = m.n_head + m.nrows + m.n_tail;
+    J.cap = slot_cap(m, pl.bulk, ctx->p.divisor, hits_per_d(ctx->p), pl.nslots);
     int rc;
     if ((rc = grow(ctx, ctx->d_counts, ctx->counts_cap, (uint64_t)pl.nslots + 1, "counts"))) return rc;
     if ((rc = grow(ctx, ctx->d_local, ctx->local_cap, (uint64_t)pl.nslots + 1, "local offsets"))) return rc;
@@ -544,6 +565,27 @@ struct DevGuard {
     ~DevGuard() { if (prev >= 0) cudaSetDevice(prev); }
 };
 
+// Every call's work uses the ctx's scratch, aux state and ring, so calls on one ctx must run in
+// order even when they are enqueued on different streams (two one-shot calls on two
+// streams raced on d_aux[0] and the scratch lists).  The guard makes a call on a stream other
+// than the previous call's wait for that call's completion event, and records its own at the
+// end.  Under stream capture (CUDA graphs) nothing is recorded or waited on: a captured call
+// must be captured on the stream the ctx's preceding work used (include/shred.h "Streams").
+struct StreamOrder {
+    shred_ctx *ctx; cudaStream_t st; bool cap = false;
+    StreamOrder(shred_ctx *c, cudaStream_t s) : ctx(c), st(s) {
+        cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
+        if (cudaStreamIsCapturing(st, &cs) != cudaSuccess) cudaGetLastError();
+        cap = cs != cudaStreamCaptureStatusNone;
+        if (!cap && ctx->last_valid && ctx->last_st != st) cudaStreamWaitEvent(st, ctx->ev_done, 0);
+    }
+    ~StreamOrder() {
+        if (cap) { ctx->last_valid = false; return; }
+        if (cudaEventRecord(ctx->ev_done, st) == cudaSuccess) { ctx->last_st = st; ctx->last_valid = true; }
+        else { cudaGetLastError(); ctx->last_valid = false; }
+    }
+};
+
 }  // namespace
 
 // ============================================================================ C ABI
@@ -690,7 +732,8 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     if (cudaFuncSetAttribute(sb_dense, cudaFuncAttributeMaxDynamicSharedMemorySize,
                              (int)(SBD_WIN / 8)) != cudaSuccess)
         return bail(SHRED_ECUDA);
-    if (cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking) != cudaSuccess)
+    if (cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking) != cudaSuccess ||
+        cudaEventCreateWithFlags(&ctx->ev_done, cudaEventDisableTiming) != cudaSuccess)
         return bail(SHRED_ECUDA);
     if (cudaDeviceSynchronize() != cudaSuccess) return bail(SHRED_ECUDA);
     *out = ctx;
@@ -705,6 +748,7 @@ void shred_destroy(shred_ctx *ctx) {
     for (auto &e : ctx->ev_free) cudaEventDestroy(e);
     for (auto &e : ctx->ev_ready) cudaEventDestroy(e);
     for (auto &e : ctx->prof_ev) cudaEventDestroy(e);
+    if (ctx->ev_done) cudaEventDestroy(ctx->ev_done);
     for (auto p : ctx->ring) cudaFree(p);
     if (ctx->copy_stream) cudaStreamDestroy(ctx->copy_stream);
     cudaFree(ctx->d_tab_img); cudaFree(ctx->d_gen); cudaFree(ctx->d_pos); cudaFree(ctx->d_counts); cudaFree(ctx->d_local); cudaFree(ctx->d_groups);
@@ -725,6 +769,7 @@ int shred_chunk(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, uint64_t *d_o
     if (len && !d_in) return fail(ctx, SHRED_EINVAL, "d_in is NULL");
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
     Aux *aux = ctx->d_aux + 0;
     if (!bounded(ctx)) {
         Plan pl;
@@ -752,6 +797,7 @@ int shred_candidates_range(shred_ctx *ctx, const uint8_t *d_in, uint64_t halo, u
     if ((len || halo) && !d_in) return fail(ctx, SHRED_EINVAL, "d_in is NULL");
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
     Aux *aux = ctx->d_aux + 0;
     Plan pl;
     if ((rc = plan_job(ctx, pl, d_in, start - halo, nullptr, 0, start, start + len, total_len))) return rc;
@@ -767,6 +813,7 @@ int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, ui
     if (n_cand && !d_cand) return fail(ctx, SHRED_EINVAL, "d_cand is NULL");
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
     Aux *aux = ctx->d_aux + 0;
     PDL(k_stream_reset, 1, 1, 0, st, aux);
     LAUNCHED("k_stream_reset");
@@ -787,6 +834,7 @@ int shred_size_bound_state(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_ca
     if (state_in[0] > end) return fail(ctx, SHRED_EINVAL, "entry state beyond the range end");
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
     Aux *aux = ctx->d_aux + 0;
     PDL(k_state_in, 1, 1, 0, st, aux, state_in[0], state_in[1] ? 1ull : 0ull);
     LAUNCHED("k_state_in");
@@ -858,6 +906,7 @@ int shred_feed(shred_ctx *ctx, const void *in, uint64_t len, uint64_t *d_out, ui
     if (rc) return rc;
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
     Aux *aux = ctx->d_aux + 1;
     PDL(k_call_begin, 1, 1, 0, st, aux);
     LAUNCHED("k_call_begin");
@@ -915,6 +964,7 @@ int shred_flush(shred_ctx *ctx, uint64_t *d_out, uint64_t cap, uint64_t *n_out, 
     if (rc) return rc;
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
     // Every forced cut strictly inside the stream was emitted by the last feed; a cut held at
     // exactly the stream end is dropped (c = N is never a cut, reading Q11).
     PDL(k_stream_reset, 1, 1, 0, st, ctx->d_aux + 1);
@@ -947,6 +997,7 @@ int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const u
     if (!len || !max_chunks) return SHRED_OK;
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
     int rc = grow(ctx, ctx->d_order, ctx->order_cap, max_chunks, "hash order");
     if (rc) return rc;
     if (max_chunks > 0xFFFFFFFFull) return fail(ctx, SHRED_EINVAL, "max_chunks must be < 2^32");
@@ -982,8 +1033,11 @@ int shred_index_reset(shred_ctx *ctx, uint64_t capacity) {
         T.cap = cap;
     }
     if (!T.stats && cudaMalloc(&T.stats, 64) != cudaSuccess) { cudaGetLastError(); return SHRED_ENOMEM; }
+    // cudaMemset runs on the legacy default stream and does not block the host; the call has no
+    // stream argument, so it completes the clear before returning (a following insert on a
+    // non-blocking stream must not see stale slots: ADVICE r01)
     if (cudaMemset(T.tag, 0, cap * 8) != cudaSuccess || cudaMemset(T.ready, 0, cap * 4) != cudaSuccess ||
-        cudaMemset(T.stats, 0, 64) != cudaSuccess)
+        cudaMemset(T.stats, 0, 64) != cudaSuccess || cudaDeviceSynchronize() != cudaSuccess)
         return fail(ctx, SHRED_ECUDA, "index reset");
     return SHRED_OK;
 }
@@ -998,6 +1052,7 @@ int shred_index_insert(shred_ctx *ctx, const uint8_t *d_digests, const uint64_t 
     if (!len || !max_chunks) return SHRED_OK;
     DevGuard g(ctx->device);
     cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
     PDL(k_dedup_insert, ctx->sm_count * 8, 256, 0, st, ctx->index, d_digests, d_cuts, d_ncuts, len, max_chunks,
                                                       d_new_flags);
     LAUNCHED("k_dedup_insert");
@@ -1033,7 +1088,7 @@ int shred_debug_plan(int path, int small_ok, int sm_count, uint64_t src_addr, ui
     plan_map(sh, src_addr, p_begin, t_begin, t_end, m, bulk, small);
     const uint64_t v[16] = {bulk, small, m.head_start, m.head_seg, m.n_head, m.b0, m.S, m.nrows,
                             m.tail_start, m.tail_seg, m.n_tail, m.nc, m.ngroups, m.rows_cta,
-                            slot_cap(m, bulk, divisor), small ? (uint64_t)CfgSmall::NTC
+                            slot_cap(m, bulk, divisor, 1, 0), small ? (uint64_t)CfgSmall::NTC
                                                               : (uint64_t)(path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC)};
     for (int i = 0; i < 16; ++i) out[i] = v[i];
     return SHRED_OK;

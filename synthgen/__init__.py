@@ -66,6 +66,46 @@ def fill_random_into(buf: np.ndarray, seed: int, offset: int = 0, block: int = 1
         buf[b:b + m] = random_bytes(seed, m, offset + b)
 
 
+_FILL_SRC = __import__("os").path.join(__import__("os").path.dirname(__file__), "splitmix_fill.c")
+_FILL_LIB = _FILL_SRC[:-len("splitmix_fill.c")] + "libsplitmix.so"
+_fill_lib = None
+
+
+def _fill():
+    """The multithreaded C filler (splitmix_fill.c, gcc), same stream definition as above."""
+    global _fill_lib
+    if _fill_lib is None:
+        import ctypes
+        import os
+        import subprocess
+        if not os.path.exists(_FILL_LIB) or os.path.getmtime(_FILL_LIB) < os.path.getmtime(_FILL_SRC):
+            tmp = _FILL_LIB + f".tmp{os.getpid()}"
+            subprocess.check_call(["gcc", "-O2", "-std=c11", "-fPIC", "-shared", "-pthread", "-o", tmp, _FILL_SRC])
+            os.replace(tmp, _FILL_LIB)
+        lib = ctypes.CDLL(_FILL_LIB)
+        lib.sg_fill.restype = ctypes.c_int
+        lib.sg_fill.argtypes = [ctypes.c_void_p, ctypes.c_uint64, ctypes.c_uint64, ctypes.c_uint64, ctypes.c_int]
+        _fill_lib = lib
+    return _fill_lib
+
+
+def fill_fast(buf: np.ndarray, seed: int, offset: int = 0, threads: int | None = None) -> np.ndarray:
+    """Bytes [offset, offset + buf.size) of stream ``seed`` into the contiguous uint8 ``buf``,
+    multithreaded C (GB/s; the numpy form above is ~0.2 GB/s).  Returns ``buf``."""
+    import os
+    assert buf.dtype == np.uint8 and buf.flags["C_CONTIGUOUS"]
+    if threads is None:
+        threads = len(os.sched_getaffinity(0))
+    if buf.size:
+        _fill().sg_fill(buf.ctypes.data, buf.size, seed & 0xFFFFFFFFFFFFFFFF, offset, threads)
+    return buf
+
+
+def random_bytes_fast(seed: int, length: int, offset: int = 0) -> np.ndarray:
+    """:func:`random_bytes` through the C filler."""
+    return fill_fast(np.empty(max(0, length), dtype=np.uint8), seed, offset)
+
+
 def _uniform(seed: int, count: int) -> np.ndarray:
     """``count`` doubles in [0,1) from the SplitMix64 stream ``seed`` (top 53 bits)."""
     w = splitmix_words(seed, 0, count)

@@ -29,6 +29,25 @@ def test_padding_edge_lengths(pkg):
     assert np.array_equal(got.cpu().numpy(), exp)
 
 
+@pytest.mark.parametrize("shift", [1, 2, 3, 5])
+def test_unaligned_input_pointer(pkg, shift):
+    """d_in = a slice x[shift:] of a device buffer (base address not 4-byte aligned): the word
+    loads align on the absolute address, and the chunk ending at the buffer end
+    reads no word past its allocation."""
+    lens = [1, 3, 55, 56, 64, 65, 127, 128, 129, 4096, 4097] + [int(v) for v in np.random.default_rng(shift).integers(1, 5000, 150)]
+    cuts = np.cumsum(lens)[:-1]
+    n = int(np.sum(lens))
+    data = synthgen.random_bytes(6, n + shift)
+    base = torch.from_numpy(data).cuda()
+    x = base[shift:]
+    assert x.data_ptr() % 4 != 0 or shift % 4 == 0
+    ch = pkg.Chunker(pkg.Params())
+    got = ch.hash_chunks(x, torch.from_numpy(cuts.astype(np.int64)).cuda())
+    assert np.array_equal(got.cpu().numpy(), oracle.chunk_digests(data[shift:], cuts))
+    # and the chunker itself on the same unaligned slice
+    assert np.array_equal(ch.chunk(x).cpu().numpy().astype(np.uint64), oracle.candidates(data[shift:]))
+
+
 def test_single_chunk_and_fips_message(pkg):
     ch = pkg.Chunker(pkg.Params())
     for m in (b"abc", b"abcdbcdecdefdefgefghfghighijhijkijkljklmklmnlmnomnopnopq", b"a" * 1000000):

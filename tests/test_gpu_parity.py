@@ -337,6 +337,41 @@ def test_marker_le_and_non_pow2_divisor(pkg):
         check_chunk(ch, data)
 
 
+@pytest.mark.parametrize("bounded", [False, True])
+def test_le_marker_dense_rate_lists_sized_by_rate(pkg, bounded):
+    """'<=' marker with r near D (hit rate (r+1)/D up to 1/2): the per-row lists are sized by the
+    set's rate, so bounded mode stays on the parallel size-rule kernels instead of
+    the one-CTA dense walk; exact vs the oracle either way (L249-L251)."""
+    data = synthgen.random_bytes(41, (6 << 20) + 333)
+    for D, r in ((8192, 4095), (8192, 511), (256, 127)):
+        p = pkg.Params(divisor=D, magic=r, marker=1, min_size=64 if bounded else 0,
+                       max_size=4096 if bounded else 0)
+        check_chunk(pkg.Chunker(p), data)
+
+
+def test_two_streams_one_ctx_are_ordered(pkg):
+    """Two one-shot calls on two different streams of one ctx (shared scratch and aux) give the
+    same results as on one stream: the library orders them."""
+    a = synthgen.random_bytes(51, (32 << 20) + 5)
+    b = synthgen.random_bytes(52, (3 << 20) + 7)
+    ch = pkg.Chunker(pkg.Params())
+    xa, xb = dev(a), dev(b)
+    oa = torch.empty(1 << 16, dtype=torch.int64, device="cuda")
+    ob = torch.empty(1 << 16, dtype=torch.int64, device="cuda")
+    na = torch.zeros(1, dtype=torch.int64, device="cuda")
+    nb = torch.zeros(1, dtype=torch.int64, device="cuda")
+    s1, s2 = torch.cuda.Stream(), torch.cuda.Stream()
+    torch.cuda.synchronize()
+    for _ in range(5):
+        ch.chunk_async(xa, oa, na, stream=s1)
+        ch.chunk_async(xb, ob, nb, stream=s2)
+    torch.cuda.synchronize()
+    ea, eb = oracle.candidates(a), oracle.candidates(b)
+    assert int(na.item()) == ea.size and int(nb.item()) == eb.size
+    assert np.array_equal(oa[:ea.size].cpu().numpy().astype(np.uint64), ea)
+    assert np.array_equal(ob[:eb.size].cpu().numpy().astype(np.uint64), eb)
+
+
 @pytest.mark.parametrize("poly", [LBFS, 0x104C11DB7, 0x20000005, None])   # K63, K32B, K32, K40
 @pytest.mark.parametrize("D", [3, 7, 10000, 3 << 20, 3 << 31, (1 << 40) + 1, 12345678901, (1 << 32) - 1])
 def test_non_pow2_divisor_hot_kernel(pkg, poly, D):

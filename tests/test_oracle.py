@@ -377,3 +377,78 @@ def test_size_bound_from_composes_over_pieces():
             cuts, s, held = oracle.size_bound_from(part, b, b == n, s, held, mn, mx)
             got += cuts.tolist()
         assert got == whole.tolist(), (trial, mn, mx, bounds)
+
+
+# --------------------------------------------------------------------------- sliced oracle runner
+@pytest.mark.parametrize("n,sl,p", [
+    ((3 << 20) + 77, 1 << 20, Params()),
+    ((1 << 20) + 5, 65536, Params(divisor=256, magic=7)),
+    (200000, 4096, Params(divisor=4, magic=3, window=5, poly=0x104C11DB7)),
+    (4096 * 3, 4096, Params(divisor=2, magic=1)),
+])
+def test_candidates_stream_equals_whole(n, sl, p):
+    """oracle.candidates_stream (slices with a w-1 overlap, used for the 16/64 GiB configs) ==
+    oracle.candidates on the whole stream, including candidates at exactly a slice boundary."""
+    whole = oracle.candidates(synthgen.random_bytes(11, n), p)
+    parts, prev_b = [], 0
+    for a, b, c in oracle.candidates_stream(11, n, p, slice_bytes=sl):
+        assert a == prev_b and (c.size == 0 or (c[0] > a and c[-1] <= b))
+        parts.append(c)
+        prev_b = b
+    assert prev_b == n
+    got = np.concatenate(parts)
+    assert np.array_equal(got, whole)
+    # the dense-density parameter sets do hit slice boundaries exactly
+    if p.divisor <= 4:
+        assert any(int(c) % sl == 0 for c in whole)
+
+
+def test_synthgen_fast_filler_matches_numpy_form():
+    for off in (0, 3, 8, 12345, (1 << 36) + 5):
+        for n in (0, 1, 7, 100, (3 << 20) | 5):
+            assert np.array_equal(synthgen.random_bytes(9, n, off), synthgen.random_bytes_fast(9, n, off))
+
+
+# --------------------------------------------------------------------------- matching index (f3)
+def test_index_hand_built_duplicates():
+    """oracle.Index against hand-worked set semantics (a chunk is new iff
+    its hash was not seen before): digests A B A C B A with lengths 1..6 -> flags 1 1 0 1 0 0,
+    3 new chunks of 1 + 2 + 4 bytes; a second batch C D -> 0 1."""
+    A, B, C, D = (np.full(32, v, np.uint8) for v in (1, 2, 3, 4))
+    ix = oracle.Index()
+    f = ix.insert(np.stack([A, B, A, C, B, A]), [1, 2, 3, 4, 5, 6])
+    assert f.tolist() == [1, 1, 0, 1, 0, 0]
+    assert (ix.chunks, ix.new_chunks, ix.new_bytes) == (6, 3, 7)
+    f = ix.insert(np.stack([C, D]), [10, 20])
+    assert f.tolist() == [0, 1]
+    assert (ix.chunks, ix.new_chunks, ix.new_bytes) == (8, 4, 27)
+    # digests differing only in the last byte are distinct keys
+    A2 = A.copy(); A2[31] ^= 1
+    assert ix.insert(np.stack([A2]), [5]).tolist() == [1]
+
+
+def test_index_snapshot_construction_closed_form():
+    """Backup-style snapshots built at the digest level (the paper's similarity-table scheme,
+    L1299-L1307): snapshot 0 = M distinct digests; snapshot s replaces each entry independently
+    with probability p_s by a fresh digest.  By construction the distinct digests number
+    M + sum_s R_s (R_s = entries replaced in snapshot s), so new_chunks and new_bytes are known
+    without the index; also equal to numpy's unique row count."""
+    rng = np.random.default_rng(5)
+    M = 4000
+    master = rng.integers(0, 256, (M, 32), dtype=np.uint8)
+    lengths = rng.integers(1, 20000, M)
+    ix = oracle.Index()
+    ix.insert(master, lengths)
+    exp_new, exp_bytes, allrows = M, int(lengths.sum()), [master]
+    for s, p in enumerate([0.05, 0.10, 0.15, 0.20, 0.25, 0.05, 0.10, 0.15, 0.20], start=1):
+        snap = master.copy()
+        rep = rng.random(M) < p
+        snap[rep] = rng.integers(0, 256, (int(rep.sum()), 32), dtype=np.uint8)
+        flags = ix.insert(snap, lengths)
+        assert np.array_equal(flags.astype(bool), rep)
+        exp_new += int(rep.sum()); exp_bytes += int(lengths[rep].sum())
+        allrows.append(snap)
+    assert (ix.new_chunks, ix.new_bytes, ix.chunks) == (exp_new, exp_bytes, 10 * M)
+    assert np.unique(np.concatenate(allrows), axis=0).shape[0] == exp_new
+    # dedup ratio = logical / unique: 10 M / (M + sum R_s) ~ 10 / (1 + sum p) = 4.44
+    assert abs(10 * M / exp_new - 10 / (1 + 1.25)) < 0.15

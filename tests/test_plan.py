@@ -79,7 +79,7 @@ def check(m, path, addr, p_begin, t_begin, t_end, divisor=8192):
         assert m["ngroups"] == -(-m["n_head"] // GEN_THREADS)
         longest = m["head_seg"]
     assert m["ngroups"] <= MAX_GROUPS
-    assert m["cap"] == min(256, 2 * longest // divisor + 16)
+    assert m["cap"] == min(4096, 2 * longest // divisor + 16)
 
 
 @pytest.mark.parametrize("path", [K63, K32, GENERIC])

@@ -14,6 +14,9 @@ ncu --metrics gpu__time_duration.sum --clock-control none -c 400 --csv --log-fil
 ncu --set full --clock-control none --import-source on -k regex:k1_bulk -s 3 -c 1 -o gpurun_out/prof_k1_$TAG \
     python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu --no-extra > gpurun_out/ncu_full_$TAG.log 2>&1
 tail -2 gpurun_out/ncu_full_$TAG.log
+# the summary and the traffic JSON from the SAME report (bench.py's roofline.traffic cites it)
+python tools/ncu_summary.py gpurun_out/prof_k1_$TAG.ncu-rep > gpurun_out/k1_bulk_ncu_full_$TAG.txt 2>&1
+python tools/ncu_traffic.py gpurun_out/prof_k1_$TAG.ncu-rep profiles/${TAG}_k1_bulk_ncu_full.txt > gpurun_out/k1_traffic_$TAG.json 2>&1
 if [ "$3" == "k32" ]; then
   ncu --set full --clock-control none --import-source on -k regex:k1_bulk -s 3 -c 1 -o gpurun_out/prof_k1k32_$TAG \
       python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu --no-extra --variant k32 > /dev/null 2>&1
