@@ -17,6 +17,16 @@ time (CUDA events).  `e2e` = the same metric through the C ABI's host-fed mode: 
 buffers -> shred_feed (async H2D on the ctx's copy stream, double-buffered device slots) ->
 shred_flush -> D2H of the cut offsets, all inside the timed region.
 
+N > 1 (torchrun, one rank per GPU): configs[3] as strong scaling (BASELINE.json: "64 GiB random
+stream byte-range sharded with halo across 1/2/4/8 B200").  The 2^36-byte stream (SplitMix64
+seed 5) is split into N byte ranges at 4 KiB-aligned starts; each rank generates its range and
+the 47 bytes before it on its GPU (untimed).  One step = dist.chunk_sharded on every rank (the
+shard's candidates + the C2 count all-gather over NCCL; no host synchronisation), timed with
+CUDA events, max over ranks.  `value` = 2^36 B / max-rank time per step.  `t1_ms` = the same
+stream chunked whole on rank 0's GPU alone (the N = 1 time of this workload).  `--weak` keeps the
+round-1 weak-scaling mode (configs[1] per rank).  N = 1 also reports `config3_64gib` (the whole
+stream on one GPU) beside the configs[1] headline.
+
 --impl reference: the CPU oracle (oracle/, R2 direct per-window reduction, all host cores) on
 a bounded sample of the same workload per step; rank 0 only.
 """
@@ -62,6 +72,18 @@ def config(n_gpus, per_rank_bytes):
             "bytes_per_step_per_gpu": per_rank_bytes,
             "l2": "inputs (1 GiB each) larger than the 126 MB L2; no flush",
             "parallelism": f"byte-range shards x{n_gpus}, count all-gather (NCCL)" if n_gpus > 1 else "1 GPU"}
+
+
+STREAM3 = 1 << 36          # configs[3]: 64 GiB
+
+
+def config3(n_gpus):
+    return {"workload": "configs[3]: 64 GiB (2^36 B) SplitMix64 stream (seed 5), byte-range sharded with a "
+                        "47-B halo across the ranks (4 KiB-aligned starts), device-resident",
+            "params": "P=0xbfe6b8a5bf378d83 (deg 63), w=48, D=8192, r=0x78, min=0, max=inf",
+            "bytes_per_step": STREAM3, "bytes_per_step_per_gpu": STREAM3 // n_gpus,
+            "l2": "shards (>= 8 GiB) larger than the 126 MB L2; no flush",
+            "parallelism": f"byte-range shards x{n_gpus}, C2 count all-gather (NCCL)"}
 
 
 # ------------------------------------------------------------------------------- clocks (NVML)
@@ -199,14 +221,18 @@ def run_reference(args, rank, world):
     oracle.build()
     cores = len(os.sched_getaffinity(0))
     per_rank = 2 * GiB
-    # each step: a bounded sample of the workload (alternating base / edited-version slices)
-    cal = synthgen.random_bytes(2, 8 << 20)
+    # each step: a bounded sample of the workload (N = 1: alternating base / edited-version slices
+    # of configs[1]; N > 1: consecutive slices of the configs[3] stream, seed 5)
+    cal = synthgen.random_bytes_fast(2, 8 << 20)
     rate, _, _ = oracle_rate(cal, cores)
     n = int(min(256 << 20, max(8 << 20, rate * 1e9 * 2.0)))
     n -= n % 4096
-    base = synthgen.random_bytes(2, n)
-    ed, _ = synthgen.edited(base, 3, n_edits=max(1, min(100, n // (1 << 20))), min_gap=8192)
-    samples = [base, ed]
+    if world == 1:
+        base = synthgen.random_bytes_fast(2, n)
+        ed, _ = synthgen.edited(base, 3, n_edits=max(1, min(100, n // (1 << 20))), min_gap=8192)
+        samples = [base, ed]
+    else:
+        samples = [synthgen.random_bytes_fast(5, n, 0), synthgen.random_bytes_fast(5, n, n)]
     for i in range(args.warmup):
         oracle.candidates(samples[i % 2], oracle.Params(), 2, cores)
     t0 = time.perf_counter()
@@ -219,13 +245,179 @@ def run_reference(args, rank, world):
     v = tot / dt / 1e9
     line = {"metric": METRIC, "value": round(v, 4), "unit": "GB/s", "n_gpus": world, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": round(dt / args.steps * 1e3, 3), "higher_is_better": True,
-            "scaling": "weak", "vs_baseline": None, "dtype": "u8", "data": "synthetic",
-            "config": config(world, per_rank), "impl": "reference",
+            "scaling": "weak" if world == 1 else "strong", "vs_baseline": None, "dtype": "u8", "data": "synthetic",
+            "config": config(world, per_rank) if world == 1 else config3(world), "impl": "reference",
             "cpu_baseline": {"value": round(v, 4), "unit": "GB/s", "cores": cores, "kind": "oracle",
-                             "sample": f"each step = {n / 2**20:.0f} MiB of the base file or its edited "
-                                       f"version (alternating), R2 oracle, {cores} threads"},
+                             "sample": (f"each step = {n / 2**20:.0f} MiB of the base file or its edited "
+                                        f"version (alternating)" if world == 1 else
+                                        f"each step = {n / 2**20:.0f} MiB of the configs[3] stream (seed 5)")
+                                       + f", R2 oracle, {cores} threads"},
             "e2e": {"value": round(v, 4), "unit": "GB/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
+
+
+# ------------------------------------------------------------------------------- N > 1: configs[3]
+def run_scaled(args, rank, world, local):
+    """configs[3] strong scaling (see the module docstring)."""
+    import torch
+    import torch.distributed as dist
+    import paper_conf_fast_bhatotiarv12_b200 as pkg
+    from paper_conf_fast_bhatotiarv12_b200 import dist as sd
+
+    backend = os.environ.get("SHRED_BENCH_BACKEND", "nccl")        # test-only override (gloo)
+    local = int(os.environ.get("SHRED_BENCH_DEVICE", local))
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if backend == "nccl":
+        dist.init_process_group("nccl", device_id=dev)
+    else:
+        dist.init_process_group(backend)
+    total = int(os.environ.get("SHRED_BENCH_STREAM", STREAM3))     # test-only override of 2^36
+    start, end = sd.shard_bounds(total, world, rank)
+    halo = sd.halo_of(start)
+    x = torch.empty(end - start + halo, dtype=torch.uint8, device=dev)
+    pkg.synth_fill(x, 5, start - halo)                              # untimed: shard + halo on device
+    ch = pkg.Chunker(pkg.Params(), device=local)
+    cap = sd._expected_cap(ch, end - start)
+    stream = torch.cuda.current_stream()
+
+    def maxr(v):                                                     # max over ranks of a float
+        t = torch.tensor([v], dtype=torch.float64, device=dev)
+        if backend != "nccl":
+            t = t.cpu()
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        return float(t.item())
+
+    for _ in range(args.warmup):
+        res = sd.chunk_sharded(x, halo, start, total, ch, cap=cap)
+    torch.cuda.synchronize()
+    n_total = res.total                                             # (synchronises; outside timing)
+    assert res.local.numel() == int(res.counts[rank])
+    dist.barrier()
+    torch.cuda.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    l0 = ch.launches
+    ch.profile(True)
+    with ClockSampler(local) as clk:
+        e0.record(stream)
+        for _ in range(args.steps):
+            sd.chunk_sharded(x, halo, start, total, ch, cap=cap)
+        e1.record(stream)
+        torch.cuda.synchronize()
+    ch.profile(False)
+    launches = ch.launches - l0
+    k_ms, k_n, k_bytes = ch.profile_read()
+    ms = maxr(e0.elapsed_time(e1))
+    value = total * args.steps / (ms * 1e-3) / 1e9
+    hbm, hbm_src = peaks()
+    k_avg = k_ms / max(1, k_n)
+    achieved = (k_bytes / max(1, k_n)) / (k_avg * 1e-3) / 1e9 if k_n else None
+    line = {"metric": METRIC, "value": round(value, 2), "unit": "GB/s", "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": round(ms / args.steps, 4), "higher_is_better": True,
+            "scaling": "strong", "vs_baseline": None, "dtype": "u8", "data": "synthetic",
+            "config": config3(world), "hbm_frac": round(value / world / hbm, 4),
+            "tG_ms": round(ms / args.steps, 4), "candidates_total": n_total,
+            "roofline": {"bound": "hbm", "achieved": round(achieved, 1) if achieved else None, "peak": hbm,
+                         "unit": "GB/s", "frac": round(achieved / hbm, 4) if achieved else None, "traffic": None,
+                         "kernel": "k1_bulk<K63> (rank 0)", "launches": k_n, "avg_launch_ms": round(k_avg, 4),
+                         "peak_source": hbm_src},
+            "clocks": clk.result(), "gpu_launches": launches}
+    try:
+        with open(os.path.join(ROOT, "tests", "golden", "oracle_fullsize.json")) as f:
+            g = json.load(f)["configs3"]
+        if g["n"] == total:
+            line["matches_oracle_count"] = n_total == g["candidates"]["count"]
+    except Exception:
+        pass
+    # bounded mode (min 2048 / max 65536) with the distributed size rule ("chain") as a side line
+    if not args.no_extra:
+        chb = pkg.Chunker(pkg.Params(min_size=2048, max_size=65536), device=local)
+        rb = sd.chunk_sharded(x, halo, start, total, chb, cap=cap)
+        torch.cuda.synchronize()
+        dist.barrier()
+        b0, b1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        b0.record(stream)
+        for _ in range(max(2, args.steps // 4)):
+            rb = sd.chunk_sharded(x, halo, start, total, chb, cap=cap)
+        b1.record(stream)
+        torch.cuda.synchronize()
+        bms = maxr(b0.elapsed_time(b1)) / max(2, args.steps // 4)
+        line["bounded_2048_65536"] = {"value": round(total / (bms * 1e-3) / 1e9, 2), "unit": "GB/s",
+                                      "rounds": rb.rounds, "mode": "chain (distributed size rule)",
+                                      "note": "includes one host synchronisation per step (the chain's convergence check)"}
+        del chb
+    # e2e: every rank feeds (a bounded sample of) its shard from pinned host memory through the
+    # C ABI (shred_feed + shred_flush + D2H of the cuts); aggregate bytes / max-rank time
+    if not args.no_e2e:
+        import synthgen
+        m = min(end - start, 2 * GiB)
+        pin = torch.empty(m, dtype=torch.uint8).pin_memory()
+        synthgen.fill_fast(pin.numpy(), 5, start, threads=max(1, len(os.sched_getaffinity(0)) // world))
+        che = pkg.Chunker(pkg.Params(), device=local)
+        che.set_ring(2, 256 << 20)
+        ecap = m // 2048 + 65536
+        eo = torch.empty(ecap, dtype=torch.int64, device=dev)
+        en = torch.zeros(1, dtype=torch.int64, device=dev)
+        en_h = torch.zeros(1, dtype=torch.int64).pin_memory()
+        res_h = torch.empty(ecap, dtype=torch.int64).pin_memory()
+        fo = torch.empty(1, dtype=torch.int64, device=dev)
+        fn = torch.zeros(1, dtype=torch.int64, device=dev)
+
+        def e2e_step():
+            che.feed_async(pin, eo, en)
+            pkg.lib().shred_flush(che._ctx, fo.data_ptr(), 1, fn.data_ptr(), stream.cuda_stream)
+            en_h.copy_(en, non_blocking=True)
+            stream.synchronize()
+            a = int(en_h[0])
+            res_h[:a].copy_(eo[:a], non_blocking=True)
+            return a
+
+        for _ in range(2):
+            e2e_step()
+        torch.cuda.synchronize()
+        dist.barrier()
+        s0, s1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        s0.record(stream)
+        es = max(2, args.steps // 4)
+        for _ in range(es):
+            a = e2e_step()
+        s1.record(stream)
+        torch.cuda.synchronize()
+        ems = maxr(s0.elapsed_time(s1))
+        line["e2e"] = {"value": round(world * m * es / (ems * 1e-3) / 1e9, 3), "unit": "GB/s",
+                       "h2d_bytes_per_step": m, "d2h_bytes_per_step": 8 * a + 8,
+                       "sample": f"each rank feeds the first {m / 2**30:.2f} GiB of its shard from pinned host memory",
+                       "api": "shred_feed(pinned host, 2 x 256 MiB device slots) + shred_flush + D2H of cuts"}
+        del pin, che
+    # t1: the whole stream on rank 0's GPU alone (same call path, one shard = the stream)
+    dist.barrier()
+    if rank == 0 and not args.no_extra:
+        try:
+            del x
+            torch.cuda.empty_cache()
+            xx = torch.empty(total, dtype=torch.uint8, device=dev)
+            pkg.synth_fill(xx, 5, 0)
+            o1 = torch.empty(sd._expected_cap(ch, total), dtype=torch.int64, device=dev)
+            n1 = torch.zeros(1, dtype=torch.int64, device=dev)
+            for _ in range(2):
+                ch.candidates_range_async(xx, 0, 0, total, o1, n1)
+            torch.cuda.synchronize()
+            t0_, t1_ = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            t0_.record(stream)
+            for _ in range(3):
+                ch.candidates_range_async(xx, 0, 0, total, o1, n1)
+            t1_.record(stream)
+            torch.cuda.synchronize()
+            line["t1_ms"] = round(t0_.elapsed_time(t1_) / 3, 4)
+            line["t1_candidates"] = int(n1.item())
+            del xx
+        except Exception as e:
+            line["t1_ms"] = None
+            line["t1_error"] = repr(e)
+    dist.barrier()
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    dist.destroy_process_group()
 
 
 # ------------------------------------------------------------------------------- our arm
@@ -239,6 +431,7 @@ def main():
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--no-extra", action="store_true", help="skip the bounded / k32 side measurements")
     ap.add_argument("--cpu-only", action="store_true", help=argparse.SUPPRESS)   # internal: fresh-process CPU leg
+    ap.add_argument("--weak", action="store_true", help="N > 1: round-1 weak scaling (configs[1] per rank)")
     ap.add_argument("--variant", default="paper", choices=["paper", "k32"],
                     help="profiling aid: k32 = P 0x104C11DB7 on the main path (not the headline)")
     args = ap.parse_args()
@@ -250,6 +443,8 @@ def main():
         return
     if args.impl == "reference":
         return run_reference(args, rank, world)
+    if world > 1 and not args.weak:
+        return run_scaled(args, rank, world, local)
     # host-core baselines first, in a fresh process, before this process creates a CUDA context
     cpu = cpu_measurements_subprocess() if (not args.no_cpu and rank == 0 and world == 1) else None
 
@@ -491,7 +686,16 @@ def main():
             c32 = pkg.Chunker(pkg.Params(poly=0x104C11DB7), device=local)
             v32 = timed(c32, base)
             line["k32_variant"] = {"value": round(v32, 2), "unit": "GB/s", "hbm_frac": round(v32 / hbm, 4),
-                                   "params": "P=0x104C11DB7 (deg 32, irreducible), other params as paper"}
+                                   "params": "P=0x104C11DB7 (deg 32, irreducible), other params as paper",
+                                   "mode": c32.mode}
+            # the multiply-reduction u32 kernel (MODE_K32T): an irreducible trinomial whose top-byte
+            # reduction is one integer product (no T lookup); ALU-bound (profiles/r02_k32_ab.txt)
+            c3t = pkg.Chunker(pkg.Params(poly=0x80002001), device=local)
+            v3t = timed(c3t, base)
+            line["k32t_variant"] = {"value": round(v3t, 2), "unit": "GB/s", "hbm_frac": round(v3t / hbm, 4),
+                                    "params": "P=x^31+x^13+1 (0x80002001, irreducible trinomial), other params as paper",
+                                    "mode": c3t.mode}
+            del c3t
             # content sensitivity. Text-like bytes (words from a fixed
             # 1,000-word list; skewed outgoing bytes for the U lookups), 64 MiB generated on the
             # host and tiled to 256 MiB on the device; paper params on the same ctx.
@@ -576,6 +780,37 @@ def main():
                                    "unit": "GB/s", "chunks": int(n0.item()) + 1,
                                    "chunk_plus_hash": round(3 * base.numel() / (h1.elapsed_time(h2) * 1e-3) / 1e9, 2),
                                    "note": "SURVEY §8(f) f2: SHA-256 per chunk of the 1 GiB base file"}
+            # configs[3] on one GPU: the whole 2^36-byte stream (seed 5) in one call; the N = 1
+            # time of the strong-scaling workload that `bench.py --gpus N` runs at N > 1
+            try:
+                free, _ = torch.cuda.mem_get_info(dev)
+                if free > STREAM3 + (8 << 30):
+                    x3 = torch.empty(STREAM3, dtype=torch.uint8, device=dev)
+                    pkg.synth_fill(x3, 5, 0)
+                    o3 = torch.empty(STREAM3 // 4096 + 65536, dtype=torch.int64, device=dev)
+                    n3 = torch.zeros(1, dtype=torch.int64, device=dev)
+                    for _ in range(2):
+                        ch.chunk_async(x3, o3, n3)
+                    torch.cuda.synchronize()
+                    q0.record(stream)
+                    for _ in range(3):
+                        ch.chunk_async(x3, o3, n3)
+                    q1.record(stream)
+                    torch.cuda.synchronize()
+                    t3 = q0.elapsed_time(q1) / 3
+                    c3 = {"ms": round(t3, 3), "value": round(STREAM3 / (t3 * 1e-3) / 1e9, 2), "unit": "GB/s",
+                          "candidates": int(n3.item()),
+                          "note": "configs[3] stream whole on 1 GPU (t1 of the N > 1 strong-scaling runs)"}
+                    try:
+                        with open(os.path.join(ROOT, "tests", "golden", "oracle_fullsize.json")) as f:
+                            c3["matches_oracle_count"] = c3["candidates"] == json.load(f)["configs3"]["candidates"]["count"]
+                    except Exception:
+                        pass
+                    line["config3_64gib"] = c3
+                    del x3, o3
+                    torch.cuda.empty_cache()
+            except Exception as e:
+                line["config3_64gib"] = {"error": repr(e)}
         except Exception as e:  # side numbers must never break the headline line
             line["extra_error"] = repr(e)
 

@@ -99,6 +99,11 @@ void        shred_destroy(shred_ctx *ctx);
 const char *shred_strerror(int code);
 const char *shred_last_error(const shred_ctx *ctx);   /* detail incl. the CUDA error string  */
 int         shred_path(const shred_ctx *ctx);         /* SHRED_PATH_* chosen at init          */
+/* The hot kernel's state mode (diagnostics): 1 K63 (u64 state, deg 41..63), 5 K40 (deg 33..40),
+   2 K32 (u32 state, T by table), 4 K32B (u32, whole-byte top byte: deg 8/16/24/32), 6 K32T (u32,
+   T as one integer product: P = x^k + Q with Q's terms >= 8 apart and below k - 7, e.g. the
+   trinomial x^31 + x^13 + 1; '==' and '<=' with D = 2^m), 3 generic. */
+int         shred_kernel_mode(const shred_ctx *ctx);
 int         shred_get_params(const shred_ctx *ctx, shred_params *out);
 
 /* An output capacity that can never overflow for `len` input bytes:
@@ -140,6 +145,16 @@ int shred_size_bound(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, ui
 int shred_size_bound_state(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_cand, uint64_t end,
                            int fin, const uint64_t state_in[2], uint64_t *d_out, uint64_t cap,
                            uint64_t *n_out, uint64_t *d_state_out, shred_stream_t stream);
+
+/* The same with everything the host does not need to know kept in device memory, so rounds of
+   the distributed size rule chain on the stream without a host synchronisation: the candidate
+   count is read from d_n_cand (device u64; at most n_cand_max, which sizes the launch), the
+   entry state from d_state_in (device, 2 x u64 {s, held}).  Otherwise as above.  d_state_in and
+   d_state_out may be the same array. */
+int shred_size_bound_state_dev(shred_ctx *ctx, const uint64_t *d_cand, const uint64_t *d_n_cand,
+                               uint64_t n_cand_max, uint64_t end, int fin, const uint64_t *d_state_in,
+                               uint64_t *d_out, uint64_t cap, uint64_t *n_out, uint64_t *d_state_out,
+                               shred_stream_t stream);
 
 /* Streaming with carried window and size-rule state (§4.1-§4.2: pinned
    buffers, async transfers, multi-buffering).  `in` is device memory or page-locked host
@@ -215,6 +230,10 @@ int shred_check_params(const shred_params *p, int *path_out, int *marker_kind_ou
    edge CTA}.  SHRED_EINVAL on inconsistent arguments. */
 int shred_debug_plan(int path, int small_ok, int sm_count, uint64_t src_addr, uint64_t p_begin,
                      uint64_t t_begin, uint64_t t_end, uint64_t divisor, uint64_t out[16]);
+/* Test hook (host logic, no GPU): 1 if the K32T kernel mode applies to poly (deg <= 32 and
+   P = x^k + Q with Q's terms >= 8 apart and below k - 7), with *mult = Q + 2^k mod 2^32, the
+   integer multiplier that gives T[t] = t(x) x^k mod P ^ (t << k mod 2^32) as t * mult mod 2^32. */
+int shred_debug_tprod(uint64_t poly, uint32_t *mult);
 int shred_profile_read(shred_ctx *ctx, double *ms, uint64_t *launches, uint64_t *bytes);
 
 #ifdef __cplusplus

@@ -67,6 +67,7 @@ def lib() -> ctypes.CDLL:
             "shred_strerror": (ctypes.c_char_p, [cint]),
             "shred_last_error": (ctypes.c_char_p, [vp]),
             "shred_path": (cint, [vp]),
+            "shred_kernel_mode": (cint, [vp]),
             "shred_get_params": (cint, [vp, P]),
             "shred_max_cuts": (u64, [vp, u64]),
             "shred_chunk": (cint, [vp, vp, u64, vp, u64, vp, vp]),
@@ -81,6 +82,7 @@ def lib() -> ctypes.CDLL:
             "shred_hash_chunks": (cint, [vp, vp, u64, vp, vp, vp, u64, vp]),
             "shred_index_reset": (cint, [vp, u64]),
             "shred_size_bound_state": (cint, [vp, vp, u64, u64, cint, ctypes.POINTER(u64), vp, u64, vp, vp, vp]),
+            "shred_size_bound_state_dev": (cint, [vp, vp, vp, u64, u64, cint, vp, vp, u64, vp, vp, vp]),
             "shred_index_insert": (cint, [vp, vp, vp, vp, u64, u64, vp, vp]),
             "shred_index_stats": (cint, [vp, ctypes.POINTER(u64)]),
             "shred_profile": (cint, [vp, cint]),
@@ -146,6 +148,12 @@ class Chunker:
     @property
     def path(self) -> str:
         return PATH_NAMES.get(lib().shred_path(self._ctx), "?")
+
+    @property
+    def mode(self) -> str:
+        """The hot kernel's state mode (k63, k40, k32, k32b, k32t, generic)."""
+        return {1: "k63", 2: "k32", 3: "generic", 4: "k32b", 5: "k40", 6: "k32t"}.get(
+            lib().shred_kernel_mode(self._ctx), "?")
 
     @property
     def launches(self) -> int:
@@ -222,6 +230,28 @@ class Chunker:
         if p.min_size:
             cap = min(cap, span // p.min_size + 2)
         return max(1, cap)
+
+    def candidates_range_async(self, x: torch.Tensor, halo: int, start: int, total_len: int,
+                               out: torch.Tensor, n_out: torch.Tensor, stream=None) -> None:
+        """Enqueue shred_candidates_range; no host synchronisation (n_out[0] = the true count,
+        min(count, len(out)) offsets written)."""
+        assert x.is_cuda and x.dtype == torch.uint8 and x.is_contiguous()
+        rc = lib().shred_candidates_range(self._ctx, x.data_ptr(), halo, start, x.numel() - halo, total_len,
+                                          out.data_ptr(), out.numel(), n_out.data_ptr(), _stream(stream))
+        self._check(rc, "shred_candidates_range")
+
+    def size_bound_state_dev(self, cands: torch.Tensor, n_cand: torch.Tensor, end: int, fin: bool,
+                             state_in: torch.Tensor, out: torch.Tensor, n_out: torch.Tensor,
+                             state_out: torch.Tensor, stream=None) -> None:
+        """Enqueue shred_size_bound_state_dev: the candidate count (n_cand[0], clamped to
+        len(cands)) and the entry state {s, held} (state_in) are device values; exit state to
+        state_out.  No host synchronisation."""
+        for t in (cands, n_cand, state_in, out, n_out, state_out):
+            assert t.is_cuda and t.dtype == torch.int64 and t.is_contiguous()
+        rc = lib().shred_size_bound_state_dev(self._ctx, cands.data_ptr(), n_cand.data_ptr(), cands.numel(), end,
+                                              int(fin), state_in.data_ptr(), out.data_ptr(), out.numel(),
+                                              n_out.data_ptr(), state_out.data_ptr(), _stream(stream))
+        self._check(rc, "shred_size_bound_state_dev")
 
     def size_bound(self, cands: torch.Tensor, total_len: int, cap: int | None = None) -> torch.Tensor:
         assert cands.is_cuda and cands.dtype == torch.int64 and cands.is_contiguous()

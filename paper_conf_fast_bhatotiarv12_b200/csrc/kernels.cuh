@@ -42,7 +42,10 @@ namespace shred {
 
 // K63: u64 state, deg 41..63; K40: u64 state, deg 33..40; K32: u32 state, deg 9..32;
 // K32B: u32 state, deg 8/16/24/32 (whole-byte top byte)
-enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3, MODE_K32B = 4, MODE_K40 = 5 };
+// K32T: u32 state, deg 9..32, P = x^k + Q with the terms of Q at least 8 apart and below k-7:
+// the reduction of the top byte, t(x) Q(x), is then an integer product (no carries between the
+// shifted copies of t), so T costs one IMAD instead of a shared-memory lookup.
+enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3, MODE_K32B = 4, MODE_K40 = 5, MODE_K32T = 6 };
 
 #ifndef SHRED_STAGES
 #define SHRED_STAGES 2   // A/B (profiles/r01_ab_variants.txt): 2 stages 1,879 GB/s > 3: 1,861 > 4: 1,854
@@ -454,6 +457,7 @@ struct BulkCtx {
     uint32_t tmul;      // 2^(32-m): (f_lo * tmul) keeps the low m bits at the top
     uint32_t rsh;       // r << (32-m)
     uint32_t tsel;      // K32B: PRMT selector 0x55s4 placing byte s = (k-8)/8 of f at bits 8..15
+    uint32_t tshr, tprod;       // K32T: k - 8, M = Q + 2^k mod 2^32
     // MK_DIV (any D = d 2^s, s < 32): f mod D == r  <=>  D | (f + D - r)  (no overflow: f < 2^63,
     // D - r <= 2^63)  <=>  rotr64((f + D - r) * d^-1 mod 2^64, s) <= floor((2^64 - 1) / D)
     uint64_t dc;        // D - r
@@ -502,8 +506,32 @@ __device__ __forceinline__ void step32(uint32_t &f, uint32_t in, uint32_t pop, c
     f = __byte_perm(f, in, 0x2104u + K) ^ T ^ U;
 }
 
+// One byte step, K32T: t = f >> (k-8) (SHF), T = t * M mod 2^32 with M = Q + 2^k mod 2^32 (the
+// carry-free product t(x) Q(x) plus the cancel term t << k of the bits the shift leaves at k..31),
+// f <- (f << 8 mod 2^32) ^ B ^ T ^ U[o].  The T lookup (and its 29-cycle LDS latency on the
+// dependency chain) is gone; only U is looked up.
+#ifndef SHRED_K32T_HI
+#define SHRED_K32T_HI 0   // 1: t = mulhi(f, 2^(40-k)) on the FMA pipe instead of SHF on the ALU pipe
+#endif
+template <int K>
+__device__ __forceinline__ void step32t(uint32_t &f, uint32_t in, uint32_t pop, const BulkCtx &c) {
+    const uint32_t T = (SHRED_K32T_HI ? __umulhi(f, c.mhi) : (f >> c.tshr)) * c.tprod;
+    const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
+    const uint32_t U = lds32(c.tab + oi);
+    f = __byte_perm(f, in, 0x2104u + K) ^ T ^ U;
+}
+
 template <int MODE>
 struct State;
+template <> struct State<MODE_K32T> {
+    uint32_t f = 0;
+    __device__ __forceinline__ void set(uint64_t v) { f = (uint32_t)v; }
+    template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
+        step32t<K>(f, in, pop, c);
+    }
+    __device__ __forceinline__ uint32_t low() const { return f; }
+    __device__ __forceinline__ uint64_t full() const { return f; }
+};
 template <> struct State<MODE_K63> {
     uint32_t fl = 0, fh = 0;
     __device__ __forceinline__ void set(uint64_t v) { fl = (uint32_t)v; fh = (uint32_t)(v >> 32); }
@@ -616,7 +644,7 @@ static __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t
 #else
 #define SHRED_MARK(ch, q)                                                                   \
     m[ch] = (MK == MK_DIV) ? or_if_div<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
-          : (MK == MK_REM && (MODE == MODE_K32 || MODE == MODE_K32B))                            \
+          : (MK == MK_REM && (MODE == MODE_K32 || MODE == MODE_K32B || MODE == MODE_K32T))       \
                 ? or_if_rem32<(1u << (4 * J + q))>(m[ch], st[ch].low(), c)                            \
           : (MK == MK_REM) ? or_if_rem<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
                            : or_if_marker<(1u << (4 * J + q)), MK>(m[ch], st[ch].low(), c);
@@ -675,6 +703,7 @@ __device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d
 
 struct BulkConst {
     uint32_t mhi, m256, tmul, rsh, tsel;
+    uint32_t tshr, tprod;      // K32T (BulkCtx)
     uint64_t dc, dinv, dlim;   // MK_DIV constants (BulkCtx)
     uint32_t dsh;
     uint64_t rm, rd, rlo, rspan;   // MK_REM constants (BulkCtx)
@@ -821,6 +850,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         c.laneU = 128u + (uint32_t)lane * 4u;
     }
     c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh; c.tsel = K.tsel;
+    c.tshr = K.tshr; c.tprod = K.tprod;
     c.dc = K.dc; c.dinv = K.dinv; c.dlim = K.dlim; c.dsh = K.dsh;
     c.rm = K.rm; c.rd = K.rd; c.rlo = K.rlo; c.rspan = K.rspan; c.rsh2 = K.rsh2;
 
@@ -950,8 +980,8 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
 // A hot-kernel instance; pick_k1 / pick_k1_small (k1_inst.cu) map parameters to instances.
 typedef void (*K1Fn)(const __grid_constant__ CUtensorMap, const uint4 *, const GenTables *, Job,
                      DevParams, BulkConst);
-K1Fn pick_k1(int k, bool byteidx, int wch, int mk, bool fn);
-K1Fn pick_k1_small(int k, bool byteidx, int wch, int mk, bool fn);
+K1Fn pick_k1(int k, bool byteidx, int wch, int mk, bool fn, bool tprod = false);
+K1Fn pick_k1_small(int k, bool byteidx, int wch, int mk, bool fn, bool tprod = false);
 
 #ifndef SHRED_K1_ONLY
 // ------------------------------------------------------------------------------ k_total
@@ -1094,6 +1124,12 @@ __global__ void k_write_u64(uint64_t *p, uint64_t v) {
 // Entry / exit of shred_size_bound_state.
 __global__ void k_state_in(Aux *aux, uint64_t s, uint64_t held) {
     pdl_entry();
+    aux->total = 0; aux->last_cand = 0; aux->out_pos = 0; aux->dense = 0;
+    aux->s = s; aux->held = held; aux->held_val = held ? s : 0;
+}
+__global__ void k_state_in_dev(Aux *aux, const uint64_t *state) {
+    pdl_entry();
+    const uint64_t s = state[0], held = state[1] ? 1ull : 0ull;
     aux->total = 0; aux->last_cand = 0; aux->out_pos = 0; aux->dense = 0;
     aux->s = s; aux->held = held; aux->held_val = held ? s : 0;
 }

@@ -91,6 +91,9 @@ void byte_times_xpow(uint64_t P, int k, uint64_t e, uint64_t out[256]) {
 #ifndef SHRED_EDGE_GS
 #define SHRED_EDGE_GS 16  // edge-CTA head/tail segment: each is a chain of w-1 + GS dependent steps
 #endif
+#ifndef SHRED_TPROD
+#define SHRED_TPROD 1     // MODE_K32T for eligible polynomials (0: table modes only, A/B)
+#endif
 #ifndef SHRED_BYTEIDX
 #define SHRED_BYTEIDX 1   // deg 8/16/24/32: PRMT table index (MODE_K32B); 0: IMAD index (MODE_K32)
 #endif
@@ -109,6 +112,7 @@ struct shred_ctx {
     shred_params p{};
     int device = 0;
     int path = 0;
+    int mode = MODE_GENERIC;             // kernels.cuh MODE_* of the hot kernel instance
     int k = 0;
     int mk = MK_EQ;                      // marker kind of the hot kernel (kernels.cuh MK_*)
     DevParams dp{};
@@ -206,6 +210,23 @@ int grow(shred_ctx *ctx, T *&ptr, uint64_t &cap, uint64_t need, const char *what
     if (e != cudaSuccess) { cudaGetLastError(); return fail(ctx, SHRED_ENOMEM, "%s: cudaMalloc(%llu B) failed", what, (unsigned long long)(n * sizeof(T))); }
     cap = n;
     return SHRED_OK;
+}
+
+// MODE_K32T eligibility: deg P = k <= 32 and Q = P - x^k has its terms at least 8 apart and
+// below k - 7, so t(x) Q(x) for a byte t is the integer product t * Q (the shifted copies of t
+// never overlap) of degree < k (no second reduction).  The multiplier adds the cancel term:
+// M = Q + 2^k mod 2^32.
+bool tprod_ok(uint64_t P, int k, uint32_t *mult) {
+    if (k < 9 || k > 32) return false;
+    const uint64_t Q = P ^ (1ull << k);
+    int prev = -100;
+    for (int e = 0; e < k; ++e) {
+        if (!((Q >> e) & 1u)) continue;
+        if (e - prev < 8 || e + 7 >= k) return false;
+        prev = e;
+    }
+    if (mult) *mult = (uint32_t)(Q + (k < 32 ? (1ull << k) : 0ull));
+    return true;
 }
 
 // Validation of shred_params (include/shred.h).
@@ -422,6 +443,9 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         K.m256 = 256u;
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
+        K.tshr = (uint32_t)(ctx->k - 8);
+        K.tprod = 0u;
+        tprod_ok(ctx->p.poly, ctx->k, &K.tprod);
         {   // MK_DIV: D = d 2^s; d^-1 mod 2^64 by Newton's iteration (d odd: d*d = 1 mod 8)
             const uint64_t D = ctx->p.divisor;
             const uint32_t sh = (uint32_t)__builtin_ctzll(D);
@@ -482,7 +506,7 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
     int rc = grow(ctx, ctx->d_sb, ctx->sb_cap, 9 * (nb + 2), "size-rule scratch");
     if (rc) return rc;
     SBArgs A;
-    A.cand = cand; A.n_dev = n_dev; A.n_host = n_host;
+    A.cand = cand; A.n_dev = n_dev; A.n_host = n_host; A.n_cap = nmax;
     A.minsz = ctx->p.min_size; A.maxsz = ctx->p.max_size; A.end = end; A.fin = fin;
     uint64_t *b = ctx->d_sb;
     A.spec_exit = b; A.spec_cnt = b + (nb + 2); A.entry = b + 2 * (nb + 2); A.offs = b + 3 * (nb + 2);
@@ -607,6 +631,7 @@ const char *shred_strerror(int code) {
 
 const char *shred_last_error(const shred_ctx *ctx) { return ctx ? ctx->last_error.c_str() : "no ctx"; }
 int shred_path(const shred_ctx *ctx) { return ctx ? ctx->path : 0; }
+int shred_kernel_mode(const shred_ctx *ctx) { return ctx ? ctx->mode : 0; }
 uint64_t shred_launch_count(const shred_ctx *ctx) { return ctx ? ctx->launches : 0; }
 
 int shred_get_params(const shred_ctx *ctx, shred_params *out) {
@@ -704,7 +729,11 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         const bool byteidx = SHRED_BYTEIDX && ctx->path == SHRED_PATH_K32 && (k == 8 || k == 16 || k == 24 || k == 32);
         const int wch = (int)((p->window + 15) / 16);
         const bool funnel = p->window % 16 != 0;
-        ctx->k1_fn = pick_k1(k, byteidx, wch, ctx->mk, funnel);
+        const bool tprod = SHRED_TPROD && ctx->path == SHRED_PATH_K32 && tprod_ok(p->poly, k, nullptr);
+        ctx->k1_fn = pick_k1(k, byteidx, wch, ctx->mk, funnel, tprod);
+        ctx->mode = tprod && (ctx->mk == MK_EQ || ctx->mk == MK_LE) ? MODE_K32T
+                  : ctx->path == SHRED_PATH_K63 ? (k >= 41 ? MODE_K63 : MODE_K40)
+                  : (byteidx ? MODE_K32B : MODE_K32);
         if (!ctx->k1_fn ||
             cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM) != cudaSuccess)
@@ -713,7 +742,7 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributePreferredSharedMemoryCarveout, SHRED_CARVEOUT);
 #endif
 #ifndef SHRED_NO_SMALL
-        ctx->k1_small_fn = pick_k1_small(k, byteidx, wch, ctx->mk, funnel);
+        ctx->k1_small_fn = pick_k1_small(k, byteidx, wch, ctx->mk, funnel, tprod);
 #endif
         if (ctx->k1_small_fn &&
             cudaFuncSetAttribute(ctx->k1_small_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
@@ -839,6 +868,28 @@ int shred_size_bound_state(shred_ctx *ctx, const uint64_t *d_cand, uint64_t n_ca
     PDL(k_state_in, 1, 1, 0, st, aux, state_in[0], state_in[1] ? 1ull : 0ull);
     LAUNCHED("k_state_in");
     if ((rc = launch_size_bound(ctx, d_cand, nullptr, n_cand, n_cand, end, fin ? 1 : 0, d_out, cap, aux,
+                                nullptr, st))) return rc;
+    PDL(k_state_out, 1, 1, 0, st, aux, d_state_out, n_out, cap);
+    LAUNCHED("k_state_out");
+    return SHRED_OK;
+}
+
+int shred_size_bound_state_dev(shred_ctx *ctx, const uint64_t *d_cand, const uint64_t *d_n_cand,
+                               uint64_t n_cand_max, uint64_t end, int fin, const uint64_t *d_state_in,
+                               uint64_t *d_out, uint64_t cap, uint64_t *n_out, uint64_t *d_state_out,
+                               shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    int rc = check_out(ctx, d_out, cap, n_out);
+    if (rc) return rc;
+    if (!d_n_cand || (n_cand_max && !d_cand) || !d_state_in || !d_state_out)
+        return fail(ctx, SHRED_EINVAL, "null pointer");
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
+    Aux *aux = ctx->d_aux + 0;
+    PDL(k_state_in_dev, 1, 1, 0, st, aux, d_state_in);
+    LAUNCHED("k_state_in_dev");
+    if ((rc = launch_size_bound(ctx, d_cand, d_n_cand, 0, n_cand_max, end, fin ? 1 : 0, d_out, cap, aux,
                                 nullptr, st))) return rc;
     PDL(k_state_out, 1, 1, 0, st, aux, d_state_out, n_out, cap);
     LAUNCHED("k_state_out");
@@ -1092,6 +1143,13 @@ int shred_debug_plan(int path, int small_ok, int sm_count, uint64_t src_addr, ui
                                                               : (uint64_t)(path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC)};
     for (int i = 0; i < 16; ++i) out[i] = v[i];
     return SHRED_OK;
+}
+
+int shred_debug_tprod(uint64_t poly, uint32_t *mult) {
+    uint32_t m = 0;
+    const int ok = tprod_ok(poly, deg64(poly), &m) ? 1 : 0;
+    if (mult) *mult = m;
+    return ok;
 }
 
 int shred_profile(shred_ctx *ctx, int enable) {

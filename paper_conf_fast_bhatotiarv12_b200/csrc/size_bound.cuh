@@ -38,6 +38,7 @@ struct SBArgs {
     const uint64_t *cand;           // ascending candidates
     const uint64_t *n_dev;          // candidate count (device), or null -> n_host
     uint64_t n_host;
+    uint64_t n_cap;                 // a device count is clamped to this (the list's capacity)
     uint64_t minsz, maxsz;          // maxsz 0 = inf
     uint64_t end;                   // stream end (fin = 1) or current fed end (fin = 0)
     int fin;
@@ -49,7 +50,11 @@ struct SBArgs {
     Aux *aux;                       // s, held, held_val, out_pos (streaming state)
 };
 
-__device__ __forceinline__ uint64_t sb_n(const SBArgs &A) { return A.n_dev ? *A.n_dev : A.n_host; }
+__device__ __forceinline__ uint64_t sb_n(const SBArgs &A) {
+    if (!A.n_dev) return A.n_host;
+    const uint64_t n = *A.n_dev;
+    return n < A.n_cap ? n : A.n_cap;
+}
 
 // One candidate: returns the number of cuts emitted (forced + accepted, held excluded).
 template <class Emit>

@@ -530,3 +530,46 @@ def test_remainder_marker_hot_kernel(pkg, poly, D):
     ch = pkg.Chunker(pkg.Params(poly=poly, window=47, divisor=D, magic=r, marker=marker))
     n = data.size
     assert np.array_equal(_feed_all(ch, data, [n // 3, 5, n - n // 3 - 5], True), oracle.chunk(data, oparams(ch.params)))
+
+
+# ------------------------------------------------------------------ K32T (T as an integer product)
+@pytest.mark.parametrize("poly", [0x80002001, 0x80040001, 0x40200001, 0x10000201, 0x800201, 0x40201])
+@pytest.mark.parametrize("window,marker", [(48, 0), (48, 1), (32, 0), (47, 0), (16, 1)])
+def test_k32t_multiply_reduction_paths(pkg, poly, window, marker):
+    """Sparse irreducible P (Q's terms >= 8 apart): the u32 kernel reduces the top byte with one
+    IMAD (MODE_K32T, L255-L258 with any irreducible div(x)); bit-exact vs the oracle with both
+    marker sets, funnel windows, bounds, a feed straddling pieces, and virtual shards."""
+    data = synthgen.random_bytes(poly & 0xFFFF, (3 << 20) + 4093)
+    D = 512 if poly < (1 << 20) else 4096
+    p = pkg.Params(poly=poly, window=window, divisor=D, magic=7 if not marker else 3, marker=marker)
+    ch = pkg.Chunker(p)
+    assert ch.mode == "k32t" and ch.path == "k32"
+    got = check_chunk(ch, data)
+    pb = pkg.Params(poly=poly, window=window, divisor=D, magic=7 if not marker else 3, marker=marker,
+                    min_size=D // 4, max_size=8 * D)
+    check_chunk(pkg.Chunker(pb), data)
+    # feed in uneven pieces (carry across pieces), then two virtual shards
+    chf = pkg.Chunker(p)
+    outs, a = [], 0
+    for step in (1 << 20, 12345, (1 << 21) + 1, len(data)):
+        outs.append(chf.feed(dev(data[a:a + step])).cpu().numpy())
+        a = min(len(data), a + step)
+    outs.append(chf.flush().cpu().numpy())
+    assert np.array_equal(np.concatenate(outs).astype(np.uint64), got)
+    n = len(data)
+    s = (n // 2) // 4096 * 4096
+    x = dev(data)
+    parts = [ch.candidates_range(x[:s], 0, 0, n), ch.candidates_range(x[s - (window - 1):], window - 1, s, n)]
+    assert np.array_equal(torch.cat(parts).cpu().numpy().astype(np.uint64), oracle.candidates(data, oparams(p)))
+
+
+def test_k32t_small_shape_and_le_marker_modes(pkg):
+    """1 MiB (the small launch shape) on K32T; '==' with 2^32 > D; mode selection table."""
+    data = synthgen.random_bytes(77, 1 << 20)
+    for p, mode in ((pkg.Params(poly=0x80002001), "k32t"),
+                    (pkg.Params(poly=0x80002001, divisor=1 << 20, magic=12345), "k32t"),
+                    (pkg.Params(poly=0x80002001, divisor=10000, magic=7), "k32"),      # MK_DIV: table mode
+                    (pkg.Params(poly=0x104C11DB7), "k32b"), (pkg.Params(), "k63")):
+        ch = pkg.Chunker(p)
+        assert ch.mode == mode, (p, ch.mode)
+        check_chunk(ch, data)

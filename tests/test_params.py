@@ -86,3 +86,32 @@ def test_path_table(check, kw, path, mk):
         pytest.skip("not irreducible")
     rc, p, m = check(**kw)
     assert rc == 0 and (p, m) == (path, mk), (kw, p, m)
+
+
+def test_k32t_multiplier_equals_the_reduction_table():
+    """K32T (T[t] as one integer product): for every eligible P (deg <= 32, Q = P - x^k with terms
+    >= 8 apart below k - 7) the library's multiplier gives, for every byte t,
+    t * M mod 2^32 == (t(x) x^k mod P) XOR (t << k mod 2^32): the reduction computed here by the
+    oracle's long division (R1), the cancel term by the definition of the u32 shift.  Ineligible
+    polynomials (overlapping copies of t, or a term too high) are refused."""
+    from paper_conf_fast_bhatotiarv12_b200 import _build
+    lib = ctypes.CDLL(_build.build())
+    f = lib.shred_debug_tprod
+    f.argtypes = [ctypes.c_uint64, ctypes.POINTER(ctypes.c_uint32)]
+    f.restype = ctypes.c_int
+    eligible = [0x80002001, 0x80040001, 0x40200001, 0x40000201, 0x10000201, 0x10002001, 0x800201,
+                0x804001, 0x40201]
+    for P in eligible:
+        assert oracle.is_irreducible(P)
+        m = ctypes.c_uint32(0)
+        assert f(P, ctypes.byref(m)) == 1, hex(P)
+        k = P.bit_length() - 1
+        for t in range(256):
+            # t(x) x^k mod P by R1 on the message t || zero bits: shift t by k bits via bytes
+            msg = t << k
+            nb = (msg.bit_length() + 7) // 8 or 1
+            red = oracle.polymod(np.frombuffer(msg.to_bytes(nb, "big"), np.uint8), P)
+            exp = red ^ ((t << k) & 0xFFFFFFFF)
+            assert (t * m.value) & 0xFFFFFFFF == exp, (hex(P), t)
+    for P in (0x104C11DB7, LBFS, 0x8000000B, 0x80000081, 0x20000005, (1 << 31) | (1 << 24) | 1):
+        assert f(P, None) == 0, hex(P)

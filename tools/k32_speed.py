@@ -13,7 +13,10 @@ import paper_conf_fast_bhatotiarv12_b200 as pkg  # noqa: E402
 n = 1 << 30
 x = torch.empty(n, dtype=torch.uint8, device="cuda")
 pkg.synth_fill(x, 2)
-cases = {"k32b (0x104C11DB7)": pkg.Params(poly=0x104C11DB7),
+cases = {"k32t (x^31+x^13+1)": pkg.Params(poly=0x80002001),
+         "k32t (x^30+x^21+1)": pkg.Params(poly=0x40200001),
+         "k32t le r=1": pkg.Params(poly=0x80002001, marker=1, magic=1),
+         "k32b (0x104C11DB7)": pkg.Params(poly=0x104C11DB7),
          "k32 (deg 29)": pkg.Params(poly=0x20000005 if len(sys.argv) < 2 else int(sys.argv[1], 0)),
          "k32b le r=1": pkg.Params(poly=0x104C11DB7, marker=1, magic=1),
          "k63 (paper)": pkg.Params()}
@@ -38,6 +41,6 @@ for name, p in cases.items():
     torch.cuda.synchronize()
     ch.profile(False)
     kms, kn, kb = ch.profile_read()
-    print(json.dumps({"case": name, "path": ch.path, "call_gbs": round(reps * n / (e0.elapsed_time(e1) * 1e-3) / 1e9, 1),
+    print(json.dumps({"case": name, "path": ch.path, "mode": ch.mode, "call_gbs": round(reps * n / (e0.elapsed_time(e1) * 1e-3) / 1e9, 1),
                       "k1_gbs": round(kb / (kms * 1e-3) / 1e9, 1), "cands": int(nn.item()),
                       "lib": os.path.basename(os.environ.get("SHRED_LIB", "libshred.so"))}), flush=True)
