@@ -116,7 +116,7 @@ class ClockSampler:
                 self.reasons |= int(get_r(self.h))
             except Exception:
                 pass
-            time.sleep(0.002)
+            time.sleep(0.0005)
 
     def __enter__(self):
         if self.ok:
@@ -565,7 +565,7 @@ def main():
         roofline["smem_datapath"] = {"ceiling_gbs": round(smem_ceiling, 1), "frac": round(achieved / smem_ceiling, 4),
                                      "bytes_per_input_byte": smem_bpb, "sms": nsm, "sm_mhz": clk_mhz,
                                      "source": "128 B/clk/SM SMEM/L1 data path (B300_MICROARCH.md); ncu "
-                                               "l1tex__data_pipe_lsu_wavefronts in profiles/r01_k1_bulk_ncu_full.txt"}
+                                               f"l1tex__data_pipe_lsu_wavefronts in {traffic_src}"}
 
     line = {"metric": METRIC, "value": round(value, 2), "unit": "GB/s", "n_gpus": world, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": round(ms_max / args.steps, 4), "higher_is_better": True,

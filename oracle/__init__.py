@@ -155,7 +155,11 @@ def candidates(data, p: Params = Params(), method: int = 2, threads: int | None 
     a = _bytes(data)
     if threads is None:
         threads = len(os.sched_getaffinity(0))
-    cap = 1 << 16
+    # output buffer sized from the expected count (hits per D positions: 1, or r + 1 for '<='), so
+    # random-like inputs run the C routine once; a larger true count re-runs with the exact size
+    # (round 1 started at 2^16 and ran every GiB-scale input twice, halving the measured rate)
+    hits = (p.magic + 1) if p.marker else 1
+    cap = max(1 << 16, int(2 * a.size * hits / p.divisor) + 4096)
     while True:
         out = np.zeros(cap, dtype=np.uint64)
         n = _L().orc_candidates(a.ctypes.data, a.size, p.window, p.poly, p.divisor, p.magic,
