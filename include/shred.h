@@ -26,7 +26,14 @@
  *   Memory      d_* = device memory (cudaMalloc / torch CUDA tensor).  n_out = device memory or
  *               mapped page-locked host memory (cudaHostAlloc; written by a kernel).
  *   Async       Calls enqueue on `stream` and return; nothing is synchronised unless stated.
- *               A ctx is bound to one device and is not re-entrant (one caller thread at a time).
+ *               Exception: a call that needs more scratch than any earlier call of the ctx
+ *               grows it synchronously (cudaDeviceSynchronize before freeing the old buffer).
+ *   Streams     A ctx is bound to one device and is not re-entrant (one caller thread at a
+ *               time).  Its calls share the ctx's scratch, state and ring, so they run in call
+ *               order: a call on a stream other than the previous call's first makes its stream
+ *               wait for the previous call's completion event (no host synchronisation).  Under
+ *               CUDA-graph capture no event is recorded or waited on: capture a ctx's calls on
+ *               the stream its preceding work used (or synchronise before capturing).
  *   Errors      Negative return codes are synchronous problems (parameters, enqueue,
  *               allocation).  Output-capacity overflow is in-band: *n_out receives the TRUE
  *               count n and min(n, cap) offsets are written (snprintf convention).  In the

@@ -11,7 +11,7 @@
 //
 //   k1_bulk<MODE,C,WCH,MK,FN>  TMA-staged hot loop (FN: w not a multiple of 16, funnel pops).  The input is viewed as a 2-D [rows][S]
 //                   tensor; each consumer thread rolls CH = 2 rows (independent chains) in one
-//                   basic block; rounds of 32 B per row arrive in a 4-stage shared-memory ring
+//                   basic block; rounds of 32 B per row arrive in a 2-stage shared-memory ring
 //                   (SWIZZLE_32B, conflict-free LDS.128) fed by a producer warp.  T/U live in
 //                   shared memory, replicated per lane so the data-dependent lookups never
 //                   bank-conflict.  The marker test sets bits of a per-16-byte hit mask
@@ -742,7 +742,7 @@ __device__ __forceinline__ void pops16(const uint4 (&lo)[CH], const uint4 (&hi)[
 
 // The hot kernel.  blockDim = NTC consumers + 1 producer warp; one CTA per SM.
 // blockIdx < nc: bulk CTA, rows blockIdx*ROWS + tid + ch*NTC (ch < CH); blockIdx == nc: the
-// edge CTA.  Rounds of ROUND = 64/CH bytes per row arrive in a 4-stage TMA ring (the 8 lanes
+// edge CTA.  Rounds of ROUND = 64/CH bytes per row arrive in a SHRED_STAGES-deep TMA ring (the 8 lanes
 // of a quarter warp read 8 consecutive rows' 16-byte chunks from 8 distinct bank groups:
 // SWIZZLE_32B for 32-byte rounds, no swizzle for 16-byte rounds).  The window is fixed at
 // w = 48 = 3 chunks of 16 B: the byte leaving the window at chunk q is the same byte slot of

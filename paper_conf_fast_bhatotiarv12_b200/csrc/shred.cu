@@ -201,6 +201,9 @@ cudaError_t pdl_launch(void (*k)(KArgs...), dim3 g, dim3 b, size_t smem, cudaStr
 #define PDL(k, g, b, smem, st, ...) do { cudaError_t _pe = pdl_launch(k, g, b, smem, st, __VA_ARGS__); \
     if (_pe != cudaSuccess) return cuda_fail(ctx, _pe, #k); } while (0)
 
+// Scratch grows synchronously: freeing the old buffer waits for the whole device
+// (cudaDeviceSynchronize), so a call that needs more scratch than any earlier call blocks the
+// host once (include/shred.h "Streams").  Steady-state calls of the same or smaller size never do.
 template <class T>
 int grow(shred_ctx *ctx, T *&ptr, uint64_t &cap, uint64_t need, const char *what) {
     if (need <= cap) return SHRED_OK;
@@ -970,8 +973,8 @@ int shred_feed(shred_ctx *ctx, const void *in, uint64_t len, uint64_t *d_out, ui
         } else {
             if ((rc = ensure_ring(ctx))) return rc;
             // Pieces of <= one slot.  The H2D copy of piece p+ring-1 is enqueued on the copy
-            // stream before piece p is processed, so transfers overlap the chunking (also in
-            // bounded mode, whose piece processing synchronises once on the candidate count).
+            // stream before piece p is processed, so transfers overlap the chunking (bounded
+            // mode too: its size-rule state stays on the device, nothing waits on the host).
             const uint8_t *h = (const uint8_t *)in;
             const uint64_t npieces = (len + ctx->ring_bytes - 1) / ctx->ring_bytes;
             const int R = ctx->ring_n;
