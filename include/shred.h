@@ -31,9 +31,11 @@
  *   Streams     A ctx is bound to one device and is not re-entrant (one caller thread at a
  *               time).  Its calls share the ctx's scratch, state and ring, so they run in call
  *               order: a call on a stream other than the previous call's first makes its stream
- *               wait for the previous call's completion event (no host synchronisation).  Under
+ *               wait for the work enqueued on that stream (an event; no host synchronisation).  Under
  *               CUDA-graph capture no event is recorded or waited on: capture a ctx's calls on
- *               the stream its preceding work used (or synchronise before capturing).
+ *               the stream its preceding work used (or synchronise before capturing).  The
+ *               previous call's stream must still exist when a call switches streams (the end
+ *               of its work is recorded on it then).
  *   Errors      Negative return codes are synchronous problems (parameters, enqueue,
  *               allocation).  Output-capacity overflow is in-band: *n_out receives the TRUE
  *               count n and min(n, cap) offsets are written (snprintf convention).  In the
@@ -231,12 +233,15 @@ int shred_check_params(const shred_params *p, int *path_out, int *marker_kind_ou
 
 /* Test hook (no device needed): the slot map planning would use for window ends [t_begin, t_end)
    of a job whose bytes start at stream position p_begin at address src_addr, for kernel path
-   `path` (SHRED_PATH_*), with (small_ok) or without the small-input launch shape, on sm_count SMs.
+   `path` (SHRED_PATH_*), with (small_ok) or without the small-input launch shape, on sm_count SMs,
+   for a window of `window` bytes (1..64: the fast paths), zero_lead = 1 if the job starts at the
+   stream start with no carried prefix (rows may then start at the stream start itself).
    out[16] = {bulk, small, head_start, head_seg, n_head, b0, S, nrows, tail_start, tail_seg,
    n_tail, bulk CTAs, slot groups, rows per CTA, per-slot list capacity for `divisor`, threads per
    edge CTA}.  SHRED_EINVAL on inconsistent arguments. */
 int shred_debug_plan(int path, int small_ok, int sm_count, uint64_t src_addr, uint64_t p_begin,
-                     uint64_t t_begin, uint64_t t_end, uint64_t divisor, uint64_t out[16]);
+                     uint64_t t_begin, uint64_t t_end, uint64_t divisor, uint32_t window, int zero_lead,
+                     uint64_t out[16]);
 /* Test hook (host logic, no GPU): 1 if the K32T kernel mode applies to poly (deg <= 32 and
    P = x^k + Q with Q's terms >= 8 apart and below k - 7), with *mult = Q + 2^k mod 2^32, the
    integer multiplier that gives T[t] = t(x) x^k mod P ^ (t << k mod 2^32) as t * mult mod 2^32. */

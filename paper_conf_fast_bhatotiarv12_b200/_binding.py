@@ -97,8 +97,14 @@ def lib() -> ctypes.CDLL:
     return _lib
 
 
+_raw_stream = getattr(torch._C, "_cuda_getCurrentRawStream", None)
+
+
 def _stream(stream) -> int:
     if stream is None:
+        # the current stream's cudaStream_t without building a torch.cuda.Stream object (~2 us)
+        if _raw_stream is not None:
+            return _raw_stream(torch.cuda.current_device())
         return torch.cuda.current_stream().cuda_stream
     if isinstance(stream, torch.cuda.Stream):
         return stream.cuda_stream
@@ -128,6 +134,7 @@ class Chunker:
             raise ShredError(f"shred_init: {lib().shred_strerror(rc).decode()} ({rc}) for {params}")
         dev = torch.device("cuda", self.device)
         self._n = torch.zeros(1, dtype=torch.int64, device=dev)
+        self._chunk = lib().shred_chunk          # bound once: the per-call path is argument marshalling only
 
     def close(self):
         if self._ctx:
@@ -178,10 +185,12 @@ class Chunker:
     # ---------------------------------------------------------------- one-shot
     def chunk_async(self, x: torch.Tensor, out: torch.Tensor, n_out: torch.Tensor, stream=None) -> None:
         """Enqueue shred_chunk; out (int64) gets the cuts, n_out[0] the true count."""
-        assert x.is_cuda and x.dtype == torch.uint8 and x.is_contiguous()
-        rc = lib().shred_chunk(self._ctx, x.data_ptr(), x.numel(), out.data_ptr(), out.numel(),
-                               n_out.data_ptr(), _stream(stream))
-        self._check(rc, "shred_chunk")
+        if x.dtype != torch.uint8 or not x.is_cuda or not x.is_contiguous():
+            raise ShredError("shred_chunk: x must be a contiguous CUDA uint8 tensor")
+        rc = self._chunk(self._ctx, x.data_ptr(), x.numel(), out.data_ptr(), out.numel(),
+                         n_out.data_ptr(), _stream(stream))
+        if rc:
+            self._check(rc, "shred_chunk")
 
     def _guess(self, n: int) -> int:
         return min(self.max_cuts(n), n // 512 + 4096) if n > 1 else 1

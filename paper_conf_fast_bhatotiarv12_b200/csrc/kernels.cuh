@@ -820,7 +820,8 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     __syncthreads();
 
     const uint32_t row0 = blockIdx.x * C::ROWS;
-    const uint32_t nrounds = (uint32_t)(J.map.S / ROUND);     // a multiple of CH (S % 64 == 0)
+    const uint32_t nrounds = (uint32_t)(J.map.S / ROUND);     // S % 32 == 0: a loop iteration (RPI
+                                                              // rounds = 64 B) may end half way
 
     if (tid >= NTC) {                                // ---- producer warp
         if (tid == NTC) {
@@ -868,16 +869,23 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         o[ch].cnt = 0; o[ch].cap = J.cap;
     }
     {
-        // warm-up: the 64 bytes before each row (b0 >= p_begin + 64 keeps them inside src)
+        // warm-up: the 16*WCH bytes before each row, from a zero state (the plan keeps them inside
+        // src: b0 >= p_begin + 16*WCH).  A row at the very start of a stream (no carry) finds
+        // virtual zero bytes before p_begin instead: zero bytes pushed into a zero state leave it
+        // zero (T[0] = U[0] = 0), and only full windows are tested (min_i).  The ring slots of
+        // the 4 - WCH chunks not rolled stay zero.
         const uint4 Z = make_uint4(0, 0, 0, 0);
 #pragma unroll
         for (int ch = 0; ch < CH; ++ch) {
 #pragma unroll
             for (int q = 0; q < 4; ++q) R[ch][q] = Z;
             if (act[ch]) {
-                const uint4 *h = reinterpret_cast<const uint4 *>(J.src + (pos0[ch] - 64u - J.p_begin));
 #pragma unroll
-                for (int q = 0; q < 4; ++q) R[ch][q] = __ldg(h + q);
+                for (int q = (C::DIRECT_WARM ? 0 : 4 - WCH); q < 4; ++q) {
+                    // chunk q holds stream bytes [pos0 - 64 + 16q, +16): inside the job's bytes?
+                    if (pos0[ch] + 16u * (uint32_t)q >= J.p_begin + 64u)
+                        R[ch][q] = __ldg(reinterpret_cast<const uint4 *>(J.src + (pos0[ch] + 16u * (uint32_t)q - 64u - J.p_begin)));
+                }
             }
         }
         if (C::DIRECT_WARM) {
@@ -903,15 +911,15 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         mbar_wait(tabbar, 0);                         // T|U image resident
         uint32_t m[CH];
 #pragma unroll
-        for (int q = 0; q < (C::DIRECT_WARM ? 0 : 4); ++q) {
+        for (int q = (C::DIRECT_WARM ? 4 : 4 - WCH); q < 4; ++q) {
+            // chunks before 4 - WCH were never pushed: their bytes pop as zero
             uint4 d[CH], p[CH];
-#pragma unroll
             uint4 lo[CH], hi[CH];
 #pragma unroll
             for (int ch = 0; ch < CH; ++ch) {
                 d[ch] = R[ch][q];
-                lo[ch] = (q >= WCH) ? R[ch][q - WCH] : Z;
-                hi[ch] = (q + 1 >= WCH) ? R[ch][q + 1 - WCH] : Z;
+                lo[ch] = (q - WCH >= 4 - WCH) ? R[ch][q - WCH] : Z;
+                hi[ch] = (q + 1 - WCH >= 4 - WCH) ? R[ch][q + 1 - WCH] : Z;
             }
             pops16<FN, CH>(lo, hi, p, K);
             chunk16xN<MODE, CH, false, MK>(st, d, p, c, m);
@@ -925,6 +933,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     for (uint32_t r = 0; r < nrounds; r += C::RPI) {
 #pragma unroll
         for (int qr = 0; qr < C::RPI; ++qr) {             // round r + qr: chunks qr*CPR .. +CPR-1
+            if (qr > 0 && r + qr >= nrounds) break;       // rows of an odd number of 32-byte rounds
             const uint32_t s = (r + qr) % STAGES;
             mbar_wait(bars + 8 * s, ((r + qr) / STAGES) & 1u);
             const uint32_t sb = stages + s * C::STAGE;

@@ -5,9 +5,11 @@ shred_debug_plan).
 Invariants checked over random lengths, stream offsets, source alignments and SM counts:
 * the head segments, the rows and the tail segments tile [t_begin, t_end) exactly, in order
   (every window end is tested once: parity with the oracle depends on it);
-* the bulk region starts 16-byte aligned in memory (TMA) and at least 64 bytes into the job's
-  bytes (the rows' warm-up reads the 64 bytes before each row);
-* rows are a multiple of 64 bytes (whole 32-byte TMA rounds, two per loop iteration);
+* the bulk region starts 16-byte aligned in memory (TMA) and at least 16*ceil(w/16) bytes into
+  the job's bytes (the rows' warm-up reads them), or at the stream start itself when the job
+  starts there with no carry (virtual zero bytes before it);
+* rows are a multiple of 32 bytes (whole 32-byte TMA rounds; a loop iteration of two rounds may
+  stop after the first);
 * the edge CTA has one thread per head and per tail segment;
 * slot groups fit the scatter kernel's table, and per-slot lists hold >= 2x the expected count.
 """
@@ -27,14 +29,15 @@ def L():
     lib = ctypes.CDLL(_build.build())
     f = lib.shred_debug_plan
     u64 = ctypes.c_uint64
-    f.argtypes = [ctypes.c_int, ctypes.c_int, ctypes.c_int, u64, u64, u64, u64, u64, ctypes.POINTER(u64)]
+    f.argtypes = [ctypes.c_int, ctypes.c_int, ctypes.c_int, u64, u64, u64, u64, u64, ctypes.c_uint32, ctypes.c_int,
+                  ctypes.POINTER(u64)]
     f.restype = ctypes.c_int
     return lib
 
 
-def plan(L, path, small_ok, sms, addr, p_begin, t_begin, t_end, divisor=8192):
+def plan(L, path, small_ok, sms, addr, p_begin, t_begin, t_end, divisor=8192, window=48, zero_lead=0):
     out = (ctypes.c_uint64 * 16)()
-    rc = L.shred_debug_plan(path, small_ok, sms, addr, p_begin, t_begin, t_end, divisor, out)
+    rc = L.shred_debug_plan(path, small_ok, sms, addr, p_begin, t_begin, t_end, divisor, window, zero_lead, out)
     assert rc == 0
     keys = ("bulk", "small", "head_start", "head_seg", "n_head", "b0", "S", "nrows", "tail_start",
             "tail_seg", "n_tail", "nc", "ngroups", "rows_cta", "cap", "edge_threads")
@@ -57,7 +60,7 @@ def segments(m, t_begin, t_end):
     return out
 
 
-def check(m, path, addr, p_begin, t_begin, t_end, divisor=8192):
+def check(m, path, addr, p_begin, t_begin, t_end, divisor=8192, window=48, zero_lead=0):
     segs = segments(m, t_begin, t_end)
     pos = t_begin
     for a, b in segs:
@@ -68,8 +71,12 @@ def check(m, path, addr, p_begin, t_begin, t_end, divisor=8192):
     if m["bulk"]:
         assert path in (K63, K32)
         assert (addr + (m["b0"] - p_begin)) % 16 == 0
-        assert m["b0"] >= p_begin + 64 and m["b0"] >= t_begin
-        assert m["S"] % 64 == 0 and m["S"] >= 64 and m["nrows"] >= 1
+        # each row warms up on the 16*ceil(w/16) bytes before it, inside the job's bytes, or it
+        # starts at the stream start itself (no carry: virtual zero bytes before it)
+        warm = 16 * ((window + 15) // 16)
+        assert m["b0"] >= t_begin
+        assert m["b0"] >= p_begin + warm or (zero_lead and m["b0"] == p_begin == t_begin)
+        assert m["S"] % 32 == 0 and m["S"] >= 32 and m["nrows"] >= 1
         assert m["n_head"] <= m["edge_threads"] and m["n_tail"] <= m["edge_threads"]
         assert m["nc"] == -(-m["nrows"] // m["rows_cta"])
         assert m["ngroups"] == m["nc"] + 2
@@ -94,8 +101,12 @@ def test_plan_tiles_every_window_end_once(L, path):
             t_begin = p_begin + int(rng.integers(0, 200))
             sms = int(rng.choice([1, 2, 132, 148, 160]))
             small_ok = int(rng.integers(0, 2))
-            m = plan(L, path, small_ok, sms, addr, p_begin, t_begin, t_begin + n)
-            check(m, path, addr, p_begin, t_begin, t_begin + n)
+            window = int(rng.choice([1, 16, 17, 47, 48, 64]))
+            zl = int(rng.integers(0, 2))
+            if zl and rng.integers(0, 2):
+                t_begin = p_begin
+            m = plan(L, path, small_ok, sms, addr, p_begin, t_begin, t_begin + n, window=window, zero_lead=zl)
+            check(m, path, addr, p_begin, t_begin, t_begin + n, window=window, zero_lead=zl)
 
 
 def test_plan_shapes(L):
@@ -103,17 +114,24 @@ def test_plan_shapes(L):
     small launch shape; below 4 KiB (or on the generic path) there are no rows."""
     m = plan(L, K63, 1, 148, 0, 0, 47, 1 << 30)
     assert m["bulk"] and not m["small"] and m["nc"] == 147 and m["rows_cta"] == 1024
-    assert m["S"] % 64 == 0 and m["nrows"] * m["S"] <= (1 << 30)
+    assert m["S"] % 32 == 0 and m["nrows"] * m["S"] <= (1 << 30)
     m = plan(L, K63, 1, 148, 0, 0, 47, 1 << 20)
     assert m["bulk"] and m["small"] and m["rows_cta"] == 256
     m = plan(L, K63, 0, 148, 0, 0, 47, 1 << 20)
     assert m["bulk"] and not m["small"]
     assert not plan(L, K63, 1, 148, 0, 0, 0, 4000)["bulk"]
     assert not plan(L, GENERIC, 1, 148, 0, 0, 0, 1 << 30)["bulk"]
+    # an aligned stream from its start, no carry: the rows begin at byte 0, no head segments;
+    # 1 MiB = 32768 rows of 32 B, no tail either (the edge CTA has nothing to roll)
+    m = plan(L, K63, 1, 148, 0, 0, 0, 1 << 20, zero_lead=1)
+    assert m["b0"] == 0 and m["n_head"] == 0 and m["n_tail"] == 0 and m["S"] == 32
+    m = plan(L, K63, 1, 148, 0, 0, 0, 1 << 20, zero_lead=0)
+    assert m["b0"] == 48 and m["n_head"] == 3
 
 
 def test_plan_rejects_inconsistent_arguments(L):
     out = (ctypes.c_uint64 * 16)()
-    assert L.shred_debug_plan(K63, 1, 148, 0, 100, 50, 1000, 8192, out) != 0   # t_begin < p_begin
-    assert L.shred_debug_plan(K63, 1, 148, 0, 0, 10, 5, 8192, out) != 0        # t_end < t_begin
-    assert L.shred_debug_plan(K63, 1, 0, 0, 0, 0, 5, 8192, out) != 0           # no SMs
+    assert L.shred_debug_plan(K63, 1, 148, 0, 100, 50, 1000, 8192, 48, 0, out) != 0   # t_begin < p_begin
+    assert L.shred_debug_plan(K63, 1, 148, 0, 0, 10, 5, 8192, 48, 0, out) != 0        # t_end < t_begin
+    assert L.shred_debug_plan(K63, 1, 0, 0, 0, 0, 5, 8192, 48, 0, out) != 0           # no SMs
+    assert L.shred_debug_plan(K63, 1, 148, 0, 0, 0, 5, 8192, 65, 0, out) != 0         # w > 64
