@@ -194,6 +194,19 @@ int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const u
                       const uint64_t *d_ncuts, uint8_t *d_digests, uint64_t max_chunks,
                       shred_stream_t stream);
 
+/* The same for several buffers in one launch sequence (e.g. the files of a backup snapshot,
+   PAPER.md L1293-L1361): every buffer's chunks join one length-sorted work list, longest first,
+   so the long sequential hash of one buffer's longest chunk overlaps the other buffers' chunks
+   instead of idling the GPU (one buffer alone is bound by its longest chunk).  jobs is a HOST
+   array of njobs descriptors (each as in shred_hash_chunks; buffers may repeat; digest arrays
+   must not overlap); launches take up to 16 jobs at a time. */
+typedef struct shred_hash_job {
+    const uint8_t *d_in; uint64_t len;
+    const uint64_t *d_cuts; const uint64_t *d_ncuts;
+    uint8_t *d_digests; uint64_t max_chunks;
+} shred_hash_job;
+int shred_hash_chunks_batch(shred_ctx *ctx, const shred_hash_job *jobs, int njobs, shred_stream_t stream);
+
 /* Matching (dedup step 3): a device index (hash set) of
    chunk digests owned by the ctx.  shred_index_reset allocates/clears it for `capacity` distinct
    digests (rounded up to a power of two, >= 2x).  shred_index_insert looks up every chunk digest

@@ -30,6 +30,11 @@ class _Params(ctypes.Structure):
                 ("min_size", ctypes.c_uint64), ("max_size", ctypes.c_uint64)]
 
 
+class _HashJob(ctypes.Structure):
+    _fields_ = [("d_in", ctypes.c_void_p), ("len", ctypes.c_uint64), ("d_cuts", ctypes.c_void_p),
+                ("d_ncuts", ctypes.c_void_p), ("d_digests", ctypes.c_void_p), ("max_chunks", ctypes.c_uint64)]
+
+
 @dataclass(frozen=True)
 class Params:
     """shred_params. Defaults = the paper's readings (Q1, Q5, Q6, Q15)."""
@@ -81,6 +86,7 @@ def lib() -> ctypes.CDLL:
             "shred_launch_count": (u64, [vp]),
             "shred_hash_chunks": (cint, [vp, vp, u64, vp, vp, vp, u64, vp]),
             "shred_index_reset": (cint, [vp, u64]),
+            "shred_hash_chunks_batch": (cint, [vp, vp, cint, vp]),
             "shred_size_bound_state": (cint, [vp, vp, u64, u64, cint, ctypes.POINTER(u64), vp, u64, vp, vp, vp]),
             "shred_size_bound_state_dev": (cint, [vp, vp, vp, u64, u64, cint, vp, vp, u64, vp, vp, vp]),
             "shred_index_insert": (cint, [vp, vp, vp, vp, u64, u64, vp, vp]),
@@ -90,7 +96,9 @@ def lib() -> ctypes.CDLL:
                                           ctypes.POINTER(u64)]),
         }
         for name, (res, args) in sig.items():
-            fn = getattr(L, name)
+            fn = getattr(L, name, None)
+            if fn is None:                      # an older A/B build (SHRED_LIB) without this call
+                continue
             fn.restype = res
             fn.argtypes = args
         _lib = L
@@ -303,6 +311,18 @@ class Chunker:
         rc = lib().shred_hash_chunks(self._ctx, x.data_ptr(), x.numel(), cuts.data_ptr(), n_cuts.data_ptr(),
                                      digests.data_ptr(), digests.numel() // 32, _stream(stream))
         self._check(rc, "shred_hash_chunks")
+
+    def hash_chunks_batch_async(self, jobs, stream=None) -> None:
+        """Enqueue shred_hash_chunks_batch: jobs = [(x, cuts, n_cuts, digests), ...] as in
+        hash_chunks_async; one length-sorted work list over every buffer's chunks."""
+        arr = (_HashJob * len(jobs))()
+        for k, (x, cuts, n_cuts, digests) in enumerate(jobs):
+            assert x.is_cuda and x.dtype == torch.uint8 and x.is_contiguous()
+            assert digests.dtype == torch.uint8 and digests.is_contiguous() and digests.numel() % 32 == 0
+            arr[k] = _HashJob(x.data_ptr(), x.numel(), cuts.data_ptr(), n_cuts.data_ptr(), digests.data_ptr(),
+                              digests.numel() // 32)
+        rc = lib().shred_hash_chunks_batch(self._ctx, ctypes.cast(arr, ctypes.c_void_p), len(jobs), _stream(stream))
+        self._check(rc, "shred_hash_chunks_batch")
 
     def hash_chunks(self, x: torch.Tensor, cuts: torch.Tensor) -> torch.Tensor:
         """(len(cuts)+1, 32) uint8 SHA-256 digests of the chunks of x (synchronises)."""

@@ -18,7 +18,12 @@
 
 namespace shred {
 
-__constant__ uint32_t kSha256K[64] = {
+// The round constants as instruction immediates: sha_k(t) with t a compile-time index of the
+// unrolled round loop folds to a constant (a __constant__ table made ptxas load them into
+// registers with LDC inside the round loop of the batched kernel: +20 % time, short-scoreboard
+// stalls, profiles/r02_hash_ab.txt).
+__device__ __forceinline__ constexpr uint32_t sha_k(int t) {
+    constexpr uint32_t k[64] = {
     0x428a2f98u, 0x71374491u, 0xb5c0fbcfu, 0xe9b5dba5u, 0x3956c25bu, 0x59f111f1u, 0x923f82a4u, 0xab1c5ed5u,
     0xd807aa98u, 0x12835b01u, 0x243185beu, 0x550c7dc3u, 0x72be5d74u, 0x80deb1feu, 0x9bdc06a7u, 0xc19bf174u,
     0xe49b69c1u, 0xefbe4786u, 0x0fc19dc6u, 0x240ca1ccu, 0x2de92c6fu, 0x4a7484aau, 0x5cb0a9dcu, 0x76f988dau,
@@ -27,6 +32,8 @@ __constant__ uint32_t kSha256K[64] = {
     0xa2bfe8a1u, 0xa81a664bu, 0xc24b8b70u, 0xc76c51a3u, 0xd192e819u, 0xd6990624u, 0xf40e3585u, 0x106aa070u,
     0x19a4c116u, 0x1e376c08u, 0x2748774cu, 0x34b0bcb5u, 0x391c0cb3u, 0x4ed8aa4au, 0x5b9cca4fu, 0x682e6ff3u,
     0x748f82eeu, 0x78a5636fu, 0x84c87814u, 0x8cc70208u, 0x90befffau, 0xa4506cebu, 0xbef9a3f7u, 0xc67178f2u};
+    return k[t];
+}
 
 __device__ __forceinline__ uint32_t rotr(uint32_t x, int n) { return __funnelshift_r(x, x, n); }
 
@@ -67,10 +74,10 @@ __device__ __forceinline__ void sha256_compress(uint32_t (&H)[8], uint32_t (&W)[
         const uint32_t ch = (e & f) ^ (~e & g);
         const uint32_t mj = (a & b) ^ (a & c) ^ (b & c);
         if (SHA_FMA == 2) {                // every addition an IMAD (x * one + y): ALU keeps the logic
-            const uint32_t t1 = (ch * one + (S1 * one + (w * one + (h * one + kSha256K[t]))));
+            const uint32_t t1 = (ch * one + (S1 * one + (w * one + (h * one + sha_k(t)))));
             h = g; g = f; f = e; e = d * one + t1; d = c; c = b; b = a; a = mj * one + (S0 * one + t1);
         } else {
-            const uint32_t hkw = fma_add(h, one, fma_add(w, one, kSha256K[t]));
+            const uint32_t hkw = fma_add(h, one, fma_add(w, one, sha_k(t)));
             const uint32_t t1 = hkw + S1 + ch;
             h = g; g = f; f = e; e = d + t1; d = c; c = b; b = a; a = t1 + S0 + mj;
         }
@@ -135,25 +142,50 @@ __device__ __forceinline__ uint32_t hash_bucket(uint64_t L) {
     return (uint32_t)(HB - 1 - (k < (uint64_t)(HB - 1) ? k : (uint64_t)(HB - 1)));   // descending
 }
 
+// A batch of buffers hashed by one launch sequence (shred_hash_chunks_batch): job b's chunks
+// take global indices [base[b], base[b] + max_chunks_b); one length-sorted work list spans all of
+// them, so the longest chunks of every buffer start first and the tail of one buffer overlaps
+// the bulk of the others (one buffer alone is bound by its longest chunk, DESIGN.md §5b f2).
+constexpr int HASH_MAX_JOBS = 16;
+struct HashJob {
+    const uint8_t *in; uint64_t len;
+    const uint64_t *cuts; const uint64_t *n_cuts;   // device count of cuts
+    uint8_t *digests; uint64_t max_chunks;
+};
+struct HashJobs {
+    int n;
+    uint64_t base[HASH_MAX_JOBS + 1];               // prefix of max_chunks (global index space)
+    HashJob job[HASH_MAX_JOBS];
+};
+
 __device__ __forceinline__ void chunk_bounds(const uint64_t *cuts, uint64_t ncut, uint64_t len, uint64_t i,
                                              uint64_t &a, uint64_t &b) {
     a = i ? cuts[i - 1] : 0;
     b = i < ncut ? cuts[i] : len;
 }
+// global index g -> (job, chunk); false if g is beyond the job's true chunk count
+__device__ __forceinline__ bool hash_locate(const HashJobs &H, uint64_t g, int &jb, uint64_t &i) {
+    jb = 0;
+    while (jb + 1 < H.n && g >= H.base[jb + 1]) ++jb;
+    i = g - H.base[jb];
+    const HashJob &J = H.job[jb];
+    const uint64_t nc = J.len ? min(*J.n_cuts + 1, J.max_chunks) : 0;
+    return i < nc;
+}
 
-__global__ void k_hash_hist(const uint64_t *__restrict__ cuts, const uint64_t *n_cuts, uint64_t len,
-                            uint64_t max_chunks, uint32_t *hist) {
+__global__ void k_hash_hist(HashJobs H, uint32_t *hist) {
     pdl_entry();
-    const uint64_t ncut = *n_cuts;
-    const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nc; i += (uint64_t)gridDim.x * blockDim.x) {
-        uint64_t a, b;
-        chunk_bounds(cuts, ncut, len, i, a, b);
+    const uint64_t tot = H.base[H.n];
+    for (uint64_t g = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; g < tot; g += (uint64_t)gridDim.x * blockDim.x) {
+        int jb; uint64_t i, a, b;
+        if (!hash_locate(H, g, jb, i)) continue;
+        chunk_bounds(H.job[jb].cuts, *H.job[jb].n_cuts, H.job[jb].len, i, a, b);
         atomicAdd(&hist[hash_bucket(b - a)], 1u);
     }
 }
 
-// One CTA: exclusive scan of the HB bucket counts (in place) and reset of the work queue.
+// One CTA: exclusive scan of the HB bucket counts (in place) and reset of the work queue; the
+// total number of chunks goes to queue[1] (the workers' bound).
 __global__ void __launch_bounds__(HB) k_hash_scan(uint32_t *hist, unsigned long long *queue) {
     pdl_entry();
     __shared__ uint32_t ws[33];
@@ -161,18 +193,17 @@ __global__ void __launch_bounds__(HB) k_hash_scan(uint32_t *hist, unsigned long 
     uint32_t tot;
     const uint32_t off = block_exscan(v, HB, 1, ws, &tot);
     hist[threadIdx.x] = off;
-    if (threadIdx.x == 0) *queue = 0;
+    if (threadIdx.x == 0) { queue[0] = 0; queue[1] = tot; }
 }
 
-__global__ void k_hash_scatter(const uint64_t *__restrict__ cuts, const uint64_t *n_cuts, uint64_t len,
-                               uint64_t max_chunks, uint32_t *offs, uint32_t *order) {
+__global__ void k_hash_scatter(HashJobs H, uint32_t *offs, uint32_t *order) {
     pdl_entry();
-    const uint64_t ncut = *n_cuts;
-    const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nc; i += (uint64_t)gridDim.x * blockDim.x) {
-        uint64_t a, b;
-        chunk_bounds(cuts, ncut, len, i, a, b);
-        order[atomicAdd(&offs[hash_bucket(b - a)], 1u)] = (uint32_t)i;
+    const uint64_t tot = H.base[H.n];
+    for (uint64_t g = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; g < tot; g += (uint64_t)gridDim.x * blockDim.x) {
+        int jb; uint64_t i, a, b;
+        if (!hash_locate(H, g, jb, i)) continue;
+        chunk_bounds(H.job[jb].cuts, *H.job[jb].n_cuts, H.job[jb].len, i, a, b);
+        order[atomicAdd(&offs[hash_bucket(b - a)], 1u)] = (uint32_t)g;
     }
 }
 
@@ -184,18 +215,15 @@ __device__ __forceinline__ void sha256_store(uint8_t *digests, uint64_t chunk, c
                       __byte_perm(H[6], 0, 0x0123), __byte_perm(H[7], 0, 0x0123));
 }
 
-// Hash every chunk.  nchunks = (*n_cuts + 1 if len > 0 else 0); chunk i ends at cuts[i]
-// (i < n) or len.  digests: 32 bytes per chunk (the SHA-256 digest bytes in order).
+// Hash every chunk of every job.  Job b: nchunks = (*n_cuts + 1 if len > 0 else 0), chunk i ends
+// at cuts[i] (i < n) or len; digests: 32 bytes per chunk (the SHA-256 digest bytes in order).
 // Warps take 32 consecutive entries of the length-sorted `order` at a time from `queue`.
 // Launched with one warp per SM sub-partition: the sequential SHA chain of the longest chunks
 // bounds the run, so few warps (each issuing at full rate) beat many (profiles/r01_hash_ab.txt).
 __global__ void __launch_bounds__(256)
-k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__restrict__ cuts,
-              const uint64_t *n_cuts, uint64_t max_chunks, uint8_t *__restrict__ digests,
-              const uint32_t *__restrict__ order, unsigned long long *queue, uint32_t one) {
+k_hash_chunks(HashJobs Hj, const uint32_t *__restrict__ order, unsigned long long *queue, uint32_t one) {
     pdl_entry();
-    const uint64_t ncut = *n_cuts;
-    const uint64_t nc = len ? min(ncut + 1, max_chunks) : 0;
+    const uint64_t nc = queue[1];
     const int lane = threadIdx.x & 31;
     uint32_t H[8], W[16];
     while (true) {
@@ -205,9 +233,13 @@ k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__re
         if (base >= nc) break;
         const uint64_t j = base + (uint64_t)lane;
         if (j < nc) {
-            const uint64_t chunk = order[j];
+            int jb; uint64_t chunk;
+            hash_locate(Hj, order[j], jb, chunk);
+            const HashJob &J = Hj.job[jb];
+            const uint8_t *in = J.in;
+            const uint64_t len = J.len;
             uint64_t a, b;
-            chunk_bounds(cuts, ncut, len, chunk, a, b);
+            chunk_bounds(J.cuts, *J.n_cuts, len, chunk, a, b);
             const uint64_t L = b - a, nblk = (L + 9 + 63) / 64;
             sha256_init(H);
             // full blocks: the 17 aligned words of block blk+1 are loaded before block blk is
@@ -239,7 +271,7 @@ k_hash_chunks(const uint8_t *__restrict__ in, uint64_t len, const uint64_t *__re
                 sha256_block(in, len, a, L, blk, W);
                 sha256_compress(H, W, one);
             }
-            sha256_store(digests, chunk, H);
+            sha256_store(J.digests, chunk, H);
         }
         __syncwarp();
     }

@@ -11,6 +11,13 @@
 #include "sha256.cuh"
 #include "dedup.cuh"
 
+#ifndef SHRED_HASH_NOPDL
+// k_hash_chunks is launched plainly, not as a programmatic dependent: launched early (during
+// k_hash_scatter) its 148 one-warp-per-SMSP CTAs were placed wherever the scatter left room,
+// several on some SMs and none on others, and the 1 GiB hash took 4.6-5.6 ms instead of 3.7
+// (profiles/r02_hash_ab.txt).  Its launch latency is negligible against milliseconds of hashing.
+#define SHRED_HASH_NOPDL 1
+#endif
 #ifndef SHRED_HASH_CTAS_PER_SM
 #define SHRED_HASH_CTAS_PER_SM 1
 #endif
@@ -1064,32 +1071,60 @@ int shred_reset(shred_ctx *ctx) {
     return SHRED_OK;
 }
 
+int shred_hash_chunks_batch(shred_ctx *ctx, const shred_hash_job *jobs, int njobs, shred_stream_t stream) {
+    if (!ctx) return SHRED_EINVAL;
+    if (njobs < 0 || (njobs && !jobs)) return fail(ctx, SHRED_EINVAL, "jobs is NULL");
+    DevGuard g(ctx->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    StreamOrder so(ctx, st);
+    for (int j0 = 0; j0 < njobs; j0 += HASH_MAX_JOBS) {      // launches of up to HASH_MAX_JOBS buffers
+        HashJobs H{};
+        uint64_t tot = 0;
+        for (int j = j0; j < njobs && H.n < HASH_MAX_JOBS; ++j) {
+            const shred_hash_job &q = jobs[j];
+            if (!q.d_ncuts || (q.len && !q.d_in) || (q.max_chunks && !q.d_digests))
+                return fail(ctx, SHRED_EINVAL, "job %d: null pointer", j);
+            if (((uintptr_t)q.d_digests & 15u) != 0) return fail(ctx, SHRED_EINVAL, "job %d: d_digests must be 16-byte aligned", j);
+            if (!q.len || !q.max_chunks) continue;
+            H.base[H.n] = tot;
+            H.job[H.n] = HashJob{q.d_in, q.len, q.d_cuts, q.d_ncuts, q.d_digests, q.max_chunks};
+            tot += q.max_chunks;
+            ++H.n;
+        }
+        if (!H.n) continue;
+        H.base[H.n] = tot;
+        if (tot > 0xFFFFFFFFull) return fail(ctx, SHRED_EINVAL, "more than 2^32 - 1 chunks in one launch");
+        int rc = grow(ctx, ctx->d_order, ctx->order_cap, tot, "hash order");
+        if (rc) return rc;
+        CK(cudaMemsetAsync(ctx->d_hhist, 0, HB * sizeof(uint32_t), st), "hash hist reset");
+        const unsigned gs = (unsigned)(ctx->sm_count * 8);
+        PDL(k_hash_hist, gs, 256, 0, st, H, ctx->d_hhist);
+        LAUNCHED("k_hash_hist");
+        PDL(k_hash_scan, 1, HB, 0, st, ctx->d_hhist, ctx->d_queue);
+        LAUNCHED("k_hash_scan");
+        PDL(k_hash_scatter, gs, 256, 0, st, H, ctx->d_hhist, ctx->d_order);
+        LAUNCHED("k_hash_scatter");
+        // one warp per SM sub-partition for one buffer (its longest chunk's warp keeps a whole
+        // sub-partition); two for a batch, whose work hides the long chains anyway
+        // (profiles/r02_hash_ab.txt: 3 x 1 GiB 548 -> 627 GB/s, one buffer 290 -> 242 GB/s)
+        const unsigned hctas = (unsigned)(ctx->sm_count * SHRED_HASH_CTAS_PER_SM * (H.n > 1 ? 2 : 1));
+#if SHRED_HASH_NOPDL
+        k_hash_chunks<<<hctas, SHRED_HASH_THREADS, 0, st>>>(H, ctx->d_order, ctx->d_queue, 1u);
+#else
+        PDL(k_hash_chunks, hctas, SHRED_HASH_THREADS, 0, st, H, ctx->d_order, ctx->d_queue, 1u);
+#endif
+        LAUNCHED("k_hash_chunks");
+    }
+    return SHRED_OK;
+}
+
 int shred_hash_chunks(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, const uint64_t *d_cuts,
                       const uint64_t *d_ncuts, uint8_t *d_digests, uint64_t max_chunks,
                       shred_stream_t stream) {
     if (!ctx) return SHRED_EINVAL;
-    if (!d_ncuts || (len && !d_in) || (max_chunks && !d_digests))
-        return fail(ctx, SHRED_EINVAL, "null pointer");
-    if (((uintptr_t)d_digests & 15u) != 0) return fail(ctx, SHRED_EINVAL, "d_digests must be 16-byte aligned");
-    if (!len || !max_chunks) return SHRED_OK;
-    DevGuard g(ctx->device);
-    cudaStream_t st = (cudaStream_t)stream;
-    StreamOrder so(ctx, st);
-    int rc = grow(ctx, ctx->d_order, ctx->order_cap, max_chunks, "hash order");
-    if (rc) return rc;
     if (max_chunks > 0xFFFFFFFFull) return fail(ctx, SHRED_EINVAL, "max_chunks must be < 2^32");
-    CK(cudaMemsetAsync(ctx->d_hhist, 0, HB * sizeof(uint32_t), st), "hash hist reset");
-    const unsigned gs = (unsigned)(ctx->sm_count * 8);
-    PDL(k_hash_hist, gs, 256, 0, st, d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist);
-    LAUNCHED("k_hash_hist");
-    PDL(k_hash_scan, 1, HB, 0, st, ctx->d_hhist, ctx->d_queue);
-    LAUNCHED("k_hash_scan");
-    PDL(k_hash_scatter, gs, 256, 0, st, d_cuts, d_ncuts, len, max_chunks, ctx->d_hhist, ctx->d_order);
-    LAUNCHED("k_hash_scatter");
-    PDL(k_hash_chunks, ctx->sm_count * SHRED_HASH_CTAS_PER_SM, SHRED_HASH_THREADS, 0, st, d_in, len, d_cuts, d_ncuts, max_chunks, d_digests,
-                                                      ctx->d_order, ctx->d_queue, 1u);
-    LAUNCHED("k_hash_chunks");
-    return SHRED_OK;
+    const shred_hash_job j{d_in, len, d_cuts, d_ncuts, d_digests, max_chunks};
+    return shred_hash_chunks_batch(ctx, &j, 1, stream);
 }
 
 int shred_index_reset(shred_ctx *ctx, uint64_t capacity) {

@@ -57,6 +57,36 @@ def test_single_chunk_and_fips_message(pkg):
         assert np.array_equal(got.cpu().numpy(), oracle.chunk_digests(np.frombuffer(m, np.uint8), []))
 
 
+def test_batched_buffers_one_work_list(pkg):
+    """shred_hash_chunks_batch: 19 buffers (more than one launch of 16) of different lengths and
+    chunkings, one repeated, each chunk's digest == hashlib (FIPS-180-pinned) of that buffer's
+    chunk; chunk counts read on the device."""
+    rng = np.random.default_rng(12)
+    ch = pkg.Chunker(pkg.Params(divisor=1024))
+    jobs, exp = [], []
+    datas = [synthgen.random_bytes(40 + k, int(rng.integers(1, 300000))) for k in range(18)] + [None]
+    datas[-1] = datas[3]
+    for k, data in enumerate(datas):
+        x = torch.from_numpy(data).cuda()
+        if k % 3 == 0:                       # the chunker's own cuts (device count)
+            cuts = torch.empty(max(1, data.size // 256), dtype=torch.int64, device="cuda")
+            nc = torch.zeros(1, dtype=torch.int64, device="cuda")
+            ch.chunk_async(x, cuts, nc)
+            torch.cuda.synchronize()
+            c = cuts[:int(nc.item())].cpu().numpy()
+        else:                                # arbitrary cuts incl. 1-byte and padding-edge chunks
+            c = np.unique(rng.integers(1, max(2, data.size), int(rng.integers(0, 60)))).astype(np.int64)
+            cuts = torch.from_numpy(c).cuda() if c.size else torch.zeros(1, dtype=torch.int64, device="cuda")
+            nc = torch.tensor([c.size], dtype=torch.int64, device="cuda")
+        dig = torch.empty((c.size + 1) * 32, dtype=torch.uint8, device="cuda")
+        jobs.append((x, cuts, nc, dig))
+        exp.append(oracle.chunk_digests(data, c))
+    ch.hash_chunks_batch_async(jobs)
+    torch.cuda.synchronize()
+    for (x, cuts, nc, dig), e in zip(jobs, exp):
+        assert np.array_equal(dig.view(-1, 32).cpu().numpy(), e)
+
+
 @pytest.mark.parametrize("bounded", [False, True])
 def test_chunk_then_hash_on_device(pkg, bounded):
     """Chunking -> hashing chained on one stream (the cut count never leaves the device)."""
