@@ -42,12 +42,28 @@ def main():
     check(pkg.Chunker(pkg.Params(divisor=3 << 32, magic=77)), data[:300000], 1)          # MK_REM '=='
     check(pkg.Chunker(pkg.Params(poly=0x104C11DB7, divisor=1000, magic=2, marker=1)), data[:300000])  # MK_REM, u32
     check(pkg.Chunker(pkg.Params(poly=0x11D, window=20, divisor=256, magic=9)), data[:300000], 4)      # degree 8
+    check(pkg.Chunker(pkg.Params(poly=0x80002001)), data)                                 # K32T, aligned start (no head)
+    check(pkg.Chunker(pkg.Params(poly=0x80002001, window=31, marker=1, magic=3)), data[:300000], 9)    # K32T funnel '<='
+    check(pkg.Chunker(pkg.Params()), data[: (1 << 20)])                                 # small shape, 32-B rows
+    check(pkg.Chunker(pkg.Params(divisor=4096, magic=77, marker=1)), data[:500000], 6)   # '<=' lists sized by rate
     # f2 / f3: SHA-256 of every chunk (hashlib oracle) and the dedup index
     chh = pkg.Chunker(pkg.Params())
     x = torch.from_numpy(data).cuda()
     cuts = chh.chunk(x)
     dig = chh.hash_chunks(x, cuts).cpu().numpy()
     assert np.array_equal(dig, oracle.chunk_digests(data, cuts.cpu().numpy().astype(np.uint64)))
+    # batched hashing over two buffers, one of them at an unaligned address
+    x2 = torch.from_numpy(data[1:200001].copy()).cuda()
+    c2 = chh.chunk(x2)
+    n1 = torch.tensor([cuts.numel()], dtype=torch.int64, device="cuda")
+    n2 = torch.tensor([c2.numel()], dtype=torch.int64, device="cuda")
+    d1 = torch.empty((cuts.numel() + 1) * 32, dtype=torch.uint8, device="cuda")
+    d2 = torch.empty((c2.numel() + 1) * 32, dtype=torch.uint8, device="cuda")
+    chh.hash_chunks_batch_async([(x, cuts, n1, d1), (x2, c2, n2, d2)])
+    torch.cuda.synchronize()
+    assert np.array_equal(d1.view(-1, 32).cpu().numpy(), dig)
+    assert np.array_equal(d2.view(-1, 32).cpu().numpy(),
+                          oracle.chunk_digests(data[1:200001], c2.cpu().numpy().astype(np.uint64)))
     chh.index_reset(1 << 12)
     n_c = torch.tensor([cuts.numel()], dtype=torch.int64, device="cuda")
     chh.index_insert_async(torch.from_numpy(dig.reshape(-1)).cuda(), cuts, n_c, data.size)
