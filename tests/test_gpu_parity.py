@@ -179,6 +179,34 @@ def test_size_bound_state_chains_over_virtual_shards(pkg):
         assert np.array_equal(np.concatenate(got).astype(np.uint64), exp)
 
 
+def test_size_bound_state_dev_chains_with_device_states(pkg):
+    """shred_size_bound_state_dev: the same chaining with the candidate count and the entry
+    state read from device memory and the exit state left there (no host value between the
+    pieces); the candidate buffer is larger than the count (the count bounds the work)."""
+    n = (7 << 20) + 99
+    data = synthgen.random_bytes(18, n)
+    p = pkg.Params(divisor=512, min_size=300, max_size=4000)
+    ch = pkg.Chunker(p)
+    cand = oracle.candidates(data, oracle.Params(divisor=512)).astype(np.int64)
+    exp = oracle.size_bound(cand.astype(np.uint64), n, 300, 4000)
+    G = 5
+    bounds = [n * g // G for g in range(G + 1)]
+    state = torch.zeros(2, dtype=torch.int64, device="cuda")
+    outs = []
+    for g in range(G):
+        a, b = bounds[g], bounds[g + 1]
+        part = cand[(cand > a) & (cand <= b)]
+        buf = torch.full((part.size + 100,), -1, dtype=torch.int64, device="cuda")
+        buf[:part.size] = torch.from_numpy(part.copy()).cuda()
+        nd = torch.tensor([part.size], dtype=torch.int64, device="cuda")
+        out = torch.empty(part.size + (b - a) // 4000 + 8, dtype=torch.int64, device="cuda")
+        no = torch.zeros(1, dtype=torch.int64, device="cuda")
+        ch.size_bound_state_dev(buf, nd, b, b == n, state, out, no, state)
+        outs.append((out, no))
+    got = np.concatenate([o[:int(k.item())].cpu().numpy() for o, k in outs]).astype(np.uint64)
+    assert np.array_equal(got, exp)
+
+
 # ------------------------------------------------------------------ streaming (config 3 shape)
 def _feed_all(ch, data, sizes, pinned):
     outs = []
