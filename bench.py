@@ -696,6 +696,13 @@ def main():
                                     "params": "P=x^31+x^13+1 (0x80002001, irreducible trinomial), other params as paper",
                                     "mode": c3t.mode}
             del c3t
+            # the u64-state analogue (MODE_K63T) for a sparse degree-63 polynomial
+            c6t = pkg.Chunker(pkg.Params(poly=0x8000000000000801), device=local)
+            v6t = timed(c6t, base)
+            line["k63t_variant"] = {"value": round(v6t, 2), "unit": "GB/s", "hbm_frac": round(v6t / hbm, 4),
+                                    "params": "P=x^63+x^11+1 (0x8000000000000801, irreducible trinomial), other params as paper",
+                                    "mode": c6t.mode}
+            del c6t
             # content sensitivity. Text-like bytes (words from a fixed
             # 1,000-word list; skewed outgoing bytes for the U lookups), 64 MiB generated on the
             # host and tiled to 256 MiB on the device; paper params on the same ctx.

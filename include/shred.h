@@ -111,7 +111,8 @@ int         shred_path(const shred_ctx *ctx);         /* SHRED_PATH_* chosen at 
 /* The hot kernel's state mode (diagnostics): 1 K63 (u64 state, deg 41..63), 5 K40 (deg 33..40),
    2 K32 (u32 state, T by table), 4 K32B (u32, whole-byte top byte: deg 8/16/24/32), 6 K32T (u32,
    T as one integer product: P = x^k + Q with Q's terms >= 8 apart and below k - 7, e.g. the
-   trinomial x^31 + x^13 + 1; '==' and '<=' with D = 2^m), 3 generic. */
+   trinomial x^31 + x^13 + 1; '==' and '<=' with D = 2^m), 7 K63T (the u64-state analogue for
+   deg 41..63 with Q's terms below 25, e.g. x^63 + x^11 + 1), 3 generic. */
 int         shred_kernel_mode(const shred_ctx *ctx);
 int         shred_get_params(const shred_ctx *ctx, shred_params *out);
 
@@ -255,10 +256,13 @@ int shred_check_params(const shred_params *p, int *path_out, int *marker_kind_ou
 int shred_debug_plan(int path, int small_ok, int sm_count, uint64_t src_addr, uint64_t p_begin,
                      uint64_t t_begin, uint64_t t_end, uint64_t divisor, uint32_t window, int zero_lead,
                      uint64_t out[16]);
-/* Test hook (host logic, no GPU): 1 if the K32T kernel mode applies to poly (deg <= 32 and
-   P = x^k + Q with Q's terms >= 8 apart and below k - 7), with *mult = Q + 2^k mod 2^32, the
-   integer multiplier that gives T[t] = t(x) x^k mod P ^ (t << k mod 2^32) as t * mult mod 2^32. */
-int shred_debug_tprod(uint64_t poly, uint32_t *mult);
+/* Test hook (host logic, no GPU): 1 if a multiply-reduction kernel mode applies to poly
+   (P = x^k + Q with Q's terms >= 8 apart): K32T for deg <= 32 with the terms below k - 7,
+   *mult = Q + 2^k mod 2^32, so T[t] = t(x) x^k mod P ^ (t << k mod 2^32) = t * mult mod 2^32;
+   K63T for deg 41..63 with the terms below 25, *mult = Q (low word of T) and
+   *mult_hi = 2^(k-32) (high word: the cancel term), so T[t] = (t * mult_hi : t * mult).
+   mult / mult_hi may be NULL. */
+int shred_debug_tprod(uint64_t poly, uint32_t *mult, uint32_t *mult_hi);
 int shred_profile_read(shred_ctx *ctx, double *ms, uint64_t *launches, uint64_t *bytes);
 
 #ifdef __cplusplus

@@ -166,8 +166,8 @@ class Chunker:
 
     @property
     def mode(self) -> str:
-        """The hot kernel's state mode (k63, k40, k32, k32b, k32t, generic)."""
-        return {1: "k63", 2: "k32", 3: "generic", 4: "k32b", 5: "k40", 6: "k32t"}.get(
+        """The hot kernel's state mode (k63, k40, k63t, k32, k32b, k32t, generic)."""
+        return {1: "k63", 2: "k32", 3: "generic", 4: "k32b", 5: "k40", 6: "k32t", 7: "k63t"}.get(
             lib().shred_kernel_mode(self._ctx), "?")
 
     @property

@@ -20,11 +20,11 @@ DEPS = SOURCES + [os.path.join(CSRC, f) for f in ("kernels.cuh", "size_bound.cuh
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 CFLAGS = ["-O3", "-std=c++17", "-lineinfo", "-gencode", "arch=compute_100a,code=sm_100a",
           "-Xcompiler", "-fPIC,-O2", "--expt-relaxed-constexpr", "-Xptxas", "-v"]
-# object -> (source, extra defines); SHRED_INST = kernels.cuh MODE_* (K63 1, K32 2, K32B 4, K40 5, K32T 6)
+# object -> (source, extra defines); SHRED_INST = kernels.cuh MODE_* (K63 1, K32 2, K32B 4, K40 5, K32T 6, K63T 7)
 UNITS = [("shred", "shred.cu", ()), ("k1_sel", "k1_inst.cu", ("SHRED_INST=0",)),
          ("k1_k63", "k1_inst.cu", ("SHRED_INST=1",)), ("k1_k32", "k1_inst.cu", ("SHRED_INST=2",)),
          ("k1_k32b", "k1_inst.cu", ("SHRED_INST=4",)), ("k1_k40", "k1_inst.cu", ("SHRED_INST=5",)),
-         ("k1_k32t", "k1_inst.cu", ("SHRED_INST=6",))]
+         ("k1_k32t", "k1_inst.cu", ("SHRED_INST=6",)), ("k1_k63t", "k1_inst.cu", ("SHRED_INST=7",))]
 
 
 def stale() -> bool:

@@ -34,13 +34,15 @@ static K1Fn pick_w(int wch, bool fn) {
 }
 template <int MODE>
 K1Fn pick_mode(int wch, int mk, bool fn) {
-    using C = typename std::conditional<MODE == MODE_K63 || MODE == MODE_K40, CfgK63, CfgK32>::type;
-    if (MODE == MODE_K32T && mk != MK_EQ && mk != MK_LE) return nullptr;   // other kinds: MODE_K32
+    using C = typename std::conditional<MODE == MODE_K63 || MODE == MODE_K40 || MODE == MODE_K63T, CfgK63,
+                                        CfgK32>::type;
+    constexpr bool TP = MODE == MODE_K32T || MODE == MODE_K63T;
+    if (TP && mk != MK_EQ && mk != MK_LE) return nullptr;   // other kinds: the table modes
     switch (mk) {
         case MK_EQ: return pick_w<MODE, C, MK_EQ>(wch, fn);
         case MK_LE: return pick_w<MODE, C, MK_LE>(wch, fn);
-        case MK_DIV: return MODE == MODE_K32T ? nullptr : pick_w<MODE, C, MK_DIV>(wch, fn);
-        case MK_REM: return MODE == MODE_K32T ? nullptr : pick_w<MODE, C, MK_REM>(wch, fn);
+        case MK_DIV: return TP ? nullptr : pick_w<MODE, C, MK_DIV>(wch, fn);
+        case MK_REM: return TP ? nullptr : pick_w<MODE, C, MK_REM>(wch, fn);
         default: return nullptr;
     }
 }
@@ -48,10 +50,15 @@ template K1Fn pick_mode<SHRED_INST>(int, int, bool);
 #else
 // The instance for (u64 state: deg 41..63 | deg 33..40; u32 state with a whole-byte top byte |
 // u32 state; ceil(w/16), marker kind, w % 16 != 0).
-// tprod: deg <= 32 and P = x^k + Q with Q's terms >= 8 apart below k - 7 (MODE_K32T, '==' and
-// '<=' with D = 2^m); otherwise the table modes.
+// tprod: P = x^k + Q with Q's terms >= 8 apart, below k - 7 (deg <= 32: MODE_K32T) or below 25
+// (deg 41..63: MODE_K63T), '==' and '<=' with D = 2^m; otherwise the table modes.
 K1Fn pick_k1(int k, bool byteidx, int wch, int mk, bool fn, bool tprod) {
-    if (k >= 41) return pick_mode<MODE_K63>(wch, mk, fn);
+    if (k >= 41) {
+        if (tprod) {
+            if (K1Fn f = pick_mode<MODE_K63T>(wch, mk, fn)) return f;
+        }
+        return pick_mode<MODE_K63>(wch, mk, fn);
+    }
     if (k >= 33) return pick_mode<MODE_K40>(wch, mk, fn);
     if (tprod) {
         if (K1Fn f = pick_mode<MODE_K32T>(wch, mk, fn)) return f;
@@ -61,7 +68,7 @@ K1Fn pick_k1(int k, bool byteidx, int wch, int mk, bool fn, bool tprod) {
 // The small-input shape (CfgSmall) exists for the paper's window with the equality marker.
 K1Fn pick_k1_small(int k, bool byteidx, int wch, int mk, bool fn, bool tprod) {
     if (wch != 3 || mk != MK_EQ || fn || (k >= 33 && k <= 40)) return nullptr;
-    if (k >= 41) return k1_bulk<MODE_K63, CfgSmall, 3, MK_EQ>;
+    if (k >= 41) return tprod ? k1_bulk<MODE_K63T, CfgSmall, 3, MK_EQ> : k1_bulk<MODE_K63, CfgSmall, 3, MK_EQ>;
     if (tprod) return k1_bulk<MODE_K32T, CfgSmall, 3, MK_EQ>;
     return byteidx ? k1_bulk<MODE_K32B, CfgSmall, 3, MK_EQ> : k1_bulk<MODE_K32, CfgSmall, 3, MK_EQ>;
 }

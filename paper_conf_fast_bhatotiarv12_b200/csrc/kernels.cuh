@@ -45,7 +45,9 @@ namespace shred {
 // K32T: u32 state, deg 9..32, P = x^k + Q with the terms of Q at least 8 apart and below k-7:
 // the reduction of the top byte, t(x) Q(x), is then an integer product (no carries between the
 // shifted copies of t), so T costs one IMAD instead of a shared-memory lookup.
-enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3, MODE_K32B = 4, MODE_K40 = 5, MODE_K32T = 6 };
+// K63T: the same for the u64 state (deg 41..63, Q's terms below 25 so t(x) Q(x) fits the low
+// word; the cancel term t << k lands in the high word): two IMADs instead of an LDS.64.
+enum { MODE_K63 = 1, MODE_K32 = 2, MODE_GENERIC = 3, MODE_K32B = 4, MODE_K40 = 5, MODE_K32T = 6, MODE_K63T = 7 };
 
 #ifndef SHRED_STAGES
 #define SHRED_STAGES 2   // A/B (profiles/r01_ab_variants.txt): 2 stages 1,879 GB/s > 3: 1,861 > 4: 1,854
@@ -457,7 +459,9 @@ struct BulkCtx {
     uint32_t tmul;      // 2^(32-m): (f_lo * tmul) keeps the low m bits at the top
     uint32_t rsh;       // r << (32-m)
     uint32_t tsel;      // K32B: PRMT selector 0x55s4 placing byte s = (k-8)/8 of f at bits 8..15
-    uint32_t tshr, tprod;       // K32T: k - 8, M = Q + 2^k mod 2^32
+    uint32_t tshr, tprod;       // K32T: k - 8, M = Q + 2^k mod 2^32; K63T: k - 40, Q
+    uint32_t tprod_hi;          // K63T: 2^(k-32) (the cancel term t << k in the high word)
+    uint32_t dm32, r32;         // D - 1 and r as u32 (MK_EQ / MK_LE, D <= 2^32; SHRED_MARK_LOP)
     // MK_DIV (any D = d 2^s, s < 32): f mod D == r  <=>  D | (f + D - r)  (no overflow: f < 2^63,
     // D - r <= 2^63)  <=>  rotr64((f + D - r) * d^-1 mod 2^64, s) <= floor((2^64 - 1) / D)
     uint64_t dc;        // D - r
@@ -477,10 +481,19 @@ struct BulkCtx {
 //   T[t] = (t x^k mod P) ^ ((t << k) mod 2^64) cancels the byte the shift leaves at bits
 //   k..k+7 (k = 63: the one bit at 2^63), U[o] = o x^{8w} mod P.  Shift-in by two PRMTs.
 // deg 33..40 (FUNNEL): the top byte straddles the two words, t = funnel(fl, fh) >> (k-8).
+// The top byte t = f >> (k-8) by SHF on the ALU pipe, not by mulhi: IMAD.HI runs on the
+// half-rate fmaheavy pipe, and on the state's dependency chain its latency showed: k63 paper path
+// 1,922 -> 1,994 GB/s (k1_bulk, 1 GiB; profiles/r02_k32_ab.txt).  0: IMAD.HI (round 1).
+#ifndef SHRED_K63_SHF
+#define SHRED_K63_SHF 1
+#endif
+#ifndef SHRED_K32_SHF
+#define SHRED_K32_SHF 1
+#endif
 template <int K, bool FUNNEL = false>
 __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, uint32_t pop,
                                        const BulkCtx &c) {
-    const uint32_t t  = FUNNEL ? __funnelshift_rc(fl, fh, c.mhi) : __umulhi(fh, c.mhi);
+    const uint32_t t  = FUNNEL ? __funnelshift_rc(fl, fh, c.mhi) : SHRED_K63_SHF ? fh >> c.tshr : __umulhi(fh, c.mhi);
     const uint32_t ti = t * c.m256 + c.laneT;
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
     const uint2 T = lds64(ti);
@@ -499,7 +512,7 @@ __device__ __forceinline__ void step32(uint32_t &f, uint32_t in, uint32_t pop, c
     if (BYTEIDX)   // deg 16/24/32: t = f >> (k-8) is a whole byte -> one PRMT builds (t << 8) | lane*4
         ti = c.tab + __byte_perm(f, c.laneT - c.tab, c.tsel);
     else
-        ti = __umulhi(f, c.mhi) * c.m256 + c.laneT;
+        ti = (SHRED_K32_SHF ? f >> c.tshr : __umulhi(f, c.mhi)) * c.m256 + c.laneT;
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
     const uint32_t T = lds32(ti);
     const uint32_t U = lds32(c.tab + oi);
@@ -521,8 +534,35 @@ __device__ __forceinline__ void step32t(uint32_t &f, uint32_t in, uint32_t pop, 
     f = __byte_perm(f, in, 0x2104u + K) ^ T ^ U;
 }
 
+// One byte step, K63T (u64 state, deg k in 41..63): t = f >> (k-8) = fh >> (k-40) (SHF),
+// T = (t * 2^(k-32) mod 2^32) : (t * Q) (the carry-free product in the low word, the cancel term
+// in the high word), f <- (f << 8 mod 2^64) ^ B ^ T ^ U[o]; U is the only lookup.
+#ifndef SHRED_K63T_SHF
+#define SHRED_K63T_SHF 1   // A/B: the top byte by IMAD.HI (fmaheavy) instead: 2,227 -> 2,087 GB/s
+#endif
+template <int K>
+__device__ __forceinline__ void step63t(uint32_t &fl, uint32_t &fh, uint32_t in, uint32_t pop,
+                                        const BulkCtx &c) {
+    const uint32_t t = SHRED_K63T_SHF ? fh >> c.tshr : __umulhi(fh, c.mhi);
+    const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
+    const uint2 U = lds64(c.tab + oi);
+    const uint32_t nh = __byte_perm(fh, fl, 0x2107u);
+    const uint32_t nl = __byte_perm(fl, in, 0x2104u + K);
+    fl = nl ^ (t * c.tprod) ^ U.x;
+    fh = nh ^ (t * c.tprod_hi) ^ U.y;
+}
+
 template <int MODE>
 struct State;
+template <> struct State<MODE_K63T> {
+    uint32_t fl = 0, fh = 0;
+    __device__ __forceinline__ void set(uint64_t v) { fl = (uint32_t)v; fh = (uint32_t)(v >> 32); }
+    template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
+        step63t<K>(fl, fh, in, pop, c);
+    }
+    __device__ __forceinline__ uint32_t low() const { return fl; }
+    __device__ __forceinline__ uint64_t full() const { return ((uint64_t)fh << 32) | fl; }
+};
 template <> struct State<MODE_K32T> {
     uint32_t f = 0;
     __device__ __forceinline__ void set(uint64_t v) { f = (uint32_t)v; }
@@ -579,15 +619,20 @@ enum { MK_EQ = 0, MK_LE = 1, MK_DIV = 2, MK_REM = 3 };
 __device__ __forceinline__ bool is_marker(uint32_t lo, const BulkCtx &c) { return lo * c.tmul == c.rsh; }
 // m | BIT if marker else m: ISETP + predicated LOP3 (the PTX predication survives ptxas).
 // LE: the "mod D <= r" marker set (L249-L251): (f_lo << (32-m)) <= (r << (32-m)).
+// SHRED_MARK_LOP: the low m bits by a LOP3 mask (ALU) instead of the IMAD shift (fmaheavy).
+#ifndef SHRED_MARK_LOP
+#define SHRED_MARK_LOP 0
+#endif
 template <uint32_t BIT, int MK>
 __device__ __forceinline__ uint32_t or_if_marker(uint32_t m, uint32_t lo, const BulkCtx &c) {
-    const uint32_t x = lo * c.tmul;
+    const uint32_t x = SHRED_MARK_LOP ? (lo & c.dm32) : lo * c.tmul;
+    const uint32_t y = SHRED_MARK_LOP ? c.r32 : c.rsh;
     if (MK == MK_LE)
         asm("{\n .reg .pred p;\n setp.le.u32 p, %1, %2;\n @p or.b32 %0, %0, %3;\n}"
-            : "+r"(m) : "r"(x), "r"(c.rsh), "n"(BIT));
+            : "+r"(m) : "r"(x), "r"(y), "n"(BIT));
     else
         asm("{\n .reg .pred p;\n setp.eq.u32 p, %1, %2;\n @p or.b32 %0, %0, %3;\n}"
-            : "+r"(m) : "r"(x), "r"(c.rsh), "n"(BIT));
+            : "+r"(m) : "r"(x), "r"(y), "n"(BIT));
     return m;
 }
 
@@ -703,7 +748,9 @@ __device__ __forceinline__ void chunk16xN(State<MODE> (&st)[CH], const uint4 (&d
 
 struct BulkConst {
     uint32_t mhi, m256, tmul, rsh, tsel;
-    uint32_t tshr, tprod;      // K32T (BulkCtx)
+    uint32_t tshr, tprod;      // K32T / K63T (BulkCtx)
+    uint32_t tprod_hi;         // K63T (BulkCtx)
+    uint32_t dm32, r32;        // BulkCtx
     uint64_t dc, dinv, dlim;   // MK_DIV constants (BulkCtx)
     uint32_t dsh;
     uint64_t rm, rd, rlo, rspan;   // MK_REM constants (BulkCtx)
@@ -843,7 +890,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     const int lane = tid & 31;
     BulkCtx c;
     c.tab = sbase;
-    if (MODE == MODE_K63 || MODE == MODE_K40) {
+    if (MODE == MODE_K63 || MODE == MODE_K40 || MODE == MODE_K63T) {
         c.laneT = sbase + (uint32_t)(lane & 15) * 8u;
         c.laneU = 128u + (uint32_t)(lane & 15) * 8u;
     } else {
@@ -851,7 +898,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
         c.laneU = 128u + (uint32_t)lane * 4u;
     }
     c.mhi = K.mhi; c.m256 = K.m256; c.tmul = K.tmul; c.rsh = K.rsh; c.tsel = K.tsel;
-    c.tshr = K.tshr; c.tprod = K.tprod;
+    c.tshr = K.tshr; c.tprod = K.tprod; c.tprod_hi = K.tprod_hi; c.dm32 = K.dm32; c.r32 = K.r32;
     c.dc = K.dc; c.dinv = K.dinv; c.dlim = K.dlim; c.dsh = K.dsh;
     c.rm = K.rm; c.rd = K.rd; c.rlo = K.rlo; c.rspan = K.rspan; c.rsh2 = K.rsh2;
 

@@ -229,16 +229,21 @@ int grow(shred_ctx *ctx, T *&ptr, uint64_t &cap, uint64_t need, const char *what
 // below k - 7, so t(x) Q(x) for a byte t is the integer product t * Q (the shifted copies of t
 // never overlap) of degree < k (no second reduction).  The multiplier adds the cancel term:
 // M = Q + 2^k mod 2^32.
-bool tprod_ok(uint64_t P, int k, uint32_t *mult) {
-    if (k < 9 || k > 32) return false;
+// Degrees 41..63 (MODE_K63T): Q's terms at least 8 apart and below 25, so t(x) Q(x) = t * Q fits
+// the low word; the cancel term (t << k) mod 2^64 is t * 2^(k-32) in the high word (mult_hi).
+bool tprod_ok(uint64_t P, int k, uint32_t *mult, uint32_t *mult_hi = nullptr) {
+    const bool u64 = k >= 41 && k <= 63;
+    if (!u64 && (k < 9 || k > 32)) return false;
+    const int top = u64 ? 32 : k;                  // every term e needs e + 7 < top
     const uint64_t Q = P ^ (1ull << k);
     int prev = -100;
     for (int e = 0; e < k; ++e) {
         if (!((Q >> e) & 1u)) continue;
-        if (e - prev < 8 || e + 7 >= k) return false;
+        if (e - prev < 8 || e + 7 >= top) return false;
         prev = e;
     }
-    if (mult) *mult = (uint32_t)(Q + (k < 32 ? (1ull << k) : 0ull));
+    if (mult) *mult = u64 ? (uint32_t)Q : (uint32_t)(Q + (k < 32 ? (1ull << k) : 0ull));
+    if (mult_hi) *mult_hi = u64 ? (1u << (k - 32)) : 0u;
     return true;
 }
 
@@ -472,9 +477,10 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         K.m256 = 256u;
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
         K.rsh = (uint32_t)(ctx->p.magic << m);
-        K.tshr = (uint32_t)(ctx->k - 8);
-        K.tprod = 0u;
-        tprod_ok(ctx->p.poly, ctx->k, &K.tprod);
+        K.tshr = (uint32_t)(ctx->k >= 41 ? ctx->k - 40 : ctx->k - 8);
+        K.tprod = 0u; K.tprod_hi = 0u;
+        K.dm32 = (uint32_t)(ctx->p.divisor - 1u); K.r32 = (uint32_t)ctx->p.magic;
+        tprod_ok(ctx->p.poly, ctx->k, &K.tprod, &K.tprod_hi);
         {   // MK_DIV: D = d 2^s; d^-1 mod 2^64 by Newton's iteration (d odd: d*d = 1 mod 8)
             const uint64_t D = ctx->p.divisor;
             const uint32_t sh = (uint32_t)__builtin_ctzll(D);
@@ -762,11 +768,11 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         const bool byteidx = SHRED_BYTEIDX && ctx->path == SHRED_PATH_K32 && (k == 8 || k == 16 || k == 24 || k == 32);
         const int wch = (int)((p->window + 15) / 16);
         const bool funnel = p->window % 16 != 0;
-        const bool tprod = SHRED_TPROD && ctx->path == SHRED_PATH_K32 && tprod_ok(p->poly, k, nullptr);
+        const bool tprod = SHRED_TPROD && (ctx->path == SHRED_PATH_K32 || k >= 41) && tprod_ok(p->poly, k, nullptr);
         ctx->k1_fn = pick_k1(k, byteidx, wch, ctx->mk, funnel, tprod);
-        ctx->mode = tprod && (ctx->mk == MK_EQ || ctx->mk == MK_LE) ? MODE_K32T
-                  : ctx->path == SHRED_PATH_K63 ? (k >= 41 ? MODE_K63 : MODE_K40)
-                  : (byteidx ? MODE_K32B : MODE_K32);
+        const bool tmode = tprod && (ctx->mk == MK_EQ || ctx->mk == MK_LE);
+        ctx->mode = ctx->path == SHRED_PATH_K63 ? (k >= 41 ? (tmode ? MODE_K63T : MODE_K63) : MODE_K40)
+                  : tmode ? MODE_K32T : (byteidx ? MODE_K32B : MODE_K32);
         if (!ctx->k1_fn ||
             cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM) != cudaSuccess)
@@ -1208,10 +1214,11 @@ int shred_debug_plan(int path, int small_ok, int sm_count, uint64_t src_addr, ui
     return SHRED_OK;
 }
 
-int shred_debug_tprod(uint64_t poly, uint32_t *mult) {
-    uint32_t m = 0;
-    const int ok = tprod_ok(poly, deg64(poly), &m) ? 1 : 0;
+int shred_debug_tprod(uint64_t poly, uint32_t *mult, uint32_t *mult_hi) {
+    uint32_t m = 0, mh = 0;
+    const int ok = tprod_ok(poly, deg64(poly), &m, &mh) ? 1 : 0;
     if (mult) *mult = m;
+    if (mult_hi) *mult_hi = mh;
     return ok;
 }
 

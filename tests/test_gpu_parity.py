@@ -561,7 +561,8 @@ def test_remainder_marker_hot_kernel(pkg, poly, D):
 
 
 # ------------------------------------------------------------------ K32T (T as an integer product)
-@pytest.mark.parametrize("poly", [0x80002001, 0x80040001, 0x40200001, 0x10000201, 0x800201, 0x40201])
+@pytest.mark.parametrize("poly", [0x80002001, 0x80040001, 0x40200001, 0x10000201, 0x800201, 0x40201,
+                                  0x8000000000000801])     # the last: K63T (u64 state)
 @pytest.mark.parametrize("window,marker", [(48, 0), (48, 1), (32, 0), (47, 0), (16, 1)])
 def test_k32t_multiply_reduction_paths(pkg, poly, window, marker):
     """Sparse irreducible P (Q's terms >= 8 apart): the u32 kernel reduces the top byte with one
@@ -571,7 +572,7 @@ def test_k32t_multiply_reduction_paths(pkg, poly, window, marker):
     D = 512 if poly < (1 << 20) else 4096
     p = pkg.Params(poly=poly, window=window, divisor=D, magic=7 if not marker else 3, marker=marker)
     ch = pkg.Chunker(p)
-    assert ch.mode == "k32t" and ch.path == "k32"
+    assert (ch.mode, ch.path) == (("k63t", "k63") if poly >> 40 else ("k32t", "k32"))
     got = check_chunk(ch, data)
     pb = pkg.Params(poly=poly, window=window, divisor=D, magic=7 if not marker else 3, marker=marker,
                     min_size=D // 4, max_size=8 * D)
@@ -597,7 +598,9 @@ def test_k32t_small_shape_and_le_marker_modes(pkg):
     for p, mode in ((pkg.Params(poly=0x80002001), "k32t"),
                     (pkg.Params(poly=0x80002001, divisor=1 << 20, magic=12345), "k32t"),
                     (pkg.Params(poly=0x80002001, divisor=10000, magic=7), "k32"),      # MK_DIV: table mode
-                    (pkg.Params(poly=0x104C11DB7), "k32b"), (pkg.Params(), "k63")):
+                    (pkg.Params(poly=0x104C11DB7), "k32b"), (pkg.Params(), "k63"),
+                    (pkg.Params(poly=0x8000000000000801), "k63t"),
+                    (pkg.Params(poly=0x8000000000000801, divisor=10000, magic=9), "k63")):
         ch = pkg.Chunker(p)
         assert ch.mode == mode, (p, ch.mode)
         check_chunk(ch, data)

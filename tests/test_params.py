@@ -97,14 +97,14 @@ def test_k32t_multiplier_equals_the_reduction_table():
     from paper_conf_fast_bhatotiarv12_b200 import _build
     lib = ctypes.CDLL(_build.build())
     f = lib.shred_debug_tprod
-    f.argtypes = [ctypes.c_uint64, ctypes.POINTER(ctypes.c_uint32)]
+    f.argtypes = [ctypes.c_uint64, ctypes.POINTER(ctypes.c_uint32), ctypes.POINTER(ctypes.c_uint32)]
     f.restype = ctypes.c_int
     eligible = [0x80002001, 0x80040001, 0x40200001, 0x40000201, 0x10000201, 0x10002001, 0x800201,
                 0x804001, 0x40201]
     for P in eligible:
         assert oracle.is_irreducible(P)
         m = ctypes.c_uint32(0)
-        assert f(P, ctypes.byref(m)) == 1, hex(P)
+        assert f(P, ctypes.byref(m), None) == 1, hex(P)
         k = P.bit_length() - 1
         for t in range(256):
             # t(x) x^k mod P by R1 on the message t || zero bits: shift t by k bits via bytes
@@ -114,4 +114,19 @@ def test_k32t_multiplier_equals_the_reduction_table():
             exp = red ^ ((t << k) & 0xFFFFFFFF)
             assert (t * m.value) & 0xFFFFFFFF == exp, (hex(P), t)
     for P in (0x104C11DB7, LBFS, 0x8000000B, 0x80000081, 0x20000005, (1 << 31) | (1 << 24) | 1):
-        assert f(P, None) == 0, hex(P)
+        assert f(P, None, None) == 0, hex(P)
+    # K63T (deg 41..63): T[t] = (t * mult_hi mod 2^32) : (t * mult) == t(x) x^k mod P ^ (t << k mod 2^64)
+    for P in (0x8000000000000801,):
+        assert oracle.is_irreducible(P)
+        m, mh = ctypes.c_uint32(0), ctypes.c_uint32(0)
+        assert f(P, ctypes.byref(m), ctypes.byref(mh)) == 1
+        k = P.bit_length() - 1
+        for t in range(256):
+            msg = t << k
+            red = oracle.polymod(np.frombuffer(msg.to_bytes((msg.bit_length() + 7) // 8 or 1, "big"), np.uint8), P)
+            exp = red ^ ((t << k) & 0xFFFFFFFFFFFFFFFF)
+            got = (((t * mh.value) & 0xFFFFFFFF) << 32) | ((t * m.value) & 0xFFFFFFFF)
+            assert got == exp, t
+    # deg 41..63 with a term too high for the low word, or too close: refused
+    for P in (LBFS, (1 << 63) | (1 << 25) | 1, (1 << 63) | (1 << 7) | 1, (1 << 50) | (1 << 30) | 1):
+        assert f(P, None, None) == 0, hex(P)

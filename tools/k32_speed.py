@@ -19,7 +19,8 @@ cases = {"k32t (x^31+x^13+1)": pkg.Params(poly=0x80002001),
          "k32b (0x104C11DB7)": pkg.Params(poly=0x104C11DB7),
          "k32 (deg 29)": pkg.Params(poly=0x20000005 if len(sys.argv) < 2 else int(sys.argv[1], 0)),
          "k32b le r=1": pkg.Params(poly=0x104C11DB7, marker=1, magic=1),
-         "k63 (paper)": pkg.Params()}
+         "k63 (paper)": pkg.Params(),
+         "k63t (x^63+x^11+1)": pkg.Params(poly=0x8000000000000801)}
 out = torch.empty(n // 512, dtype=torch.int64, device="cuda")
 nn = torch.zeros(1, dtype=torch.int64, device="cuda")
 for name, p in cases.items():
