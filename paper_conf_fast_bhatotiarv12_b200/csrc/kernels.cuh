@@ -490,11 +490,14 @@ struct BulkCtx {
 #ifndef SHRED_K32_SHF
 #define SHRED_K32_SHF 1
 #endif
+#ifndef SHRED_TIDX_LEA
+#define SHRED_TIDX_LEA 1  // T row index (t << 8) + lane by LEA (ALU), not IMAD (fmaheavy): k63 1,997 -> 2,005 GB/s
+#endif
 template <int K, bool FUNNEL = false>
 __device__ __forceinline__ void step63(uint32_t &fl, uint32_t &fh, uint32_t in, uint32_t pop,
                                        const BulkCtx &c) {
     const uint32_t t  = FUNNEL ? __funnelshift_rc(fl, fh, c.mhi) : SHRED_K63_SHF ? fh >> c.tshr : __umulhi(fh, c.mhi);
-    const uint32_t ti = t * c.m256 + c.laneT;
+    const uint32_t ti = SHRED_TIDX_LEA ? (t << 8) + c.laneT : t * c.m256 + c.laneT;
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
     const uint2 T = lds64(ti);
     const uint2 U = lds64(c.tab + oi);
@@ -512,7 +515,8 @@ __device__ __forceinline__ void step32(uint32_t &f, uint32_t in, uint32_t pop, c
     if (BYTEIDX)   // deg 16/24/32: t = f >> (k-8) is a whole byte -> one PRMT builds (t << 8) | lane*4
         ti = c.tab + __byte_perm(f, c.laneT - c.tab, c.tsel);
     else
-        ti = (SHRED_K32_SHF ? f >> c.tshr : __umulhi(f, c.mhi)) * c.m256 + c.laneT;
+        ti = SHRED_TIDX_LEA ? ((f >> c.tshr) << 8) + c.laneT
+                            : (SHRED_K32_SHF ? f >> c.tshr : __umulhi(f, c.mhi)) * c.m256 + c.laneT;
     const uint32_t oi = __byte_perm(pop, c.laneU, 0x5504u | (K << 4));
     const uint32_t T = lds32(ti);
     const uint32_t U = lds32(c.tab + oi);
