@@ -764,6 +764,7 @@ def main():
             ch.chunk_async(base, out0, n0)
             ch.chunk_async(edited, out1, n1)
             ch.hash_chunks_async(base, out0, n0, digs[0])
+            ch.hash_chunks_batch_async([(base, out0, n0, d) for d in digs])     # grows the work list once
             torch.cuda.synchronize()
             h0, h1, h2, h3 = (torch.cuda.Event(enable_timing=True) for _ in range(4))
             h0.record(stream)
