@@ -1,10 +1,11 @@
 """Multi-process (gloo, world size 2 and 3, CPU) tests of the sharding orchestration (dist.py).
 
 The per-shard engine here is the CPU oracle (test infrastructure), so these tests pin the
-host logic: shard bounds, halos, the count all-gather and global offsets (C2), and the bounded
-mode's candidate all-gather + global size rule (C3).  The CUDA engine is the same interface
-(Chunker.candidates_range / size_bound) and is covered by tests/test_gpu_parity.py (virtual
-shards) on one GPU.
+host logic: shard bounds, halos, the count all-gather and global offsets (C2), the distributed
+size rule ("chain") and the C3 gather — through both engine interfaces dist.chunk_sharded
+accepts: the synchronous one and the asynchronous one the CUDA Chunker has (counts, entry and
+exit states in tensors; an undersized candidate buffer redone exactly).  The CUDA engine itself
+runs the same code in tests/test_gpu_dist.py (2-3 processes on one GPU).
 """
 import os
 import socket
@@ -45,6 +46,28 @@ class OracleEngine:
                                                   self.params.min_size, self.params.max_size).astype(np.int64))
 
 
+class OracleAsyncEngine(OracleEngine):
+    """The asynchronous engine interface of the CUDA Chunker (candidates_range_async,
+    size_bound_state_dev: counts and entry/exit states in tensors, outputs into caller buffers),
+    backed by the oracle on CPU tensors, so the CPU tests run chunk_sharded's device-style path
+    (no host values between the chain's rounds) too."""
+
+    def candidates_range_async(self, x, halo, start, total_len, out, n_out):
+        c = self.candidates_range(x, halo, start, total_len)
+        n_out[0] = c.numel()
+        m = min(c.numel(), out.numel())
+        out[:m] = c[:m]
+
+    def size_bound_state_dev(self, cands, n_cand, end, fin, state_in, out, n_out, state_out):
+        n = min(int(n_cand[0]), cands.numel())
+        cuts, s2, h2 = self.size_bound_state(cands[:n], end, fin, int(state_in[0]), bool(state_in[1]))
+        n_out[0] = cuts.numel()
+        m = min(cuts.numel(), out.numel())
+        out[:m] = cuts[:m]
+        state_out[0] = s2
+        state_out[1] = int(h2)
+
+
 def _free_port():
     s = socket.socket()
     s.bind(("127.0.0.1", 0))
@@ -53,7 +76,7 @@ def _free_port():
     return p
 
 
-def _worker(rank, world, port, n, seed, params, q, mode="chain"):
+def _worker(rank, world, port, n, seed, params, q, mode="chain", asyn=False):
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
     dist.init_process_group("gloo", rank=rank, world_size=world)
@@ -67,8 +90,8 @@ def _worker(rank, world, port, n, seed, params, q, mode="chain"):
         own = torch.from_numpy(data[start:end].copy())
         x2 = sd.exchange_halo(own, start, params.window)            # C1 over the process group
         assert np.array_equal(x2.numpy(), x.numpy())
-        eng = OracleEngine(params, data)
-        res = sd.chunk_sharded(x, halo, start, n, eng, mode=mode)
+        eng = (OracleAsyncEngine if asyn else OracleEngine)(params, data)
+        res = sd.chunk_sharded(x, halo, start, n, eng, mode=mode, cap=64 if asyn else None)
         allc = sd.gather_all(res).numpy()
         q.put((rank, res.base, res.total, res.local.numpy().tolist(), allc.tolist(),
                None if res.cuts is None else res.cuts.numpy().tolist(), res.cut_base, res.rounds))
@@ -76,11 +99,11 @@ def _worker(rank, world, port, n, seed, params, q, mode="chain"):
         dist.destroy_process_group()
 
 
-def _run(world, n, seed, params, mode="chain"):
+def _run(world, n, seed, params, mode="chain", asyn=False):
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    procs = [ctx.Process(target=_worker, args=(r, world, port, n, seed, params, q, mode)) for r in range(world)]
+    procs = [ctx.Process(target=_worker, args=(r, world, port, n, seed, params, q, mode, asyn)) for r in range(world)]
     for p in procs:
         p.start()
     out = [q.get(timeout=300) for _ in range(world)]
@@ -106,13 +129,29 @@ def test_sharded_unbounded_matches_whole_stream(world):
     assert cat == exp
 
 
-@pytest.mark.parametrize("world,mode", [(2, "gather"), (2, "chain"), (3, "chain")])
-def test_sharded_bounded_global_size_rule(world, mode):
+@pytest.mark.parametrize("world", [2, 3])
+def test_sharded_unbounded_async_engine_overflow_redo(world):
+    """The asynchronous path with a deliberately small candidate buffer (64 entries): the counts
+    exchanged are the true ones, and reading `local` redoes the overflowed shard exactly."""
+    n = (1 << 20) + 12345
+    params = oracle.Params(divisor=1024)
+    exp = oracle.candidates(synthgen.random_bytes(7, n), params).astype(np.int64).tolist()
+    out = _run(world, n, 7, params, asyn=True)
+    cat = []
+    for rank, base, total, local, allc, cuts, cut_base, rounds in out:
+        assert base == len(cat) and total == len(exp)
+        cat += local
+    assert cat == exp
+
+
+@pytest.mark.parametrize("world,mode,asyn", [(2, "gather", False), (2, "chain", False), (3, "chain", False),
+                                             (2, "chain", True), (3, "chain", True)])
+def test_sharded_bounded_global_size_rule(world, mode, asyn):
     n = (1 << 20) + 999
     params = oracle.Params(divisor=512, min_size=128, max_size=4096)
     data = synthgen.random_bytes(9, n)
     exp = oracle.chunk(data, params).astype(np.int64).tolist()
-    out = _run(world, n, 9, params, mode)
+    out = _run(world, n, 9, params, mode, asyn)
     if mode == "gather":
         for rank, base, total, local, allc, cuts, cut_base, rounds in out:
             assert cuts == exp

@@ -104,3 +104,26 @@ def test_bounded_chain_phase_locked_needs_more_rounds():
         assert o["cut_base"] == len(cat)
         cat += o["cuts"]
     assert cat == exp
+
+
+def test_bench_strong_scaling_mode_two_ranks():
+    """bench.py's N > 1 mode (configs[3] strong scaling) end to end with 2 ranks on one GPU
+    (gloo, a 64 MiB stream instead of 64 GiB): one JSON line from rank 0 whose total candidate
+    count equals the oracle's on that stream and whose t1 run (the whole stream on rank 0)
+    finds the same count."""
+    import json
+    import subprocess
+    import sys
+    n = 64 << 20
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = dict(os.environ, SHRED_BENCH_BACKEND="gloo", SHRED_BENCH_DEVICE="0", SHRED_BENCH_STREAM=str(n))
+    r = subprocess.run([sys.executable, "-m", "torch.distributed.run", "--nnodes=1", "--nproc-per-node", "2",
+                        "--master-addr", "127.0.0.1", "--master-port", str(_free_port()),
+                        os.path.join(root, "bench.py"), "--gpus", "2", "--steps", "3", "--warmup", "3",
+                        "--no-e2e"], capture_output=True, text=True, env=env, cwd=root, timeout=600)
+    assert r.returncode == 0, r.stderr[-2000:]
+    line = json.loads([ln for ln in r.stdout.splitlines() if ln.startswith("{")][-1])
+    exp = oracle.candidates(synthgen.random_bytes_fast(5, n), oracle.Params()).size
+    assert line["n_gpus"] == 2 and line["scaling"] == "strong"
+    assert line["candidates_total"] == exp and line["t1_candidates"] == exp
+    assert line["value"] > 0 and line["gpu_launches"] > 0
