@@ -112,22 +112,32 @@ __device__ __forceinline__ void sha256_block(const uint8_t *__restrict__ in, uin
         }
         return;
     }
+    // a padded tail block: the message words by the same aligned loads (only words that start
+    // inside the buffer are read), the bytes at or past L replaced by the padding: 0x80 at byte
+    // L, zeros, the 64-bit bit length in the last block's words 14-15 (FIPS 180-4 §5.1.1).
+    // Round 1 built these blocks a byte at a time with one dependent global load per byte.
     const uint64_t nblk = (L + 9 + 63) / 64;          // blocks of the padded message
-    const uint64_t lenpos = nblk * 64 - 8;            // where the 64-bit bit length starts
-    const uint64_t bits = L * 8;
-#pragma unroll 1
+    const int64_t valid = (int64_t)L - (int64_t)m0;   // message bytes in this block (may be <= 0)
+    const uint32_t sh = (uint32_t)(pa & 3) * 8;
+    const uint32_t *src = reinterpret_cast<const uint32_t *>(wa);
+    uint32_t prev = (valid > 0 && wa < lim) ? __ldg(src) : 0u;
+#pragma unroll
     for (int k = 0; k < 16; ++k) {
-        uint32_t v = 0;
-        for (int q = 0; q < 4; ++q) {
-            const uint64_t m = m0 + 4 * k + q;
-            uint32_t byte;
-            if (m < L) byte = in[a + m];
-            else if (m == L) byte = 0x80u;
-            else if (m >= lenpos) byte = (uint32_t)(bits >> (8 * (7 - (m - lenpos)))) & 0xFFu;
-            else byte = 0;
-            v = (v << 8) | byte;
+        const uintptr_t na = wa + 4u * (uint32_t)(k + 1);
+        const uint32_t nxt = (valid > 4 * k && na < lim) ? __ldg(src + k + 1) : 0u;
+        uint32_t be = __byte_perm(__funnelshift_r(prev, nxt, sh), 0, 0x0123);   // big-endian word
+        prev = nxt;
+        const int64_t nv = valid - 4 * k;                                        // message bytes in it
+        if (nv < 4) {
+            be = nv <= 0 ? 0u : (be & (0xFFFFFFFFu << (32 - 8 * (int)nv)));
+            if (nv >= 0) be |= 0x80u << (24 - 8 * (int)nv);                      // the 0x80 byte
         }
-        W[k] = v;
+        W[k] = be;
+    }
+    if (blk + 1 == nblk) {
+        const uint64_t bits = L * 8;
+        W[14] = (uint32_t)(bits >> 32);
+        W[15] = (uint32_t)bits;
     }
 }
 
@@ -274,6 +284,173 @@ k_hash_chunks(HashJobs Hj, const uint32_t *__restrict__ order, unsigned long lon
             sha256_store(J.digests, chunk, H);
         }
         __syncwarp();
+    }
+}
+
+// ---- warp-specialised hashing (one buffer: the longest chunks' chains set the time).  A CTA
+// holds HWS_PAIRS pairs of warps.  The schedule warp of a pair takes 32 length-sorted chunks from
+// the queue, loads each lane's message blocks and expands them to the 64-word schedule W[0..63]
+// (sigma0/sigma1: ~8 ALU ops per round for 48 of the 64 rounds) into a shared ring; the
+// compress warp runs only the 64 rounds (S0, S1, Ch, Maj: ~10 ALU ops per round, W read by one
+// LDS).  The two warps of a pair sit on different SM sub-partitions (compress warp p on SMSP p,
+// its schedule warp on SMSP p+1 mod 4), so once only the longest chunks are left their chain
+// runs on one sub-partition's ALU with the schedule work on another's.  mbarriers per pair:
+// full/free per W slot, info_full/info_free for the batch description.
+constexpr int HWS_PAIRS = 4;
+constexpr int HWS_THREADS = 64 * HWS_PAIRS;
+#ifndef SHRED_HWS_SLOTS
+#define SHRED_HWS_SLOTS 4
+#endif
+constexpr int HWS_SLOTS = SHRED_HWS_SLOTS;   // W ring depth (blocks the schedule warp may run ahead)
+struct HwsPair {
+    unsigned long long bar[2 * HWS_SLOTS + 2];   // full[slots], free[slots], info_full, info_free
+    uint64_t dig[32];                       // per lane: digest destination (0 = no chunk)
+    uint32_t nblk[32];                      // per lane: blocks of the padded message
+    uint32_t nmax;                          // the batch's longest; 0xFFFFFFFF = no more work
+};
+constexpr size_t HWS_RING = (size_t)HWS_SLOTS * 64 * 32 * 4;   // bytes of W ring per pair (slots x 64 words x 32 lanes)
+constexpr size_t HWS_SMEM = HWS_PAIRS * (HWS_RING + sizeof(HwsPair)) + 128;
+
+__global__ void __launch_bounds__(HWS_THREADS, 1)
+k_hash_chunks_ws(HashJobs Hj, const uint32_t *__restrict__ order, unsigned long long *queue, uint32_t one) {
+    pdl_entry();
+    extern __shared__ __align__(128) uint8_t hws_smem[];
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const bool comp = warp < HWS_PAIRS;
+    const int pair = comp ? warp : (warp - HWS_PAIRS + HWS_PAIRS - 1) % HWS_PAIRS;
+    uint32_t *ring = reinterpret_cast<uint32_t *>(hws_smem + pair * HWS_RING);
+    HwsPair &P = reinterpret_cast<HwsPair *>(hws_smem + HWS_PAIRS * HWS_RING)[pair];
+    const uint32_t bfull = smem_u32(&P.bar[0]), bfree = smem_u32(&P.bar[HWS_SLOTS]);
+    const uint32_t binfo_full = smem_u32(&P.bar[2 * HWS_SLOTS]), binfo_free = smem_u32(&P.bar[2 * HWS_SLOTS + 1]);
+    if (comp && lane == 0) {
+        for (int k = 0; k < 2 * HWS_SLOTS + 2; ++k) mbar_init(smem_u32(&P.bar[k]), 1);
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    }
+    __syncthreads();
+    const uint64_t nc = queue[1];
+    uint32_t gb = 0;                         // blocks passed through the ring (phase counter)
+    if (!comp) {                             // ---- schedule warp
+        uint32_t W[16];
+        for (uint32_t it = 0;; ++it) {
+            if (it > 0) mbar_wait(binfo_free, (it - 1) & 1u);
+            unsigned long long base = 0;
+            if (lane == 0) base = atomicAdd(queue, 32ull);
+            base = __shfl_sync(0xffffffffu, base, 0);
+            const uint64_t j = base + (uint64_t)lane;
+            // job fields copied to registers (a pointer into the kernel parameters would force a
+            // stack copy of them)
+            const uint8_t *jin = nullptr;
+            uint64_t jlen = 0, a = 0, L = 0, chunk = 0, dig = 0;
+            uint32_t nb = 0;
+            if (base < nc && j < nc) {
+                int jb;
+                hash_locate(Hj, order[j], jb, chunk);
+                const HashJob &J = Hj.job[jb];
+                jin = J.in; jlen = J.len;
+                uint64_t b;
+                chunk_bounds(J.cuts, *J.n_cuts, J.len, chunk, a, b);
+                L = b - a;
+                nb = (uint32_t)((L + 9 + 63) / 64);
+                dig = reinterpret_cast<uint64_t>(J.digests + chunk * 32);
+            }
+            uint32_t mx = nb;
+#pragma unroll
+            for (int d = 16; d; d >>= 1) mx = max(mx, __shfl_xor_sync(0xffffffffu, mx, d));
+            P.nblk[lane] = nb;
+            P.dig[lane] = dig;
+            if (lane == 0) P.nmax = base < nc ? mx : 0xFFFFFFFFu;
+            __syncwarp();
+            if (lane == 0) mbar_arrive(binfo_full);
+            if (base >= nc) break;
+            // full blocks by 17 aligned word loads issued one block ahead (their latency hides
+            // behind the previous block's expansion); the padded tail blocks by the byte path
+            const uintptr_t pa = reinterpret_cast<uintptr_t>(jin) + a;
+            const uintptr_t lim = (reinterpret_cast<uintptr_t>(jin) + jlen + 3) & ~(uintptr_t)3;
+            const uint32_t sh = (uint32_t)(pa & 3) * 8;
+            const uint32_t *src0 = reinterpret_cast<const uint32_t *>(pa & ~(uintptr_t)3);
+            uint32_t nfull = (uint32_t)(L / 64);
+            if (nfull && (pa & ~(uintptr_t)3) + 64ull * nfull + 4 > lim) --nfull;
+            uint32_t Rw[17];
+            if (nfull) {
+#pragma unroll
+                for (int k = 0; k < 17; ++k) Rw[k] = __ldg(src0 + k);
+            }
+            for (uint32_t blk = 0; blk < mx; ++blk, ++gb) {
+                const uint32_t slot = gb % HWS_SLOTS;
+                if (gb >= HWS_SLOTS) mbar_wait(bfree + 8 * slot, ((gb / HWS_SLOTS) - 1) & 1u);
+                if (blk < nb) {
+                    if (blk < nfull) {
+#pragma unroll
+                        for (int k = 0; k < 16; ++k) W[k] = __byte_perm(__funnelshift_r(Rw[k], Rw[k + 1], sh), 0, 0x0123);
+                        if (blk + 1 < nfull) {
+                            const uint32_t *nx = src0 + 16 * (blk + 1);
+#pragma unroll
+                            for (int k = 0; k < 17; ++k) Rw[k] = __ldg(nx + k);
+                        }
+                    } else {
+                        sha256_block(jin, jlen, a, L, blk, W);
+                    }
+                    uint32_t *dst = ring + slot * (64 * 32) + lane;
+#pragma unroll
+                    for (int t = 0; t < 64; ++t) {
+                        uint32_t w;
+                        if (t < 16) {
+                            w = W[t];
+                        } else {
+                            const uint32_t w15 = W[(t - 15) & 15], w2 = W[(t - 2) & 15];
+                            const uint32_t s0 = rotr(w15, 7) ^ rotr(w15, 18) ^ (w15 >> 3);
+                            const uint32_t s1 = rotr(w2, 17) ^ rotr(w2, 19) ^ (w2 >> 10);
+                            w = W[t & 15] = s1 + s0 + W[t & 15] + W[(t - 7) & 15];
+                        }
+                        dst[t * 32] = w;
+                    }
+                }
+                __syncwarp();
+                if (lane == 0) mbar_arrive(bfull + 8 * slot);
+            }
+        }
+        return;
+    }
+    // ---- compress warp
+    for (uint32_t it = 0;; ++it) {
+        mbar_wait(binfo_full, it & 1u);
+        const uint32_t mx = P.nmax, nb = P.nblk[lane];
+        uint8_t *dg = reinterpret_cast<uint8_t *>(P.dig[lane]);
+        __syncwarp();
+        if (mx == 0xFFFFFFFFu) break;
+        uint32_t H[8];
+        sha256_init(H);
+        for (uint32_t blk = 0; blk < mx; ++blk, ++gb) {
+            const uint32_t slot = gb % HWS_SLOTS;
+            mbar_wait(bfull + 8 * slot, (gb / HWS_SLOTS) & 1u);
+            if (blk < nb) {
+                const uint32_t *src = ring + slot * (64 * 32) + lane;
+                uint32_t a = H[0], b = H[1], c = H[2], d = H[3], e = H[4], f = H[5], g = H[6], h = H[7];
+#pragma unroll
+                for (int t = 0; t < 64; ++t) {
+                    // The chain e -> e' is S1 (3 rotates + LOP3) then one IADD3: the terms that do
+                    // not depend on this round's e or a (h + K + w, and d + h + K + w) are
+                    // IMADs off the chain.  This warp runs alone on its sub-partition once only
+                    // the longest chunks remain, so latency, not ALU throughput, sets its speed
+                    // (the all-IMAD additions of k_hash_chunks: ~2.3 K cycles per block here).
+                    const uint32_t w = src[t * 32];
+                    const uint32_t hkw = w * one + (h * one + sha_k(t));
+                    const uint32_t dhkw = d * one + hkw;
+                    const uint32_t S1 = rotr(e, 6) ^ rotr(e, 11) ^ rotr(e, 25);
+                    const uint32_t S0 = rotr(a, 2) ^ rotr(a, 13) ^ rotr(a, 22);
+                    const uint32_t ch = (e & f) ^ (~e & g);
+                    const uint32_t mj = (a & b) ^ (a & c) ^ (b & c);
+                    const uint32_t t1 = hkw + S1 + ch;
+                    h = g; g = f; f = e; e = dhkw + S1 + ch; d = c; c = b; b = a; a = t1 + S0 + mj;
+                }
+                H[0] += a; H[1] += b; H[2] += c; H[3] += d; H[4] += e; H[5] += f; H[6] += g; H[7] += h;
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(bfree + 8 * slot);
+        }
+        if (dg) sha256_store(dg, 0, H);
+        __syncwarp();
+        if (lane == 0) mbar_arrive(binfo_free);
     }
 }
 

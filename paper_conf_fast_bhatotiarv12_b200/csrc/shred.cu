@@ -18,6 +18,9 @@
 // (profiles/r02_hash_ab.txt).  Its launch latency is negligible against milliseconds of hashing.
 #define SHRED_HASH_NOPDL 1
 #endif
+#ifndef SHRED_HASH_WS
+#define SHRED_HASH_WS 1   // one buffer: k_hash_chunks_ws (0: k_hash_chunks, A/B)
+#endif
 #ifndef SHRED_HASH_CTAS_PER_SM
 #define SHRED_HASH_CTAS_PER_SM 1
 #endif
@@ -798,7 +801,9 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
         }
     }
     if (cudaFuncSetAttribute(sb_dense, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                             (int)(SBD_WIN / 8)) != cudaSuccess)
+                             (int)(SBD_WIN / 8)) != cudaSuccess ||
+        cudaFuncSetAttribute(k_hash_chunks_ws, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             (int)HWS_SMEM) != cudaSuccess)
         return bail(SHRED_ECUDA);
     if (cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking) != cudaSuccess ||
         cudaEventCreateWithFlags(&ctx->ev_done, cudaEventDisableTiming) != cudaSuccess)
@@ -1114,11 +1119,16 @@ int shred_hash_chunks_batch(shred_ctx *ctx, const shred_hash_job *jobs, int njob
         // sub-partition); two for a batch, whose work hides the long chains anyway
         // (profiles/r02_hash_ab.txt: 3 x 1 GiB 548 -> 627 GB/s, one buffer 290 -> 242 GB/s)
         const unsigned hctas = (unsigned)(ctx->sm_count * SHRED_HASH_CTAS_PER_SM * (H.n > 1 ? 2 : 1));
+        if (SHRED_HASH_WS && H.n == 1) {
+            // one buffer: the warp-specialised kernel (schedule and rounds on two SM sub-partitions)
+            k_hash_chunks_ws<<<(unsigned)ctx->sm_count, HWS_THREADS, HWS_SMEM, st>>>(H, ctx->d_order, ctx->d_queue, 1u);
+        } else {
 #if SHRED_HASH_NOPDL
-        k_hash_chunks<<<hctas, SHRED_HASH_THREADS, 0, st>>>(H, ctx->d_order, ctx->d_queue, 1u);
+            k_hash_chunks<<<hctas, SHRED_HASH_THREADS, 0, st>>>(H, ctx->d_order, ctx->d_queue, 1u);
 #else
-        PDL(k_hash_chunks, hctas, SHRED_HASH_THREADS, 0, st, H, ctx->d_order, ctx->d_queue, 1u);
+            PDL(k_hash_chunks, hctas, SHRED_HASH_THREADS, 0, st, H, ctx->d_order, ctx->d_queue, 1u);
 #endif
+        }
         LAUNCHED("k_hash_chunks");
     }
     return SHRED_OK;
