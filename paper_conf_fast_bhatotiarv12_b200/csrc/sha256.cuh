@@ -296,7 +296,10 @@ k_hash_chunks(HashJobs Hj, const uint32_t *__restrict__ order, unsigned long lon
 // its schedule warp on SMSP p+1 mod 4), so once only the longest chunks are left their chain
 // runs on one sub-partition's ALU with the schedule work on another's.  mbarriers per pair:
 // full/free per W slot, info_full/info_free for the batch description.
-constexpr int HWS_PAIRS = 4;
+#ifndef SHRED_HWS_PAIRS
+#define SHRED_HWS_PAIRS 4
+#endif
+constexpr int HWS_PAIRS = SHRED_HWS_PAIRS;
 constexpr int HWS_THREADS = 64 * HWS_PAIRS;
 #ifndef SHRED_HWS_SLOTS
 #define SHRED_HWS_SLOTS 4

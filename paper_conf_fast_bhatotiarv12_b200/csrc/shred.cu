@@ -21,6 +21,9 @@
 #ifndef SHRED_HASH_WS
 #define SHRED_HASH_WS 1   // one buffer: k_hash_chunks_ws (0: k_hash_chunks, A/B)
 #endif
+#ifndef SHRED_HASH_WS_BATCH
+#define SHRED_HASH_WS_BATCH 1   // batches too (0: k_hash_chunks, 2 CTAs per SM, A/B)
+#endif
 #ifndef SHRED_HASH_CTAS_PER_SM
 #define SHRED_HASH_CTAS_PER_SM 1
 #endif
@@ -1119,7 +1122,7 @@ int shred_hash_chunks_batch(shred_ctx *ctx, const shred_hash_job *jobs, int njob
         // sub-partition); two for a batch, whose work hides the long chains anyway
         // (profiles/r02_hash_ab.txt: 3 x 1 GiB 548 -> 627 GB/s, one buffer 290 -> 242 GB/s)
         const unsigned hctas = (unsigned)(ctx->sm_count * SHRED_HASH_CTAS_PER_SM * (H.n > 1 ? 2 : 1));
-        if (SHRED_HASH_WS && H.n == 1) {
+        if (SHRED_HASH_WS && (H.n == 1 || SHRED_HASH_WS_BATCH)) {
             // one buffer: the warp-specialised kernel (schedule and rounds on two SM sub-partitions)
             k_hash_chunks_ws<<<(unsigned)ctx->sm_count, HWS_THREADS, HWS_SMEM, st>>>(H, ctx->d_order, ctx->d_queue, 1u);
         } else {
