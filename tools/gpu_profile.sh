@@ -21,3 +21,7 @@ if [ "$3" == "k32" ]; then
   ncu --set full --clock-control none --import-source on -k regex:k1_bulk -s 3 -c 1 -o gpurun_out/prof_k1k32_$TAG \
       python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu --no-extra --variant k32 > /dev/null 2>&1
 fi
+# f2: the batched SHA-256 launch (3 x 1 GiB, the bench's hash_sha256 value), same summary tool
+ncu --set full --clock-control none --import-source on -k regex:k_hash_chunks -s 1 -c 1 -o gpurun_out/prof_hash_$TAG \
+    python tools/hash_once.py > gpurun_out/ncu_hash_$TAG.log 2>&1
+python tools/ncu_summary.py gpurun_out/prof_hash_$TAG.ncu-rep > gpurun_out/hash_ncu_full_$TAG.txt 2>&1
