@@ -120,6 +120,10 @@ class ClockSampler:
 
     def __enter__(self):
         if self.ok:
+            # the timed region can be ~20 ms: with the default 5 ms GIL switch interval the
+            # sampler thread got as few as 1 sample in it, so switch threads every 0.1 ms meanwhile
+            self._swi = sys.getswitchinterval()
+            sys.setswitchinterval(1e-4)
             self.t = threading.Thread(target=self._run, daemon=True)
             self.t.start()
         return self
@@ -128,6 +132,7 @@ class ClockSampler:
         if self.ok:
             self._stop.set()
             self.t.join()
+            sys.setswitchinterval(self._swi)
 
     def result(self):
         if not self.ok or not self.samples:
