@@ -311,6 +311,20 @@ struct HwsPair {
     uint32_t nblk[32];                      // per lane: blocks of the padded message
     uint32_t nmax;                          // the batch's longest; 0xFFFFFFFF = no more work
 };
+// Every lane arrives on the pair's mbarriers (count 32), so each lane's own shared-memory writes
+// (W words, batch fields) are released by its own arrive and acquired by the waiting warp: the
+// ordering needs no argument about __syncwarp cumulativity, and compute-sanitizer racecheck
+// models it (a __syncwarp + one elected arrive reported 200 false hazards).
+#ifndef SHRED_HWS_ALL_ARRIVE
+#define SHRED_HWS_ALL_ARRIVE 1
+#endif
+#if SHRED_HWS_ALL_ARRIVE
+constexpr uint32_t HWS_ARRIVALS = 32;
+#define HWS_ARRIVE(bar) mbar_arrive(bar)
+#else
+constexpr uint32_t HWS_ARRIVALS = 1;
+#define HWS_ARRIVE(bar) do { __syncwarp(); if (lane == 0) mbar_arrive(bar); } while (0)
+#endif
 constexpr size_t HWS_RING = (size_t)HWS_SLOTS * 64 * 32 * 4;   // bytes of W ring per pair (slots x 64 words x 32 lanes)
 constexpr size_t HWS_SMEM = HWS_PAIRS * (HWS_RING + sizeof(HwsPair)) + 128;
 
@@ -326,7 +340,7 @@ k_hash_chunks_ws(HashJobs Hj, const uint32_t *__restrict__ order, unsigned long 
     const uint32_t bfull = smem_u32(&P.bar[0]), bfree = smem_u32(&P.bar[HWS_SLOTS]);
     const uint32_t binfo_full = smem_u32(&P.bar[2 * HWS_SLOTS]), binfo_free = smem_u32(&P.bar[2 * HWS_SLOTS + 1]);
     if (comp && lane == 0) {
-        for (int k = 0; k < 2 * HWS_SLOTS + 2; ++k) mbar_init(smem_u32(&P.bar[k]), 1);
+        for (int k = 0; k < 2 * HWS_SLOTS + 2; ++k) mbar_init(smem_u32(&P.bar[k]), HWS_ARRIVALS);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
     }
     __syncthreads();
@@ -362,11 +376,10 @@ k_hash_chunks_ws(HashJobs Hj, const uint32_t *__restrict__ order, unsigned long 
             P.nblk[lane] = nb;
             P.dig[lane] = dig;
             if (lane == 0) P.nmax = base < nc ? mx : 0xFFFFFFFFu;
-            __syncwarp();
-            if (lane == 0) mbar_arrive(binfo_full);
+            HWS_ARRIVE(binfo_full);
             if (base >= nc) break;
             // full blocks by 17 aligned word loads issued one block ahead (their latency hides
-            // behind the previous block's expansion); the padded tail blocks by the byte path
+            // behind the previous block's expansion); the padded tail blocks by sha256_block
             const uintptr_t pa = reinterpret_cast<uintptr_t>(jin) + a;
             const uintptr_t lim = (reinterpret_cast<uintptr_t>(jin) + jlen + 3) & ~(uintptr_t)3;
             const uint32_t sh = (uint32_t)(pa & 3) * 8;
@@ -408,8 +421,7 @@ k_hash_chunks_ws(HashJobs Hj, const uint32_t *__restrict__ order, unsigned long 
                         dst[t * 32] = w;
                     }
                 }
-                __syncwarp();
-                if (lane == 0) mbar_arrive(bfull + 8 * slot);
+                HWS_ARRIVE(bfull + 8 * slot);
             }
         }
         return;
@@ -448,12 +460,10 @@ k_hash_chunks_ws(HashJobs Hj, const uint32_t *__restrict__ order, unsigned long 
                 }
                 H[0] += a; H[1] += b; H[2] += c; H[3] += d; H[4] += e; H[5] += f; H[6] += g; H[7] += h;
             }
-            __syncwarp();
-            if (lane == 0) mbar_arrive(bfree + 8 * slot);
+            HWS_ARRIVE(bfree + 8 * slot);
         }
         if (dg) sha256_store(dg, 0, H);
-        __syncwarp();
-        if (lane == 0) mbar_arrive(binfo_free);
+        HWS_ARRIVE(binfo_free);
     }
 }
 

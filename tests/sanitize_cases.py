@@ -59,11 +59,13 @@ def main():
     n2 = torch.tensor([c2.numel()], dtype=torch.int64, device="cuda")
     d1 = torch.empty((cuts.numel() + 1) * 32, dtype=torch.uint8, device="cuda")
     d2 = torch.empty((c2.numel() + 1) * 32, dtype=torch.uint8, device="cuda")
+    dig2 = chh.hash_chunks(x2, c2).cpu().numpy()                  # one unaligned buffer (ws kernel)
     chh.hash_chunks_batch_async([(x, cuts, n1, d1), (x2, c2, n2, d2)])
     torch.cuda.synchronize()
     assert np.array_equal(d1.view(-1, 32).cpu().numpy(), dig)
     assert np.array_equal(d2.view(-1, 32).cpu().numpy(),
                           oracle.chunk_digests(data[1:200001], c2.cpu().numpy().astype(np.uint64)))
+    assert np.array_equal(d2.view(-1, 32).cpu().numpy(), dig2)
     chh.index_reset(1 << 12)
     n_c = torch.tensor([cuts.numel()], dtype=torch.int64, device="cuda")
     chh.index_insert_async(torch.from_numpy(dig.reshape(-1)).cuda(), cuts, n_c, data.size)

@@ -141,3 +141,26 @@ def test_index_dedup_across_snapshots_vs_oracle(pkg):
         uniq_batch = {bytes(x) for x in d}
         if len(uniq_batch) == len(d):                             # no duplicates inside the batch
             assert np.array_equal(got_flags, exp_flags)
+
+
+@pytest.mark.parametrize("shift", [0, 1, 3])
+@pytest.mark.parametrize("last", [1, 55, 56, 63, 64, 65, 119, 128])
+def test_last_chunk_at_buffer_end(pkg, shift, last):
+    """The padding blocks of the chunk that ends at the buffer's last byte: the word loads stop at
+    the last word that starts inside the buffer, whatever the alignment (one buffer and batched)."""
+    lens = [100, 64, 7, last]
+    cuts = np.cumsum(lens)[:-1]
+    n = int(np.sum(lens))
+    data = synthgen.random_bytes(11 + last, n + shift)
+    base = torch.from_numpy(data).cuda()
+    x = base[shift:]
+    ch = pkg.Chunker(pkg.Params())
+    c = torch.from_numpy(cuts.astype(np.int64)).cuda()
+    exp = oracle.chunk_digests(data[shift:], cuts)
+    assert np.array_equal(ch.hash_chunks(x, c).cpu().numpy(), exp)
+    nc = torch.tensor([c.numel()], dtype=torch.int64, device="cuda")
+    d = [torch.empty((c.numel() + 1) * 32, dtype=torch.uint8, device="cuda") for _ in range(2)]
+    ch.hash_chunks_batch_async([(x, c, nc, d[0]), (x, c, nc, d[1])])
+    torch.cuda.synchronize()
+    for di in d:
+        assert np.array_equal(di.view(-1, 32).cpu().numpy(), exp)
