@@ -325,6 +325,9 @@ constexpr uint32_t HWS_ARRIVALS = 32;
 constexpr uint32_t HWS_ARRIVALS = 1;
 #define HWS_ARRIVE(bar) do { __syncwarp(); if (lane == 0) mbar_arrive(bar); } while (0)
 #endif
+#ifndef SHRED_HWS_ADD
+#define SHRED_HWS_ADD 0   // compress-round additions on the FMA pipe: 0 none, 1 a's, 2 a's and t1's (A/B)
+#endif
 constexpr size_t HWS_RING = (size_t)HWS_SLOTS * 64 * 32 * 4;   // bytes of W ring per pair (slots x 64 words x 32 lanes)
 constexpr size_t HWS_SMEM = HWS_PAIRS * (HWS_RING + sizeof(HwsPair)) + 128;
 
@@ -455,8 +458,18 @@ k_hash_chunks_ws(HashJobs Hj, const uint32_t *__restrict__ order, unsigned long 
                     const uint32_t S0 = rotr(a, 2) ^ rotr(a, 13) ^ rotr(a, 22);
                     const uint32_t ch = (e & f) ^ (~e & g);
                     const uint32_t mj = (a & b) ^ (a & c) ^ (b & c);
+#if SHRED_HWS_ADD == 0
                     const uint32_t t1 = hkw + S1 + ch;
                     h = g; g = f; f = e; e = dhkw + S1 + ch; d = c; c = b; b = a; a = t1 + S0 + mj;
+#elif SHRED_HWS_ADD == 1
+                    const uint32_t t1 = hkw + S1 + ch;
+                    h = g; g = f; f = e; e = dhkw + S1 + ch; d = c; c = b; b = a;
+                    a = mj * one + (S0 * one + t1);
+#else
+                    const uint32_t t1 = S1 * one + (ch * one + hkw);
+                    h = g; g = f; f = e; e = dhkw + S1 + ch; d = c; c = b; b = a;
+                    a = mj * one + (S0 * one + t1);
+#endif
                 }
                 H[0] += a; H[1] += b; H[2] += c; H[3] += d; H[4] += e; H[5] += f; H[6] += g; H[7] += h;
             }
