@@ -162,34 +162,65 @@ def cpu_model() -> str:
     return "unknown"
 
 
-def cpu_measurements(runs: int = 3, budget_s: float = 4.0) -> dict:
+def oracle_samples(world: int, cores: int):
+    """The bounded sample both arms time the oracle on (so that the main arm's cpu_baseline and
+    the reference arm measure the same thing): slices of n <= 256 MiB, sized to ~2 s of oracle work
+    on this host. N = 1: the configs[1] base file's first n bytes and its edited version
+    (alternating); N > 1: consecutive slices of the configs[3] stream (seed 5)."""
+    import synthgen
+    cal = synthgen.random_bytes_fast(2, 8 << 20)
+    rate, _, _ = oracle_rate(cal, cores)                   # calibration (also warms the tables)
+    n = int(min(256 << 20, max(8 << 20, rate * 1e9 * 2.0)))
+    n -= n % 4096
+    if world == 1:
+        base = synthgen.random_bytes_fast(2, n)
+        ed, _ = synthgen.edited(base, 3, n_edits=max(1, min(100, n // (1 << 20))), min_gap=8192)
+        return n, [base, ed]
+    return n, [synthgen.random_bytes_fast(5, n, 0), synthgen.random_bytes_fast(5, n, n)]
+
+
+def oracle_steps(samples, steps: int, cores: int):
+    """Time `steps` oracle calls over the alternating samples; returns (total bytes, seconds,
+    per-step GB/s)."""
+    import oracle
+    tot, per = 0, []
+    t0 = time.perf_counter()
+    for i in range(steps):
+        s = samples[i % len(samples)]
+        t = time.perf_counter()
+        oracle.candidates(s, oracle.Params(), 2, cores)
+        per.append(s.size / (time.perf_counter() - t) / 1e9)
+        tot += s.size
+    return tot, time.perf_counter() - t0, per
+
+
+def cpu_measurements(runs: int = 3) -> dict:
     """The host-core baselines, measured in a FRESH process with no CUDA context (bench.py
-    --cpu-only, started before the parent touches the GPU): the oracle (R2, all cores) on a
-    bounded prefix of the configs[1] base file, median of `runs`, and the paper's §5.1
-    multithreaded rolling chunker on the whole file.  Round 1 measured the oracle in-process
-    after the CUDA work and got half the rate of the same code in a fresh process."""
+    --cpu-only, started before the parent touches the GPU): the oracle (R2, all cores) on the same
+    bounded sample and with the same timing code as the reference arm (`oracle_samples`,
+    `oracle_steps`; round 1 timed it in-process after the CUDA work at half the rate, and early
+    round 2 on a different sample), and the paper's §5.1 multithreaded rolling chunker
+    on the whole 1 GiB base file."""
     import oracle
     import synthgen
     oracle.build()
     cores = sorted(os.sched_getaffinity(0))
     nc = len(cores)
-    host = synthgen.random_bytes_fast(2, GiB)             # = the device's synth_fill(seed 2)
-    rate, _, _ = oracle_rate(host[: 8 << 20], nc)          # calibration (also warms the tables)
-    n = int(min(host.size, max(16 << 20, rate * 1e9 * budget_s)))
-    n -= n % 4096
-    rates, ncand = [], 0
-    for _ in range(runs):
-        r, dt, ncand = oracle_rate(host[:n], nc)
-        rates.append(r)
-    rate1, dt1, _ = oracle_rate(host[: 8 << 20], 1)
+    n, samples = oracle_samples(1, nc)
+    oracle_steps(samples, 1, nc)                            # warm-up step (as the reference arm's)
+    tot, dt, per = oracle_steps(samples, 2 * runs, nc)
+    rate1, dt1, _ = oracle_rate(samples[0][: 8 << 20], 1)
     out = {"cpu_baseline": {
-        "value": round(float(np.median(rates)), 4), "unit": "GB/s", "cores": nc, "kind": "oracle",
-        "sample": f"first {n / 2**20:.0f} MiB of the configs[1] base file (SplitMix64 seed 2), R2 direct "
-                  f"per-window reduction (48 table lookups/window), {nc} threads, median of {runs} runs "
-                  f"({', '.join(f'{r:.4f}' for r in rates)} GB/s), fresh process without a CUDA context",
-        "runs": [round(r, 4) for r in rates], "affinity": f"cpus {cores[0]}-{cores[-1]} ({nc})",
+        "value": round(tot / dt / 1e9, 4), "unit": "GB/s", "cores": nc, "kind": "oracle",
+        "sample": f"{2 * runs} steps of {n / 2**20:.0f} MiB, alternating the configs[1] base file's first "
+                  f"{n / 2**20:.0f} MiB (SplitMix64 seed 2) and its edited version, R2 direct per-window "
+                  f"reduction (48 table lookups/window), {nc} threads, fresh process without a CUDA "
+                  f"context; the reference arm's sample and timing code",
+        "runs": [round(r, 4) for r in per], "median_step": round(float(np.median(per)), 4),
+        "affinity": f"cpus {cores[0]}-{cores[-1]} ({nc})",
         "value_1core": round(rate1, 4), "sample_1core": f"first 8 MiB, 1 thread, {dt1:.1f} s",
         "cpu_model": cpu_model()}}
+    host = synthgen.random_bytes_fast(2, GiB)             # = the device's synth_fill(seed 2)
     try:
         import cpu_baseline as cb
         cb.build()
@@ -226,27 +257,11 @@ def run_reference(args, rank, world):
     oracle.build()
     cores = len(os.sched_getaffinity(0))
     per_rank = 2 * GiB
-    # each step: a bounded sample of the workload (N = 1: alternating base / edited-version slices
-    # of configs[1]; N > 1: consecutive slices of the configs[3] stream, seed 5)
-    cal = synthgen.random_bytes_fast(2, 8 << 20)
-    rate, _, _ = oracle_rate(cal, cores)
-    n = int(min(256 << 20, max(8 << 20, rate * 1e9 * 2.0)))
-    n -= n % 4096
-    if world == 1:
-        base = synthgen.random_bytes_fast(2, n)
-        ed, _ = synthgen.edited(base, 3, n_edits=max(1, min(100, n // (1 << 20))), min_gap=8192)
-        samples = [base, ed]
-    else:
-        samples = [synthgen.random_bytes_fast(5, n, 0), synthgen.random_bytes_fast(5, n, n)]
-    for i in range(args.warmup):
-        oracle.candidates(samples[i % 2], oracle.Params(), 2, cores)
-    t0 = time.perf_counter()
-    tot = 0
-    for i in range(args.steps):
-        s = samples[i % 2]
-        oracle.candidates(s, oracle.Params(), 2, cores)
-        tot += s.size
-    dt = time.perf_counter() - t0
+    # each step: a bounded sample of the workload (oracle_samples; the main arm's cpu_baseline
+    # times the same sample with the same code)
+    n, samples = oracle_samples(world, cores)
+    oracle_steps(samples, args.warmup, cores)
+    tot, dt, _ = oracle_steps(samples, args.steps, cores)
     v = tot / dt / 1e9
     line = {"metric": METRIC, "value": round(v, 4), "unit": "GB/s", "n_gpus": world, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": round(dt / args.steps * 1e3, 3), "higher_is_better": True,

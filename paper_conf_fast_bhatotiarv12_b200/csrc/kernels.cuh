@@ -603,11 +603,14 @@ template <> struct State<MODE_K32> {
     __device__ __forceinline__ uint32_t low() const { return f; }
     __device__ __forceinline__ uint64_t full() const { return f; }
 };
+#ifndef SHRED_K32B_HI
+#define SHRED_K32B_HI 0   // 1: K32B builds the T index by IMAD.HI + IMAD (fmaheavy) instead of one PRMT (ALU)
+#endif
 template <> struct State<MODE_K32B> {
     uint32_t f = 0;
     __device__ __forceinline__ void set(uint64_t v) { f = (uint32_t)v; }
     template <int K> __device__ __forceinline__ void step(uint32_t in, uint32_t pop, const BulkCtx &c) {
-        step32<K, true>(f, in, pop, c);
+        step32<K, !SHRED_K32B_HI>(f, in, pop, c);
     }
     __device__ __forceinline__ uint32_t low() const { return f; }
     __device__ __forceinline__ uint64_t full() const { return f; }
@@ -623,14 +626,25 @@ enum { MK_EQ = 0, MK_LE = 1, MK_DIV = 2, MK_REM = 3 };
 __device__ __forceinline__ bool is_marker(uint32_t lo, const BulkCtx &c) { return lo * c.tmul == c.rsh; }
 // m | BIT if marker else m: ISETP + predicated LOP3 (the PTX predication survives ptxas).
 // LE: the "mod D <= r" marker set (L249-L251): (f_lo << (32-m)) <= (r << (32-m)).
-// SHRED_MARK_LOP: the low m bits by a LOP3 mask (ALU) instead of the IMAD shift (fmaheavy).
+// SHRED_MARK_LOP 1: the low m bits by a LOP3 mask (ALU) instead of the IMAD shift (fmaheavy).
+// FUSED ('==' only; the u32-state modes): one LOP3 that writes the predicate
+// ((lo ^ r) & (D-1)) != 0 (r < D) and no IMAD: 1 ALU op instead of IMAD (fmaheavy) + ISETP (ALU).
+// Measured (round 2, 1 GiB k1_bulk, profiles/r02_k32_ab.txt): K32T 2,850 -> 2,960 GB/s, K32 (deg 29)
+// 2,602 -> 2,671, K32B 2,778 -> 2,789; the u64-state modes lose 0.6-0.8 % (LSU-bound; IMAD form kept).
+// SHRED_MARK_LOP 2 forces the fused form on every mode, -1 on none (A/B).
 #ifndef SHRED_MARK_LOP
 #define SHRED_MARK_LOP 0
 #endif
-template <uint32_t BIT, int MK>
+template <uint32_t BIT, int MK, bool FUSED = false>
 __device__ __forceinline__ uint32_t or_if_marker(uint32_t m, uint32_t lo, const BulkCtx &c) {
-    const uint32_t x = SHRED_MARK_LOP ? (lo & c.dm32) : lo * c.tmul;
-    const uint32_t y = SHRED_MARK_LOP ? c.r32 : c.rsh;
+    if (MK == MK_EQ && SHRED_MARK_LOP != -1 && (FUSED || SHRED_MARK_LOP == 2)) {
+        asm("{\n .reg .pred p;\n .reg .b32 t;\n lop3.b32 t, %1, %2, %3, 0x28;\n setp.eq.u32 p, t, 0;\n"
+            " @p or.b32 %0, %0, %4;\n}"
+            : "+r"(m) : "r"(lo), "r"(c.r32), "r"(c.dm32), "n"(BIT));
+        return m;
+    }
+    const uint32_t x = SHRED_MARK_LOP == 1 ? (lo & c.dm32) : lo * c.tmul;
+    const uint32_t y = SHRED_MARK_LOP == 1 ? c.r32 : c.rsh;
     if (MK == MK_LE)
         asm("{\n .reg .pred p;\n setp.le.u32 p, %1, %2;\n @p or.b32 %0, %0, %3;\n}"
             : "+r"(m) : "r"(x), "r"(y), "n"(BIT));
@@ -696,7 +710,9 @@ static __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t
           : (MK == MK_REM && (MODE == MODE_K32 || MODE == MODE_K32B || MODE == MODE_K32T))       \
                 ? or_if_rem32<(1u << (4 * J + q))>(m[ch], st[ch].low(), c)                            \
           : (MK == MK_REM) ? or_if_rem<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
-                           : or_if_marker<(1u << (4 * J + q)), MK>(m[ch], st[ch].low(), c);
+                           : or_if_marker<(1u << (4 * J + q)), MK,                                        \
+                                         MODE == MODE_K32T || MODE == MODE_K32 || MODE == MODE_K32B>(  \
+                                 m[ch], st[ch].low(), c);
 #endif
 template <int MODE, int CH, bool TEST, int J, int MK>
 __device__ __forceinline__ void word4xN(State<MODE> (&st)[CH], const uint32_t (&in)[CH],

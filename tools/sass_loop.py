@@ -8,9 +8,9 @@ LSU: LDS/STS/LDG/...).  Static counts: a body executed once per loop iteration.
 import re
 import sys
 
-ALU = ("LOP3", "PRMT", "ISETP", "SEL", "IADD3", "SHF", "LEA", "PLOP3", "FMNMX", "IMNMX", "VIADD",
-       "POPC", "FLO", "BMSK", "SGXT", "LOP", "MOV", "VIMNMX", "R2P", "P2R", "ISCADD")
-FMA = ("IMAD", "FFMA", "FMUL", "FADD", "HFMA2")
+ALU = ("LOP3", "PRMT", "ISETP", "SEL", "IADD3", "SHF", "LEA", "PLOP3", "FMNMX", "IMNMX",
+       "POPC", "FLO", "BMSK", "SGXT", "LOP", "MOV", "VIMNMX", "R2P", "P2R", "ISCADD", "FSETP")
+FMA = ("IMAD", "FFMA", "FMUL", "FADD", "HFMA2", "VIADD")   # VIADD: fmaheavy (tools/pipe_probe.cu)
 LSU = ("LDS", "STS", "LDG", "STG", "LD", "ST", "LDSM", "ATOMS", "SHFL", "LDC")
 
 
