@@ -452,8 +452,8 @@ def main():
     ap.add_argument("--no-extra", action="store_true", help="skip the bounded / k32 side measurements")
     ap.add_argument("--cpu-only", action="store_true", help=argparse.SUPPRESS)   # internal: fresh-process CPU leg
     ap.add_argument("--weak", action="store_true", help="N > 1: round-1 weak scaling (configs[1] per rank)")
-    ap.add_argument("--variant", default="paper", choices=["paper", "k32"],
-                    help="profiling aid: k32 = P 0x104C11DB7 on the main path (not the headline)")
+    ap.add_argument("--variant", default="paper", choices=["paper", "k32", "k32t"],
+                    help="profiling aid: k32 = P 0x104C11DB7, k32t = x^31+x^13+1 on the main path (not the headline)")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
 
@@ -499,7 +499,7 @@ def main():
     edited = torch.from_numpy(ed_np).to(dev)
     per_rank_bytes = int(base.numel() + edited.numel())
 
-    main_params = pkg.Params() if args.variant == "paper" else pkg.Params(poly=0x104C11DB7)
+    main_params = pkg.Params(poly={"paper": pkg.Params().poly, "k32": 0x104C11DB7, "k32t": 0x80002001}[args.variant])
     ch = pkg.Chunker(main_params, device=local)
     cap = GiB // 2048 + 65536
     out0 = torch.empty(cap, dtype=torch.int64, device=dev)

@@ -702,17 +702,36 @@ static __device__ __noinline__ void emit_mask(uint32_t m, uint64_t pos, uint64_t
 }
 
 // One word (4 bytes) of CH interleaved chains; hit bits accumulate into m[ch] (bit 4J+q).
+// PACKM: with two chains per thread the hit bits of both share one register (chain 1 at bits
+// 16..31), so a chunk costs one mask init (SEL) and one "any hit" test for the pair instead of
+// one each per chain (ALU-pipe ops: the u32-state kernels are ALU-bound).
+#ifndef SHRED_PACKM
+#define SHRED_PACKM 1
+#endif
+template <int CH> struct Pack { static constexpr bool on = SHRED_PACKM && CH == 2; };
 #if SHRED_HITMODE == 0
 #define SHRED_MARK(ch, q) m[ch] |= is_marker(st[ch].low(), c) ? (1u << (4 * J + q)) : 0u;
 #else
-#define SHRED_MARK(ch, q)                                                                   \
-    m[ch] = (MK == MK_DIV) ? or_if_div<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
-          : (MK == MK_REM && (MODE == MODE_K32 || MODE == MODE_K32B || MODE == MODE_K32T))       \
-                ? or_if_rem32<(1u << (4 * J + q))>(m[ch], st[ch].low(), c)                            \
-          : (MK == MK_REM) ? or_if_rem<(1u << (4 * J + q))>(m[ch], st[ch].full(), c)          \
-                           : or_if_marker<(1u << (4 * J + q)), MK,                                        \
-                                         MODE == MODE_K32T || MODE == MODE_K32 || MODE == MODE_K32B>(  \
-                                 m[ch], st[ch].low(), c);
+// the hit test of position 4J+Q for every chain, chain index CHI a compile-time constant (the
+// hit bit is an immediate operand of the predicated add)
+template <int MODE, int CH, int J, int Q, int MK, int CHI = 0>
+__device__ __forceinline__ void mark_chains(State<MODE> (&st)[CH], uint32_t (&m)[CH], const BulkCtx &c) {
+    if constexpr (CHI < CH) {
+        constexpr int MI = Pack<CH>::on ? 0 : CHI;
+        constexpr uint32_t BIT = 1u << (4 * J + Q + (Pack<CH>::on ? 16 * CHI : 0));
+        constexpr bool U32 = MODE == MODE_K32 || MODE == MODE_K32B || MODE == MODE_K32T;
+        if constexpr (MK == MK_DIV)
+            m[MI] = or_if_div<BIT>(m[MI], st[CHI].full(), c);
+        else if constexpr (MK == MK_REM && U32)
+            m[MI] = or_if_rem32<BIT>(m[MI], st[CHI].low(), c);
+        else if constexpr (MK == MK_REM)
+            m[MI] = or_if_rem<BIT>(m[MI], st[CHI].full(), c);
+        else
+            m[MI] = or_if_marker<BIT, MK, U32>(m[MI], st[CHI].low(), c);
+        mark_chains<MODE, CH, J, Q, MK, CHI + 1>(st, m, c);
+    }
+}
+#define SHRED_MARK(ch, q) if (ch == 0) mark_chains<MODE, CH, J, q, MK>(st, m, c);
 #endif
 template <int MODE, int CH, bool TEST, int J, int MK>
 __device__ __forceinline__ void word4xN(State<MODE> (&st)[CH], const uint32_t (&in)[CH],
@@ -1030,10 +1049,24 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                 }
                 chunk16xN<MODE, CH, true, MK>(st, d, p, c, m);
 #pragma unroll
-                for (int ch = 0; ch < CH; ++ch) {
-                    R[ch][cq] = D[ch][u];
-                    if (m[ch] && act[ch])
-                        emit_mask(m[ch], pos0[ch] + (uint64_t)(r + qr) * ROUND + 16u * u, J.min_i, J.c_limit, o[ch]);
+                for (int ch = 0; ch < CH; ++ch) R[ch][cq] = D[ch][u];
+                // rows past nrows (TMA zero fill; only in the last CTA) are tested only once a
+                // chunk has a hit (zero windows are markers when r = 0 or '<='): one "any hit"
+                // test per chunk for the pair of chains
+                if (Pack<CH>::on) {
+                    if (m[0]) {
+#pragma unroll
+                        for (int ch = 0; ch < CH; ++ch) {
+                            const uint32_t mc = (m[0] >> (16 * ch)) & 0xFFFFu;
+                            if (mc && act[ch])
+                                emit_mask(mc, pos0[ch] + (uint64_t)(r + qr) * ROUND + 16u * u, J.min_i, J.c_limit, o[ch]);
+                        }
+                    }
+                } else {
+#pragma unroll
+                    for (int ch = 0; ch < CH; ++ch)
+                        if (m[ch] && act[ch])
+                            emit_mask(m[ch], pos0[ch] + (uint64_t)(r + qr) * ROUND + 16u * u, J.min_i, J.c_limit, o[ch]);
                 }
             }
         }
