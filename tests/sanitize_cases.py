@@ -45,6 +45,8 @@ def main():
     check(pkg.Chunker(pkg.Params(poly=0x80002001)), data)                                 # K32T, aligned start (no head)
     check(pkg.Chunker(pkg.Params(poly=0x80002001, window=31, marker=1, magic=3)), data[:300000], 9)    # K32T funnel '<='
     check(pkg.Chunker(pkg.Params()), data[: (1 << 20)])                                 # small shape, 32-B rows
+    check(pkg.Chunker(pkg.Params(poly=0x80002001, magic=0)), data, 2)       # K32T, r = 0: zero-filled rows past nrows are markers
+    check(pkg.Chunker(pkg.Params(poly=0x80002001, marker=1, magic=1)), data[:700001], 1)   # K32T '<=' (packed hit masks)
     check(pkg.Chunker(pkg.Params(divisor=4096, magic=77, marker=1)), data[:500000], 6)   # '<=' lists sized by rate
     # f2 / f3: SHA-256 of every chunk (hashlib oracle) and the dedup index
     chh = pkg.Chunker(pkg.Params())

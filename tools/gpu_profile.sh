@@ -18,8 +18,10 @@ tail -2 gpurun_out/ncu_full_$TAG.log
 python tools/ncu_summary.py gpurun_out/prof_k1_$TAG.ncu-rep > gpurun_out/k1_bulk_ncu_full_$TAG.txt 2>&1
 python tools/ncu_traffic.py gpurun_out/prof_k1_$TAG.ncu-rep profiles/${TAG}_k1_bulk_ncu_full.txt > gpurun_out/k1_traffic_$TAG.json 2>&1
 if [ "$3" == "k32" ]; then
-  ncu --set full --clock-control none --import-source on -k regex:k1_bulk -s 3 -c 1 -o gpurun_out/prof_k1k32_$TAG \
-      python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu --no-extra --variant k32 > /dev/null 2>&1
+  # the k <= 32 kernel on the sparse trinomial x^31+x^13+1 (K32T, bench k32t_variant)
+  ncu --set full --clock-control none --import-source on -k regex:k1_bulk -s 3 -c 1 -o gpurun_out/prof_k1k32t_$TAG \
+      python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu --no-extra --variant k32t > /dev/null 2>&1
+  python tools/ncu_summary.py gpurun_out/prof_k1k32t_$TAG.ncu-rep > gpurun_out/k32t_ncu_full_$TAG.txt 2>&1
 fi
 # f2: the batched SHA-256 launch (3 x 1 GiB, the bench's hash_sha256 value), same summary tool
 ncu --set full --clock-control none --import-source on -k regex:k_hash_chunks -s 1 -c 1 -o gpurun_out/prof_hash_$TAG \
