@@ -739,42 +739,50 @@ def main():
             small = base[: 1 << 20]
             o_s = torch.empty(4096, dtype=torch.int64, device=dev)
             n_s = torch.zeros(1, dtype=torch.int64, device=dev)
-            # warm-up long enough (~10 ms of back-to-back calls) for the SM clock to settle after the
-            # host-side phases above; a short burst can run below the boost clock
-            for _ in range(800):
-                ch.chunk_async(small, o_s, n_s)
-            torch.cuda.synchronize()
-            q0, q1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-            q0.record(stream)
-            for _ in range(1000):
-                ch.chunk_async(small, o_s, n_s)
-            q1.record(stream)
-            torch.cuda.synchronize()
-            us = q0.elapsed_time(q1) * 1e3 / 1000
-            # the same call captured once into a CUDA graph and replayed (no per-call launches)
-            gs = torch.cuda.Stream()
-            gs.wait_stream(stream)
-            with torch.cuda.stream(gs):
-                ch.chunk_async(small, o_s, n_s, stream=gs)
-            torch.cuda.synchronize()
-            cg = torch.cuda.CUDAGraph()
-            with torch.cuda.graph(cg, stream=gs):
-                for _ in range(20):                      # 20 calls per graph: no per-call launch cost
-                    ch.chunk_async(small, o_s, n_s, stream=gs)
-            cg.replay()
-            torch.cuda.synchronize()
-            for _ in range(20):
+
+            def small_latency(chx):
+                # warm-up long enough (~10 ms of back-to-back calls) for the SM clock to settle
+                # after the host-side phases above; a short burst can run below the boost clock
+                for _ in range(800):
+                    chx.chunk_async(small, o_s, n_s)
+                torch.cuda.synchronize()
+                q0, q1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                q0.record(stream)
+                for _ in range(1000):
+                    chx.chunk_async(small, o_s, n_s)
+                q1.record(stream)
+                torch.cuda.synchronize()
+                us = q0.elapsed_time(q1) * 1e3 / 1000
+                # the same call captured once into a CUDA graph and replayed (no per-call launches)
+                gs = torch.cuda.Stream()
+                gs.wait_stream(stream)
+                with torch.cuda.stream(gs):
+                    chx.chunk_async(small, o_s, n_s, stream=gs)
+                torch.cuda.synchronize()
+                cg = torch.cuda.CUDAGraph()
+                with torch.cuda.graph(cg, stream=gs):
+                    for _ in range(20):                  # 20 calls per graph: no per-call launch cost
+                        chx.chunk_async(small, o_s, n_s, stream=gs)
                 cg.replay()
-            q0.record(stream)
-            for _ in range(50):
-                cg.replay()
-            q1.record(stream)
-            torch.cuda.synchronize()
-            us_graph = q0.elapsed_time(q1) * 1e3 / 1000
+                torch.cuda.synchronize()
+                for _ in range(20):
+                    cg.replay()
+                q0.record(stream)
+                for _ in range(50):
+                    cg.replay()
+                q1.record(stream)
+                torch.cuda.synchronize()
+                return us, q0.elapsed_time(q1) * 1e3 / 1000, int(n_s.item())
+
+            us_b, us_graph_b, n_b = small_latency(pkg.Chunker(pkg.Params(min_size=2048, max_size=65536), device=local))
+            us, us_graph, n_small = small_latency(ch)
             line["config1_1mib"] = {"us_per_call": round(us, 2), "us_per_call_in_graph": round(us_graph, 2),
                                     "gbs": round((1 << 20) / (us * 1e-6) / 1e9, 1),
-                                    "candidates": int(n_s.item()),
-                                    "note": "configs[0] size, device-resident, back-to-back calls on one stream"}
+                                    "candidates": n_small,
+                                    "bounded_us_per_call": round(us_b, 2),
+                                    "bounded_us_per_call_in_graph": round(us_graph_b, 2), "bounded_cuts": n_b,
+                                    "note": "configs[0] size, device-resident, back-to-back calls on one stream; "
+                                            "bounded_*: the same call with the size rule on (min 2048 / max 65536)"}
             # f2: SHA-256 of every chunk.  One buffer alone is bound by its longest chunk (a
             # sequential hash on one lane); a batch of buffers shares one length-sorted work
             # list (shred_hash_chunks_batch), so the long chains overlap the other buffers' work.

@@ -1225,6 +1225,14 @@ __global__ void k_stream_reset(Aux *aux) {
     aux->s = 0; aux->held = 0; aux->held_val = 0; aux->dense = 0;
 }
 
+// A piece with no window ends: no candidates (the count the size rule reads, the dense flag and
+// the caller's count if given).
+__global__ void k_no_slots(Aux *aux, uint64_t *n_direct) {
+    pdl_entry();
+    aux->total = 0; aux->ncand = 0; aux->dense = 0;
+    if (n_direct) *n_direct = 0;
+}
+
 __global__ void k_write_u64(uint64_t *p, uint64_t v) {
     pdl_entry();
     *p = v;

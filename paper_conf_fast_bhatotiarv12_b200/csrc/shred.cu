@@ -523,9 +523,8 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
 int launch_scatter(shred_ctx *ctx, Plan &pl, uint64_t *dst, uint64_t dst_cap, Aux *aux, int streaming,
                    uint64_t *n_direct, cudaStream_t st) {
     if (pl.nslots == 0) {
-        PDL(k_write_u64, 1, 1, 0, st, &aux->total, 0);
-        LAUNCHED("k_write_u64");
-        if (n_direct) { PDL(k_write_u64, 1, 1, 0, st, n_direct, 0); LAUNCHED("k_write_u64"); }
+        PDL(k_no_slots, 1, 1, 0, st, aux, n_direct);
+        LAUNCHED("k_no_slots");
         return SHRED_OK;
     }
     PDL(k_scatter, (pl.nslots + SCATTER_THREADS - 1) / SCATTER_THREADS, SCATTER_THREADS, 0, st, 
@@ -553,7 +552,7 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
     A.spec_exit = b; A.spec_cnt = b + (nb + 2); A.entry = b + 2 * (nb + 2); A.offs = b + 3 * (nb + 2);
     A.delta = (int64_t *)(b + 4 * (nb + 2)); A.ok = (uint32_t *)(b + 5 * (nb + 2));
     A.cta_sum = b + 6 * (nb + 2); A.cta_ok = b + 7 * (nb + 2); A.cta_off = b + 8 * (nb + 2);
-    A.dst = dst; A.dst_cap = cap; A.aux = aux;
+    A.dst = dst; A.dst_cap = cap; A.aux = aux; A.tile = SB_THREADS;
     // tiles of SB_THREADS blocks, at most 8 CTAs per SM (grid-stride over the true tile count)
     const uint64_t gmax = (uint64_t)ctx->sm_count * 8;
     uint64_t g = (nb + SB_THREADS - 1) / SB_THREADS;
@@ -805,6 +804,8 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
     }
     if (cudaFuncSetAttribute(sb_dense, cudaFuncAttributeMaxDynamicSharedMemorySize,
                              (int)(SBD_WIN / 8)) != cudaSuccess ||
+        cudaFuncSetAttribute(sb_one, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             (int)(SBD_WIN / 8 > SBO_SMEM ? SBD_WIN / 8 : SBO_SMEM)) != cudaSuccess ||
         cudaFuncSetAttribute(k_hash_chunks_ws, cudaFuncAttributeMaxDynamicSharedMemorySize,
                              (int)HWS_SMEM) != cudaSuccess)
         return bail(SHRED_ECUDA);
@@ -837,6 +838,51 @@ void shred_destroy(shred_ctx *ctx) {
     delete ctx;
 }
 
+// SBArgs of a one-shot bounded call whose ordered candidate list is ctx->d_cand (capacity ccap,
+// count in aux->ncand), with the size-rule scratch for it.
+int one_shot_sbargs(shred_ctx *ctx, uint64_t ccap, uint64_t len, uint64_t *d_out, uint64_t cap, uint32_t tile,
+                    SBArgs &A) {
+    Aux *aux = ctx->d_aux + 0;
+    const uint64_t nb = (ccap + SB_B - 1) / SB_B;
+    int rc = grow(ctx, ctx->d_sb, ctx->sb_cap, 9 * (nb + 2), "size-rule scratch");
+    if (rc) return rc;
+    A.cand = ctx->d_cand; A.n_dev = &aux->ncand; A.n_host = 0; A.n_cap = ccap;
+    A.minsz = ctx->p.min_size; A.maxsz = ctx->p.max_size; A.end = len; A.fin = 1;
+    uint64_t *b = ctx->d_sb;
+    A.spec_exit = b; A.spec_cnt = b + (nb + 2); A.entry = b + 2 * (nb + 2); A.offs = b + 3 * (nb + 2);
+    A.delta = (int64_t *)(b + 4 * (nb + 2)); A.ok = (uint32_t *)(b + 5 * (nb + 2));
+    A.cta_sum = b + 6 * (nb + 2); A.cta_ok = b + 7 * (nb + 2); A.cta_off = b + 8 * (nb + 2);
+    A.dst = d_out; A.dst_cap = cap; A.aux = aux; A.tile = tile;
+    return SHRED_OK;
+}
+
+// One-shot bounded call on a small input: k1 -> k_scatter (ordered candidates) -> sb_one (the
+// whole size rule, the state set-up and the call end in one CTA).  Three launches instead of
+// eight; the multi-CTA sb_* chain is launch-latency bound at these sizes (1 MiB: 27 us per call).
+int chunk_bounded_one(shred_ctx *ctx, Plan &pl, uint64_t len, uint64_t *d_out, uint64_t cap,
+                      uint64_t *n_out, cudaStream_t st) {
+    Aux *aux = ctx->d_aux + 0;
+    int rc;
+    if ((rc = launch_detect(ctx, pl, st))) return rc;
+    const uint64_t ccap = (uint64_t)pl.nslots * pl.J.cap + 1;
+    if ((rc = grow(ctx, ctx->d_cand, ctx->cand_cap, ccap, "candidate list"))) return rc;
+    if ((rc = launch_scatter(ctx, pl, ctx->d_cand, ccap, aux, 0, nullptr, st))) return rc;
+    SBArgs A{};
+    if ((rc = one_shot_sbargs(ctx, ccap, len, d_out, cap, SBO_THREADS, A))) return rc;
+    size_t smem = 0;
+    if (pl.nslots) {
+        uint64_t maxseg = pl.J.map.S;
+        if (pl.J.map.head_seg > maxseg) maxseg = pl.J.map.head_seg;
+        if (pl.J.map.tail_seg > maxseg) maxseg = pl.J.map.tail_seg;
+        if (maxseg > SBD_WIN) maxseg = SBD_WIN;
+        smem = (size_t)((maxseg + 31) / 32) * 4;
+    }
+    if (smem < SBO_SMEM) smem = SBO_SMEM;
+    PDL(sb_one, 1, SBO_THREADS, smem, st, pl.J, ctx->dp, ctx->d_gen, pl.nslots, A, n_out, cap);
+    LAUNCHED("sb_one");
+    return SHRED_OK;
+}
+
 int shred_chunk(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, uint64_t *d_out, uint64_t cap,
                 uint64_t *n_out, shred_stream_t stream) {
     if (!ctx) return SHRED_EINVAL;
@@ -847,12 +893,17 @@ int shred_chunk(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, uint64_t *d_o
     cudaStream_t st = (cudaStream_t)stream;
     StreamOrder so(ctx, st);
     Aux *aux = ctx->d_aux + 0;
+    Plan pl;
+    if ((rc = plan_job(ctx, pl, d_in, 0, nullptr, 0, 0, len, len))) return rc;
     if (!bounded(ctx)) {
-        Plan pl;
-        if ((rc = plan_job(ctx, pl, d_in, 0, nullptr, 0, 0, len, len))) return rc;
         if ((rc = launch_detect(ctx, pl, st))) return rc;
         return launch_scatter(ctx, pl, d_out, cap, aux, 0, n_out, st);
     }
+    // few expected candidates (random-like data fits sb_one's shared-memory form): one CTA runs
+    // the whole size rule (exact for any count; dense inputs take its global or sb_dense form)
+    if (SB_ONE_MAX_LEN && len <= SB_ONE_MAX_LEN &&
+        (long double)len * (long double)hits_per_d(ctx->p) / (long double)ctx->p.divisor <= (long double)SB_ONE_EXPECT)
+        return chunk_bounded_one(ctx, pl, len, d_out, cap, n_out, st);
     PDL(k_stream_reset, 1, 1, 0, st, aux);
     LAUNCHED("k_stream_reset");
     if ((rc = run_piece(ctx, aux, d_in, 0, nullptr, 0, 0, len, len, 1, d_out, cap, st))) return rc;

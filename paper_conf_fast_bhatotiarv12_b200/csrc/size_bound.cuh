@@ -48,6 +48,7 @@ struct SBArgs {
     uint64_t *cta_sum, *cta_ok, *cta_off;            // [ncta] per spec_check CTA (two-level scan)
     uint64_t *dst; uint64_t dst_cap;
     Aux *aux;                       // s, held, held_val, out_pos (streaming state)
+    uint32_t tile;                  // blocks per tile = the threads of the CTA running the phases
 };
 
 __device__ __forceinline__ uint64_t sb_n(const SBArgs &A) {
@@ -85,13 +86,14 @@ __device__ __forceinline__ uint64_t sb_tail_count(uint64_t s, const SBArgs &A) {
 // then block b from its own guess and, in lockstep, from X until the two states coincide.
 // Tiles of SB_THREADS blocks; CTA i takes tiles i, i + gridDim.x, ... (the grid is sized for the
 // capacity bound, the tile count comes from the true count on the device).
-__global__ void __launch_bounds__(SB_THREADS) sb_spec_check(SBArgs A) {
-    pdl_entry();
-    if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
+// The phases are device functions so that one CTA can run them back to back (sb_one): tiles of
+// A.tile = blockDim.x blocks, CTA `bid` of `nblk` takes tiles bid, bid + nblk, ...
+__device__ __forceinline__ void sb_spec_body(const SBArgs &A, uint32_t bid, uint32_t nblk) {
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
-    for (uint64_t tile = blockIdx.x; tile * SB_THREADS < nb; tile += gridDim.x) {
-    const uint64_t b = tile * SB_THREADS + threadIdx.x;
+    const uint32_t T = blockDim.x;
+    for (uint64_t tile = bid; tile * T < nb; tile += nblk) {
+    const uint64_t b = tile * T + threadIdx.x;
     uint64_t cnt = 0;
     bool synced = true;
     if (b < nb) {
@@ -134,7 +136,7 @@ __global__ void __launch_bounds__(SB_THREADS) sb_spec_check(SBArgs A) {
         cnt = (uint64_t)((int64_t)cg + ct - cg_sync);
     }
     // per-CTA sum of the counts (valid if every block synced) and AND of the sync flags
-    __shared__ uint64_t red[SB_THREADS / 32];
+    __shared__ uint64_t red[32];
     uint64_t x = cnt;
     for (int d = 16; d; d >>= 1) x += __shfl_xor_sync(0xffffffffu, x, d);
     const int all = __syncthreads_and(synced ? 1 : 0);
@@ -142,25 +144,27 @@ __global__ void __launch_bounds__(SB_THREADS) sb_spec_check(SBArgs A) {
     __syncthreads();
     if (threadIdx.x == 0) {
         uint64_t t = 0;
-        for (int w = 0; w < SB_THREADS / 32; ++w) t += red[w];
+        for (uint32_t w = 0; w < T / 32; ++w) t += red[w];
         A.cta_sum[tile] = t;
         A.cta_ok[tile] = all ? 1u : 0u;
     }
     __syncthreads();                          // red reused by the next tile
     }
 }
+__global__ void __launch_bounds__(SB_THREADS) sb_spec_check(SBArgs A) {
+    pdl_entry();
+    if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
+    sb_spec_body(A, blockIdx.x, gridDim.x);
+}
 
 // One CTA: entries, offsets, totals and the streaming state.  Each thread owns a contiguous
 // range of blocks; one block scan of the range sums gives every block's offset.
-__global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
-    pdl_entry();
-    __shared__ uint32_t ws[33];
+__device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
     __shared__ uint64_t wsum[33];
-    if (A.aux->dense) return;
     const uint64_t n = sb_n(A);
     const uint32_t nb = (uint32_t)((n + SB_B - 1) / SB_B);
     const uint32_t tid = threadIdx.x;
-    const uint32_t nc = (nb + SB_THREADS - 1) / SB_THREADS;         // spec_check CTAs with blocks
+    const uint32_t nc = (nb + A.tile - 1) / A.tile;                 // tiles with blocks
     const uint32_t per = (nc + blockDim.x - 1) / blockDim.x;
     const uint32_t ca = min(nc, tid * per), cb = min(nc, ca + per);
     uint64_t sum = 0;
@@ -183,7 +187,7 @@ __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
         __syncthreads();
         if (tid == 0) {
             uint64_t r = 0;
-            for (int w = 0; w < 32; ++w) { uint64_t x = wsum[w]; wsum[w] = r; r += x; }
+            for (uint32_t w = 0; w < (blockDim.x >> 5); ++w) { uint64_t x = wsum[w]; wsum[w] = r; r += x; }
             wsum[32] = r;
         }
         __syncthreads();
@@ -248,17 +252,21 @@ __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
     aux->held = (uint64_t)held;
     aux->held_val = held ? A.end : 0;
 }
+__global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
+    pdl_entry();
+    if (A.aux->dense) return;
+    sb_plan_body(A);
+}
 
 // Every block writes its cuts; thread nb writes the forced cuts after the last candidate.
-__global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
-    pdl_entry();
-    if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
+__device__ __forceinline__ void sb_emit_body(const SBArgs &A, uint32_t bid, uint32_t nblk) {
     const uint64_t n = sb_n(A);
     const uint64_t nb = (n + SB_B - 1) / SB_B;
     const bool fast = A.aux->sb_fast != 0;
-    __shared__ uint64_t ws[SB_THREADS / 32 + 1];
-    for (uint64_t tile = blockIdx.x; tile * SB_THREADS <= nb; tile += gridDim.x) {
-        const uint64_t b = tile * SB_THREADS + threadIdx.x;
+    const uint32_t T = blockDim.x;
+    __shared__ uint64_t ws[33];
+    for (uint64_t tile = bid; tile * T <= nb; tile += nblk) {
+        const uint64_t b = tile * T + threadIdx.x;
         uint64_t s = 0, o = 0;
         if (fast) {
             // entry = the previous block's spec exit; offset = tile offset + in-tile exclusive prefix
@@ -298,6 +306,11 @@ __global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
             if (first + j < last) sb_step(s, v[j], A, held, emit);
     }
 }
+__global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
+    pdl_entry();
+    if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
+    sb_emit_body(A, blockIdx.x, gridDim.x);
+}
 
 // ------------------------------------------------------------------------------ sb_dense
 // Exact fallback when the ordered candidate list could not hold every candidate (only possible
@@ -307,11 +320,9 @@ __global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
 // windows of SBD_WIN window ends) that warp 0 then scans in order.
 constexpr int SBD_THREADS = 256;
 constexpr uint64_t SBD_WIN = 1ull << 20;              // window ends per bitmap pass (128 KiB)
-__global__ void __launch_bounds__(SBD_THREADS)
-sb_dense(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots, SBArgs A) {
-    pdl_entry();
+__device__ __forceinline__ void sb_dense_body(const Job &J, const DevParams &P, const GenTables *__restrict__ gt,
+                                              uint32_t nslots, const SBArgs &A) {
     Aux *aux = A.aux;
-    if (!aux->dense) return;
     extern __shared__ uint32_t bm[];
     __shared__ uint64_t sT[256], sU[256];
     for (int i = threadIdx.x; i < 256; i += blockDim.x) { sT[i] = gt->T[i]; sU[i] = gt->U[i]; }
@@ -374,6 +385,167 @@ sb_dense(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots, 
         aux->s = s + mt * A.maxsz;
         aux->held = (uint64_t)held;
         aux->held_val = held ? A.end : 0;
+    }
+}
+__global__ void __launch_bounds__(SBD_THREADS)
+sb_dense(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots, SBArgs A) {
+    pdl_entry();
+    if (!A.aux->dense) return;
+    sb_dense_body(J, P, gt, nslots, A);
+}
+
+// ------------------------------------------------------------------------------ sb_one
+// A whole one-shot bounded call's size rule in ONE CTA, plus the call's state set-up and end
+// (k_stream_reset / k_call_end): the chain after k_scatter is one launch instead of five.  Used
+// for inputs up to SB_ONE_MAX_LEN, where the multi-CTA chain is bound by its dependent global
+// round trips and launches (1 MiB: 26.5 us per call in a CUDA graph, 7.3 unbounded).
+// Fast form (n <= 8,176 candidates): the candidates are loaded into shared memory once and
+// the three phases of the parallel rule run there, one block of SB_B candidates per thread:
+//   spec  thread b runs block b from its guess g_b = c[16b - 1] (block 0: s = 0) -> exit E_b,
+//         count C_b; and, in lockstep, from X = E_{b-1} (block b-1 rerun from ITS guess by the
+//         same thread) until the two states coincide -> delta_b, synced_b;
+//   plan  every block synced: the true entry of block b is E_{b-1} (induction from block 0,
+//         which is exact), offsets = exclusive scan of C_b + delta_b; otherwise thread 0 walks
+//         the blocks in order, re-walking candidate by candidate those whose entry is not the
+//         one their sync assumed;
+//   emit  block b reruns from its true entry and writes its cuts; the last thread writes the
+//         forced cuts after the last candidate.
+// Larger counts run the global-memory phases above (sb_*_body); dense lists sb_dense_body.
+constexpr int SBO_THREADS = 512;
+constexpr uint32_t SBO_SMEM_N = SBO_THREADS * SB_B;       // 8192 candidates, 64 KiB
+constexpr size_t SBO_SMEM = (size_t)SBO_SMEM_N * 8 + (size_t)SBO_THREADS * 8 * 4;
+#ifndef SHRED_SB_ONE_MAX
+#define SHRED_SB_ONE_MAX (256ull << 20)  // A/B: 0 = always the multi-CTA chain
+#endif
+constexpr uint64_t SB_ONE_MAX_LEN = SHRED_SB_ONE_MAX;
+constexpr uint64_t SB_ONE_EXPECT = 6144;  // expected candidates (len (r+1 | 1) / D) up to which sb_one runs
+
+__device__ __forceinline__ void sb_one_smem(const SBArgs &A, uint32_t n, uint64_t *n_out, uint64_t cap,
+                                            bool loaded = false) {
+    extern __shared__ uint64_t sm64[];
+    uint64_t *sc = sm64;                                   // candidates [n]
+    uint64_t *ex = sc + SBO_SMEM_N;                        // spec exit E_b
+    uint64_t *cn = ex + SBO_THREADS;                       // count along the true path (synced)
+    uint64_t *en = cn + SBO_THREADS;                       // true entry
+    uint64_t *of = en + SBO_THREADS;                       // output offset
+    __shared__ uint32_t okb[SBO_THREADS];
+    __shared__ uint64_t wsum[SBO_THREADS / 32 + 1];
+    const uint32_t tid = threadIdx.x;
+    if (!loaded)
+        for (uint32_t i = tid; i < n; i += SBO_THREADS) sc[i] = A.cand[i];
+    __syncthreads();
+    const uint32_t nb = (n + SB_B - 1) / SB_B;
+    const uint32_t b = tid;
+    int h0 = 0;
+    uint64_t cnt = 0;
+    bool synced = true;
+    if (b < nb) {
+        const uint32_t first = b * SB_B, last = min(n, first + SB_B);
+        uint64_t X = 0;
+        if (b) {
+            const uint32_t pf = first - SB_B;
+            X = (b - 1) ? sc[pf - 1] : 0ull;
+            for (uint32_t j = pf; j < first; ++j) sb_step(X, sc[j], A, h0, NoEmit{});
+        }
+        uint64_t sg = b ? sc[first - 1] : 0ull, st = X;
+        uint64_t cg = 0;
+        int64_t ct = 0, cgs = 0;
+        synced = (b == 0) || (X == sg);
+        for (uint32_t j = first; j < last; ++j) {
+            const uint64_t k = sb_step(sg, sc[j], A, h0, NoEmit{});
+            cg += k;
+            if (!synced) {
+                ct += (int64_t)sb_step(st, sc[j], A, h0, NoEmit{});
+                cgs += (int64_t)k;
+                synced = st == sg;
+            }
+        }
+        ex[b] = sg;
+        cnt = (uint64_t)((int64_t)cg + ct - cgs);
+        cn[b] = cnt;
+        okb[b] = synced ? 1u : 0u;
+    }
+    const int all_ok = __syncthreads_and(synced ? 1 : 0);
+    if (all_ok) {
+        uint64_t incl = cnt;                               // block exclusive scan of the counts
+        for (int d = 1; d < 32; d <<= 1) {
+            const uint64_t u = __shfl_up_sync(0xffffffffu, incl, d);
+            if ((tid & 31) >= (uint32_t)d) incl += u;
+        }
+        if ((tid & 31) == 31) wsum[tid >> 5] = incl;
+        __syncthreads();
+        if (tid == 0) {
+            uint64_t r = 0;
+            for (int w = 0; w < SBO_THREADS / 32; ++w) { const uint64_t x = wsum[w]; wsum[w] = r; r += x; }
+            wsum[SBO_THREADS / 32] = r;
+        }
+        __syncthreads();
+        if (b < nb) { of[b] = wsum[tid >> 5] + incl - cnt; en[b] = b ? ex[b - 1] : 0ull; }
+        if (tid == 0) { of[nb] = wsum[SBO_THREADS / 32]; en[nb] = nb ? ex[nb - 1] : 0ull; }
+    } else if (tid == 0) {
+        // exact sequential walk: a block keeps its spec result if its true entry is the state
+        // its sync assumed (E_{b-1}) and it synced, else it is re-walked
+        uint64_t s = 0, off = 0;
+        int h = 0;
+        for (uint32_t k = 0; k < nb; ++k) {
+            en[k] = s; of[k] = off;
+            if (k == 0 || (okb[k] && s == ex[k - 1])) {
+                off += cn[k];
+                s = ex[k];
+            } else {
+                const uint32_t first = k * SB_B, last = min(n, first + SB_B);
+                for (uint32_t j = first; j < last; ++j) off += sb_step(s, sc[j], A, h, NoEmit{});
+            }
+        }
+        en[nb] = s; of[nb] = off;
+    }
+    __syncthreads();
+    uint64_t *dst = A.dst;
+    if (b <= nb) {
+        uint64_t s = en[b], o = of[b];
+        auto emit = [&](uint64_t v) { if (o < cap) dst[o] = v; ++o; };
+        if (b == nb) {
+            const uint64_t mt = sb_tail_count(s, A);
+            for (uint64_t j = 1; j <= mt; ++j) emit(s + j * A.maxsz);
+            Aux *aux = A.aux;                              // the call's end (k_call_end)
+            aux->out_pos = o; aux->total = o;
+            aux->s = s + mt * A.maxsz; aux->held = 0; aux->held_val = 0;
+            *n_out = o;
+            if (o > cap) aux->overflow = 1;
+        } else {
+            const uint32_t first = b * SB_B, last = min(n, first + SB_B);
+            int h = 0;
+            for (uint32_t j = first; j < last; ++j) sb_step(s, sc[j], A, h, emit);
+        }
+    }
+}
+
+__global__ void __launch_bounds__(SBO_THREADS)
+sb_one(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots, SBArgs A, uint64_t *n_out,
+       uint64_t cap) {
+    pdl_entry();
+    Aux *aux = A.aux;
+    const uint64_t dense = aux->dense, n = sb_n(A);
+    if (!dense && n <= SBO_SMEM_N - SB_B) {                // nb < SBO_THREADS: thread nb writes the tail
+        sb_one_smem(A, (uint32_t)n, n_out, cap);
+        return;
+    }
+    __syncthreads();                                       // every thread has read the state
+    if (threadIdx.x == 0) { aux->s = 0; aux->held = 0; aux->held_val = 0; aux->out_pos = 0; }
+    __syncthreads();
+    if (dense) {
+        sb_dense_body(J, P, gt, nslots, A);
+    } else {
+        sb_spec_body(A, 0, 1);
+        __syncthreads();
+        sb_plan_body(A);
+        __syncthreads();
+        sb_emit_body(A, 0, 1);
+    }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        *n_out = aux->out_pos;
+        if (aux->out_pos > cap) aux->overflow = 1;
     }
 }
 

@@ -604,3 +604,38 @@ def test_k32t_small_shape_and_le_marker_modes(pkg):
         ch = pkg.Chunker(p)
         assert ch.mode == mode, (p, ch.mode)
         check_chunk(ch, data)
+
+
+# ------------------------------------------------------------------ one-CTA size rule (sb_one)
+def _periodic_marker_pattern(period: int, p) -> bytes:
+    """A random `period`-byte pattern one of whose window phases is a marker under p (found with
+    the oracle), so its repetition has a candidate every `period` bytes."""
+    rng = np.random.default_rng(period)
+    for _ in range(200000):
+        pat = bytes(rng.integers(0, 256, period, dtype=np.uint8))
+        if oracle.candidates(synthgen.periodic(pat, 3 * period + p.window), oparams(p)).size:
+            return pat
+    raise AssertionError("no marker pattern found")
+
+
+@pytest.mark.parametrize("kind", ["random", "periodic64", "dense04d5", "short"])
+def test_bounded_one_shot_one_cta_paths(pkg, kind):
+    """One-shot bounded calls with few expected candidates run the whole size rule in one CTA
+    (sb_one): its shared-memory form (random data), its global-memory phases (> 8,176 actual
+    candidates without list overflow: a 64-byte period with a marker, 16 K candidates per MiB),
+    and its dense form (list overflow, `04 D5`); all equal the oracle (L259-L265)."""
+    p = pkg.Params(min_size=16, max_size=200) if kind != "random" else pkg.Params(min_size=2048, max_size=65536)
+    n = (1 << 20) + 13
+    if kind == "random":
+        data = synthgen.random_bytes(77, n)
+    elif kind == "periodic64":
+        data = synthgen.periodic(_periodic_marker_pattern(64, pkg.Params()), n)
+    elif kind == "dense04d5":
+        data = synthgen.periodic(b"\x04\xd5", n)
+    else:
+        data = synthgen.random_bytes(78, 1000)
+    got = check_chunk(pkg.Chunker(p), data)
+    if kind == "periodic64":
+        assert oracle.candidates(data, oparams(p)).size > 8176
+    if kind != "short":
+        assert got.size > 0

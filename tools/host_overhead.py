@@ -10,7 +10,7 @@ import paper_conf_fast_bhatotiarv12_b200 as pkg  # noqa: E402
 
 x = torch.empty(1 << 20, dtype=torch.uint8, device="cuda")
 pkg.synth_fill(x, 1)
-ch = pkg.Chunker(pkg.Params())
+ch = pkg.Chunker(pkg.Params(min_size=2048, max_size=65536) if "--bounded" in sys.argv else pkg.Params())
 o = torch.empty(4096, dtype=torch.int64, device="cuda")
 n = torch.zeros(1, dtype=torch.int64, device="cuda")
 lib = pkg.lib()

@@ -1,7 +1,7 @@
 """Per-call latency and rate of shred_chunk over input sizes (device-resident, paper params and
 the k32 variant): the launch-shape switch (small shape below ~19 MB) shows up here.
 
-Usage (GPU box): python tools/size_latency.py [--json out.jsonl]
+Usage (GPU box): python tools/size_latency.py [--json out.jsonl] [--bounded]
 """
 import argparse
 import json
@@ -19,9 +19,13 @@ SIZES = [64 << 10, 256 << 10, 1 << 20, 4 << 20, 16 << 20, 19 << 20, 24 << 20, 64
 def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--json", default=None)
+    ap.add_argument("--bounded", action="store_true", help="also the size rule on (min 2048 / max 65536)")
     a = ap.parse_args()
     out = open(a.json, "w") if a.json else None
-    for name, p in (("paper", pkg.Params()), ("k32", pkg.Params(poly=0x104C11DB7))):
+    cases = [("paper", pkg.Params()), ("k32", pkg.Params(poly=0x104C11DB7))]
+    if a.bounded:
+        cases.append(("paper_bounded", pkg.Params(min_size=2048, max_size=65536)))
+    for name, p in cases:
         ch = pkg.Chunker(p)
         for n in SIZES:
             x = torch.empty(n, dtype=torch.uint8, device="cuda")
