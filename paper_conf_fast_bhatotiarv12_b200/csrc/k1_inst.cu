@@ -2,7 +2,7 @@
 //
 // _build.py compiles this file once per SHRED_INST value (in parallel) and links the objects
 // with shred.cu:  SHRED_INST = MODE_K63 / MODE_K40 / MODE_K32 / MODE_K32B instantiates
-// k1_bulk<MODE, Cfg, ceil(w/16), marker kind, funnel> for that mode (24 instances), and
+// k1_bulk<MODE, Cfg, ceil(w/16) (0: w > 64), marker kind, funnel> for that mode, and
 // SHRED_INST = 0 the dispatchers pick_k1 / pick_k1_small plus the small-input shapes.
 #define SHRED_K1_ONLY
 #include <type_traits>
@@ -21,6 +21,8 @@ template <int MODE> K1Fn pick_mode(int wch, int mk, bool fn);
 template <int MODE, class C, int MK>
 static K1Fn pick_w(int wch, bool fn) {
     switch (wch * 2 + (fn ? 1 : 0)) {           // fn: w not a multiple of 16 (funnel-shifted pops)
+        case 0: return k1_bulk<MODE, C, 0, MK, false>;   // wch 0: long windows (w > 64, pops by TMA)
+        case 1: return k1_bulk<MODE, C, 0, MK, true>;
         case 2: return k1_bulk<MODE, C, 1, MK, false>;
         case 3: return k1_bulk<MODE, C, 1, MK, true>;
         case 4: return k1_bulk<MODE, C, 2, MK, false>;

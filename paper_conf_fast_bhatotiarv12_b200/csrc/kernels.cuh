@@ -105,6 +105,16 @@ using CfgK32 = BulkCfg<SHRED_K32_CH, SHRED_K32_NT>;
 #define SHRED_SMALL_NT 128    // 128 consumers x 2 rows; 64 (128-row CTAs, 129 CTAs for 1 MiB): slower (r01_ab_variants)
 #endif
 using CfgSmall = BulkCfg<2, SHRED_SMALL_NT, SHRED_DIRECT_WARM != 0>;
+// Long windows (w > 64, the hot kernel's WCH = 0 instances): the bytes leaving the window come
+// from a second TMA tile per stage, [16 * ceil(w/16)] bytes behind the data tile, 48 bytes per row
+// and round (the round's two aligned pop chunks plus the next one for the funnel), unswizzled
+// (rows 48 B apart: the 8 rows of a quarter warp hit 8 distinct bank groups).
+constexpr int LW_POPW = 48;
+template <class C> struct LwLayout {
+    static constexpr int POP_STAGE = C::ROWS * LW_POPW;
+    static constexpr int BAR_OFF = TAB_BYTES + STAGES * (C::STAGE + POP_STAGE);
+    static constexpr int SMEM = BAR_OFF + 2048;
+};
 
 // Slot id -> range of window-end positions.  Slots are numbered in stream order:
 // [0, n_head) generic head segments, then the bulk rows, then generic tail segments.
@@ -798,6 +808,7 @@ struct BulkConst {
     uint32_t w;                // window bytes (DIRECT_WARM)
     uint32_t fu, fsel;  // FN windows (w % 16 != 0): e = 16*ceil(w/16) - w = 4*fu + v, fsel = PRMT
                         // selector of bytes v..v+3 (0x3210 + 0x1111 v)
+    uint32_t wa;        // ceil(w/16): the long-window mode's warm-up chunks and pop distance
 };
 
 // The 16 bytes leaving the window at chunk q are bytes [16(q-A) + e, +16), A = WCH = ceil(w/16),
@@ -836,8 +847,10 @@ __device__ __forceinline__ void pops16(const uint4 (&lo)[CH], const uint4 (&hi)[
 // (w in {16, 32, 48, 64}) generalises the pop distance; MK selects the marker kind.
 template <int MODE, class C, int WCH, int MK, bool FN = false>
 __global__ void __launch_bounds__(C::NTC + 32, 1)
-k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_img,
-        const GenTables *__restrict__ gt, Job J, DevParams P, BulkConst K) {
+k1_bulk(const __grid_constant__ CUtensorMap tmap, const __grid_constant__ CUtensorMap tmap_pop,
+        const uint4 *__restrict__ tab_img, const GenTables *__restrict__ gt, Job J, DevParams P, BulkConst K) {
+    constexpr bool LW = WCH == 0;                    // long window (w > 64): pops from a TMA tile
+    constexpr int BAR_OFF = LW ? LwLayout<C>::BAR_OFF : C::BAR_OFF;
     if (SHRED_PDL_EARLY) pdl_trigger(); else pdl_entry();
     constexpr int CH = C::CH, NTC = C::NTC, ROUND = C::ROUND, CPR = C::CPR;
     extern __shared__ uint8_t smem_raw[];
@@ -845,8 +858,9 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
     uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
     const uint32_t sbase = smem_u32(smem);
     const uint32_t stages = sbase + TAB_BYTES;
-    const uint32_t bars = sbase + C::BAR_OFF;      // full[s] at +8s, empty[s] at +64+8s
-    uint32_t *ws = reinterpret_cast<uint32_t *>(smem + C::BAR_OFF + 128);
+    const uint32_t bars = sbase + BAR_OFF;         // full[s] at +8s, empty[s] at +64+8s
+    uint32_t *ws = reinterpret_cast<uint32_t *>(smem + BAR_OFF + 128);
+    const uint32_t popst = stages + STAGES * C::STAGE;       // LW: the pop tiles
     const int tid = threadIdx.x;
 
     if (blockIdx.x == J.map.nc) {                    // ---- edge CTA: head + tail, generic loop
@@ -914,12 +928,19 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
             for (uint32_t r = 0; r < nrounds; ++r) {
                 const uint32_t s = r % STAGES;
                 if (r >= STAGES) mbar_wait_sleep(bars + 64 + 8 * s, ((r / STAGES) - 1u) & 1u);
-                mbar_expect_tx(bars + 8 * s, C::STAGE);
+                mbar_expect_tx(bars + 8 * s, LW ? C::STAGE + LwLayout<C>::POP_STAGE : C::STAGE);
                 const uint32_t dst = stages + s * C::STAGE;
 #pragma unroll
                 for (int q = 0; q < C::ROWS / C::BOX; ++q)
                     tma_load_2d(dst + q * C::BOX * ROUND, &tmap, (int)(r * ROUND), (int)(row0 + q * C::BOX),
                                 bars + 8 * s);
+                if (LW) {
+                    const uint32_t pd = popst + s * LwLayout<C>::POP_STAGE;
+#pragma unroll
+                    for (int q = 0; q < C::ROWS / C::BOX; ++q)
+                        tma_load_2d(pd + q * C::BOX * LW_POPW, &tmap_pop, (int)(r * ROUND), (int)(row0 + q * C::BOX),
+                                    bars + 8 * s);
+                }
             }
         }
         return;
@@ -1010,6 +1031,39 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
             pops16<FN, CH>(lo, hi, p, K);
             chunk16xN<MODE, CH, false, MK>(st, d, p, c, m);
         }
+        if (LW) {
+            // long window: roll the 16*wa bytes before the row (inside src: the plan keeps b0 >=
+            // p_begin + 16*wa) from a zero state.  Their pops lie before the warm-up start
+            // (virtual zeros), except in the last chunk: bytes [16 - e, 16) of its pops are the
+            // warm-up's first e bytes (e = 16*wa - w), i.e. the funnel of (zero, first chunk).
+            uint4 first[CH], nxt[CH];
+            auto wload = [&](int ch, uint32_t k) {     // warm-up chunk k of chain ch
+                return act[ch] ? __ldg(reinterpret_cast<const uint4 *>(
+                                     J.src + (pos0[ch] - 16ull * K.wa + 16ull * k - J.p_begin)))
+                               : Z;
+            };
+#pragma unroll
+            for (int ch = 0; ch < CH; ++ch) nxt[ch] = wload(ch, 0);
+            for (uint32_t k = 0; k < K.wa; ++k) {
+                uint4 d[CH], p[CH];
+#pragma unroll
+                for (int ch = 0; ch < CH; ++ch) {
+                    d[ch] = nxt[ch];                     // the next chunk's load overlaps this one's steps
+                    if (k + 1 < K.wa) nxt[ch] = wload(ch, k + 1);
+                    if (k == 0) first[ch] = d[ch];
+                }
+                if (k + 1 == K.wa) {
+                    uint4 zl[CH];
+#pragma unroll
+                    for (int ch = 0; ch < CH; ++ch) zl[ch] = Z;
+                    pops16<FN, CH>(zl, first, p, K);
+                } else {
+#pragma unroll
+                    for (int ch = 0; ch < CH; ++ch) p[ch] = Z;
+                }
+                chunk16xN<MODE, CH, false, MK>(st, d, p, c, m);
+            }
+        }
     }
 
     // TMA swizzle of the 16-byte chunk index (rows of ROUND bytes; tid + ch*NTC has the same
@@ -1029,6 +1083,25 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
 #pragma unroll
                 for (int u = 0; u < CPR; ++u)
                     D[ch][u] = lds128(sb + (uint32_t)(tid + ch * NTC) * ROUND + (((uint32_t)u ^ swz) << 4));
+            // LW: the round's pop chunks (aligned, 16*wa bytes behind) and the next one (funnel)
+            uint4 PQ[CH][LW ? CPR + 1 : 1];
+            if (LW) {
+                const uint32_t pb = popst + s * LwLayout<C>::POP_STAGE;
+#pragma unroll
+                for (int ch = 0; ch < CH; ++ch)
+#pragma unroll
+                    for (int u = 0; u < (LW ? CPR + 1 : 1); ++u)
+                        if (u < CPR || FN) PQ[ch][u] = lds128(pb + (uint32_t)(tid + ch * NTC) * LW_POPW + 16u * u);
+                if (FN && r + qr + 1 == nrounds) {
+                    // the last round's funnel chunk lies past the pop tile's rows (zero fill): the
+                    // same bytes from global memory (the row's own data, 16*wa - S + ... behind)
+#pragma unroll
+                    for (int ch = 0; ch < CH; ++ch)
+                        if (act[ch])
+                            PQ[ch][CPR] = __ldg(reinterpret_cast<const uint4 *>(
+                                J.src + (pos0[ch] + (uint64_t)nrounds * ROUND - 16ull * K.wa - J.p_begin)));
+                }
+            }
             __syncwarp();
             if (lane == 0) mbar_arrive(bars + 64 + 8 * s);
 #pragma unroll
@@ -1042,8 +1115,13 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
                     uint4 lo[CH], hi[CH];
 #pragma unroll
                     for (int ch = 0; ch < CH; ++ch) {
-                        lo[ch] = R[ch][(cq + 4 - WCH) & 3];
-                        hi[ch] = (WCH == 1) ? D[ch][u] : R[ch][(cq + 5 - WCH) & 3];
+                        if (LW) {
+                            lo[ch] = PQ[ch][u];
+                            hi[ch] = PQ[ch][LW ? u + 1 : 0];
+                        } else {
+                            lo[ch] = R[ch][(cq + 4 - WCH) & 3];
+                            hi[ch] = (WCH == 1) ? D[ch][u] : R[ch][(cq + 5 - WCH) & 3];
+                        }
                     }
                     pops16<FN, CH>(lo, hi, p, K);
                 }
@@ -1087,8 +1165,8 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const uint4 *__restrict__ tab_
 }
 
 // A hot-kernel instance; pick_k1 / pick_k1_small (k1_inst.cu) map parameters to instances.
-typedef void (*K1Fn)(const __grid_constant__ CUtensorMap, const uint4 *, const GenTables *, Job,
-                     DevParams, BulkConst);
+typedef void (*K1Fn)(const __grid_constant__ CUtensorMap, const __grid_constant__ CUtensorMap, const uint4 *,
+                     const GenTables *, Job, DevParams, BulkConst);
 K1Fn pick_k1(int k, bool byteidx, int wch, int mk, bool fn, bool tprod = false);
 K1Fn pick_k1_small(int k, bool byteidx, int wch, int mk, bool fn, bool tprod = false);
 

@@ -137,6 +137,7 @@ struct shred_ctx {
     uint64_t tm_key[4] = {0, 0, 0, 0};
     bool tm_valid = false;
     K1Fn k1_fn = nullptr;                // the hot-kernel instance for these parameters
+    int k1_smem = 0;                     // its dynamic shared memory
     K1Fn k1_small_fn = nullptr;          // the same with the small-input shape (or null)
     int sm_count = 148;
 
@@ -274,11 +275,13 @@ int validate(const shred_params *p, shred_ctx *ctx) {
 // the low word, the '==' marker with any D = d 2^s (s < 32) by the divisibility test on the
 // full state (MK_DIV), and every other D by the remainder itself (MK_REM).  u64 state: deg 33..63 (top byte by mulhi, or a funnel shift for k <= 40);
 // u32 state: deg 9..32, and 8 (its top byte is the whole state: the PRMT byte index of
-// MODE_K32B).  Windows > 64: the generic loop.
+// MODE_K32B).  Windows 65..LW_MAX: the same kernel with the pops from a second TMA tile (WCH = 0
+// instances, "long windows"); longer ones: the generic loop.
+constexpr uint32_t LW_MAX = 4096;   // longest window of the hot kernel (16 ceil(w/16) <= GS * NTC)
 int select_path(const shred_params *p, int *mk) {
     const int k = deg64(p->poly);
     const bool pow2 = (p->divisor & (p->divisor - 1)) == 0;
-    const bool fast_w = p->window >= 1 && p->window <= 64;
+    const bool fast_w = p->window >= 1 && p->window <= LW_MAX;
     if (pow2 && p->divisor <= (1ull << 32)) *mk = p->marker == SHRED_MARKER_LE ? MK_LE : MK_EQ;
     else if (p->marker == SHRED_MARKER_EQ && __builtin_ctzll(p->divisor) < 32) *mk = MK_DIV;
     else *mk = MK_REM;
@@ -296,6 +299,7 @@ struct Plan {
     uint32_t nslots = 0;
     uint32_t bulk_ctas = 0;
     CUtensorMap tmap;
+    CUtensorMap tmap_pop;                // long windows: the pop tiles (16 ceil(w/16) bytes behind)
 };
 
 // The pure part of planning (no device state; shred_debug_plan exposes it to CPU tests): the
@@ -408,7 +412,7 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
     SlotMap &m = J.map;
     const MapShape sh{ctx->path == SHRED_PATH_K63 || ctx->path == SHRED_PATH_K32, ctx->path == SHRED_PATH_K63,
                       ctx->k1_small_fn != nullptr, ctx->sm_count, 16u * ((ctx->p.window + 15u) / 16u),
-                      prefix_len == 0};
+                      prefix_len == 0 && ctx->p.window <= 64};   // long windows: pop tiles stay inside src
     const uint64_t S = plan_map(sh, (uint64_t)(uintptr_t)src, p_begin, t_begin, t_end, m, pl.bulk, pl.small);
     if (pl.bulk) {
         const uint64_t ROUND = CfgK63::ROUND;
@@ -436,6 +440,17 @@ int plan_job(shred_ctx *ctx, Plan &pl, const uint8_t *src, uint64_t p_begin, con
             ctx->tm_cache = pl.tmap;
             memcpy(ctx->tm_key, key, sizeof key);
             ctx->tm_valid = true;
+        }
+        if (ctx->p.window > 64) {
+            // long windows: rows of the same geometry 16 ceil(w/16) bytes earlier (the plan keeps
+            // b0 - 16 ceil(w/16) >= p_begin), 48-byte boxes (two pop chunks + the funnel's next)
+            const uint64_t back = 16ull * ((ctx->p.window + 15u) / 16u);
+            cuuint32_t pbox[2] = {(cuuint32_t)LW_POPW, box[1]};
+            CUresult r = ctx->encode(&pl.tmap_pop, CU_TENSOR_MAP_DATA_TYPE_UINT8, 2,
+                                     (void *)(src + (m.b0 - back - p_begin)), gdim, gstride, pbox, estr,
+                                     CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE,
+                                     (CUtensorMapL2promotion)SHRED_L2PROMO, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+            if (r != CUDA_SUCCESS) return fail(ctx, SHRED_ECUDA, "cuTensorMapEncodeTiled (pops) failed (%d)", (int)r);
         }
     }
     pl.nslots = m.n_head + m.nrows + m.n_tail;
@@ -479,6 +494,7 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
                                             : (ctx->k >= 9 ? (1u << (40 - ctx->k)) : 0u);   // deg 8: byte index
         const uint32_t e = (uint32_t)(16 * ((ctx->p.window + 15) / 16) - ctx->p.window);
         K.fu = e / 4;
+        K.wa = (uint32_t)((ctx->p.window + 15) / 16);
         K.fsel = 0x3210u + 0x1111u * (e % 4);
         K.m256 = 256u;
         K.tmul = 1u << m;                                           // 2^(32 - log2 D)
@@ -504,11 +520,12 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
         }
         K.tsel = 0x5504u | ((uint32_t)((ctx->k - 8) / 8) << 4);         // byte (k-8)/8 -> bits 8..15
         K.pos = ctx->d_pos; K.w = ctx->p.window;
-        int smem = ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM;
+        int smem = ctx->k1_smem;
         int threads = (ctx->path == SHRED_PATH_K63 ? CfgK63::NTC : CfgK32::NTC) + 32;
         K1Fn fn = ctx->k1_fn;
         if (pl.small) { smem = CfgSmall::SMEM; threads = CfgSmall::NTC + 32; fn = ctx->k1_small_fn; }
-        PDL(fn, pl.bulk_ctas, threads, smem, st, pl.tmap, ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
+        PDL(fn, pl.bulk_ctas, threads, smem, st, pl.tmap, ctx->p.window > 64 ? pl.tmap_pop : pl.tmap,
+            ctx->d_tab_img, ctx->d_gen, pl.J, ctx->dp, K);
         LAUNCHED("k1_bulk");
         if (e1) CK(cudaEventRecord(e1, st), "profile record");
     } else {
@@ -771,16 +788,17 @@ int shred_init(const shred_params *p, int device, shred_ctx **out) {
             return bail(SHRED_ECUDA);
         ctx->encode = (EncodeTiledFn)fn;
         const bool byteidx = SHRED_BYTEIDX && ctx->path == SHRED_PATH_K32 && (k == 8 || k == 16 || k == 24 || k == 32);
-        const int wch = (int)((p->window + 15) / 16);
+        const int wch = p->window <= 64 ? (int)((p->window + 15) / 16) : 0;   // 0: long window
         const bool funnel = p->window % 16 != 0;
         const bool tprod = SHRED_TPROD && (ctx->path == SHRED_PATH_K32 || k >= 41) && tprod_ok(p->poly, k, nullptr);
         ctx->k1_fn = pick_k1(k, byteidx, wch, ctx->mk, funnel, tprod);
         const bool tmode = tprod && (ctx->mk == MK_EQ || ctx->mk == MK_LE);
         ctx->mode = ctx->path == SHRED_PATH_K63 ? (k >= 41 ? (tmode ? MODE_K63T : MODE_K63) : MODE_K40)
                   : tmode ? MODE_K32T : (byteidx ? MODE_K32B : MODE_K32);
+        ctx->k1_smem = ctx->path == SHRED_PATH_K63 ? (wch ? CfgK63::SMEM : LwLayout<CfgK63>::SMEM)
+                                                   : (wch ? CfgK32::SMEM : LwLayout<CfgK32>::SMEM);
         if (!ctx->k1_fn ||
-            cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                 ctx->path == SHRED_PATH_K63 ? CfgK63::SMEM : CfgK32::SMEM) != cudaSuccess)
+            cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributeMaxDynamicSharedMemorySize, ctx->k1_smem) != cudaSuccess)
             return bail(SHRED_ECUDA);
 #ifdef SHRED_CARVEOUT   // A/B only: force the L1/SMEM split of the hot kernel (percent of max smem)
         cudaFuncSetAttribute(ctx->k1_fn, cudaFuncAttributePreferredSharedMemoryCarveout, SHRED_CARVEOUT);
@@ -1263,7 +1281,7 @@ int shred_check_params(const shred_params *p, int *path_out, int *marker_kind_ou
 int shred_debug_plan(int path, int small_ok, int sm_count, uint64_t src_addr, uint64_t p_begin,
                      uint64_t t_begin, uint64_t t_end, uint64_t divisor, uint32_t window, int zero_lead,
                      uint64_t out[16]) {
-    if (!out || t_end < t_begin || t_begin < p_begin || sm_count < 1 || divisor < 2 || window < 1 || window > 64)
+    if (!out || t_end < t_begin || t_begin < p_begin || sm_count < 1 || divisor < 2 || window < 1 || window > LW_MAX)
         return SHRED_EINVAL;
     const MapShape sh{path == SHRED_PATH_K63 || path == SHRED_PATH_K32, path == SHRED_PATH_K63, small_ok != 0,
                       sm_count, 16u * ((window + 15u) / 16u), zero_lead != 0};

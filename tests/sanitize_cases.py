@@ -37,7 +37,8 @@ def main():
     check(pkg.Chunker(pkg.Params(min_size=3)), synthgen.periodic(b"\x04\xd5", 100000))
     check(pkg.Chunker(pkg.Params(divisor=10000, magic=1234)), data, 5)          # MK_DIV
     check(pkg.Chunker(pkg.Params(window=47, divisor=4096, magic=9, marker=1)), data[:300000], 2)   # funnel, '<='
-    check(pkg.Chunker(pkg.Params(window=65)), data[:100000])                       # generic
+    check(pkg.Chunker(pkg.Params(window=65)), data[:100000])                       # long window
+    check(pkg.Chunker(pkg.Params(window=200, marker=1, magic=3, divisor=1024)), data[:300000], 3)   # long window '<=', funnel
     check(pkg.Chunker(pkg.Params(divisor=12345, magic=3, marker=1)), data[:400000], 7)   # MK_REM, u64
     check(pkg.Chunker(pkg.Params(divisor=3 << 32, magic=77)), data[:300000], 1)          # MK_REM '=='
     check(pkg.Chunker(pkg.Params(poly=0x104C11DB7, divisor=1000, magic=2, marker=1)), data[:300000])  # MK_REM, u32

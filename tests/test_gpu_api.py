@@ -107,7 +107,8 @@ def test_init_validation_and_paths(pkg):
     assert pkg.Chunker(pkg.Params(poly=0x104C11DB7)).path == "k32"
     assert pkg.Chunker(pkg.Params(window=47)).path == "k63"
     assert pkg.Chunker(pkg.Params(window=47, marker=1)).path == "k63"
-    assert pkg.Chunker(pkg.Params(window=65)).path == "generic"
+    assert pkg.Chunker(pkg.Params(window=65)).path == "k63"                       # long window
+    assert pkg.Chunker(pkg.Params(window=4096)).path == "k63"
     ch = pkg.Chunker(pkg.Params(min_size=100))
     assert ch.max_cuts(1001) == 1000 // 100 + 1
     got = pkg._binding._Params()

@@ -6,11 +6,11 @@ Each case draws (from one fixed seed, so the ids are stable and a failure reprod
   (K32T x^31+x^13+1, K63T x^63+x^11+1), 0x104C11DB7 (K32B), x^31+x^3+1 (K32, T table),
   x^8+x^4+x^3+x^2+1 (degree 8), or a dense random irreducible of degree 9..63 (L255-L258: "an
   irreducible polynomial div(x) of degree k", k left open);
-* w in 1..64 (hot kernel, every pop shape) or 65..200 (generic loop);
+* w in 1..64 (hot kernel, register pops) or 65..200 (hot kernel, pops from a second TMA tile);
 * D = 2^m ('==' and '<=', L447-L451 / L249-L251) or any other D (remainder kernels, reading Q8);
 * r < D; min/max bounds on or off (the size rule of §8(c), L259-L265);
 * the input: SplitMix64 bytes, text-like words, a short periodic pattern, or zeros;
-  length 0..3.5 MiB (the generic loop's cases stay below 400 KiB), base offset 0..15;
+  length 0..3.5 MiB (windows > 64 below 400 KiB), base offset 0..15;
 * the call: one-shot `shred_chunk`; `shred_feed` in random pieces (pinned host or device, ring of
   2-3 slots) + `shred_flush`; or G = 2..5 byte-range shards (`shred_candidates_range` with the
   min(w-1, start) halo) concatenated, then the global size rule (`shred_size_bound`).

@@ -2,7 +2,7 @@
 
 Bar: bit-exact (integer work).  Sizes span several tiles/rows and ragged tails; edge cases are
 empty/short inputs, unaligned bases, adversarial candidate density (list overflow + re-roll),
-all-zero / all-0xFF, and every kernel path (k63, k32, generic).
+all-zero / all-0xFF, and every kernel path (k63, k32, long windows, generic).
 """
 import numpy as np
 import pytest
@@ -114,14 +114,21 @@ def test_launch_shapes_around_small_threshold(pkg, poly, n):
         check_chunk(pkg.Chunker(p), data)
 
 
-def test_generic_path_variants(pkg):
+def test_long_window_variants(pkg):
+    """Windows > 64 on the hot kernel (pops from the second TMA tile, 16 ceil(w/16) bytes behind),
+    every marker kind and state mode; inputs below 4 KiB take the generic loop."""
     for p in (pkg.Params(window=65), pkg.Params(window=80, divisor=256, magic=7, marker=1),
               pkg.Params(poly=0x11D, window=70, divisor=128, magic=5, marker=1),
               pkg.Params(window=100, divisor=3000, magic=2999, marker=1),
-              pkg.Params(window=65, divisor=1 << 40, magic=12345)):
+              pkg.Params(window=65, divisor=1 << 40, magic=12345),
+              pkg.Params(poly=0x80002001, window=96), pkg.Params(poly=0x104C11DB7, window=129, divisor=512),
+              pkg.Params(poly=0x8000000000000801, window=255, divisor=1024, magic=3),
+              pkg.Params(window=4096, divisor=256), pkg.Params(window=1000, min_size=512, max_size=4096)):
         ch = pkg.Chunker(p)
-        assert ch.path == "generic"
+        assert ch.path in ("k63", "k32")
         check_chunk(ch, synthgen.random_bytes(11, 300000))
+        check_chunk(ch, synthgen.random_bytes(12, (3 << 20) + 77), offset=5)
+        check_chunk(ch, synthgen.random_bytes(13, 3000))                       # generic loop
     # the '<=' marker with any window <= 64 runs on the hot kernel (funnel-shifted pops)
     for p in (pkg.Params(window=1, divisor=256, magic=7, marker=1),
               pkg.Params(poly=(1 << 63) | 3, window=24, divisor=1024, marker=1)):

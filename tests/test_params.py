@@ -71,11 +71,11 @@ def test_parameter_ranges(check):
     (dict(), K63, MK_EQ),                                                # the paper's reading
     (dict(marker=1, magic=3), K63, MK_LE),
     (dict(window=47), K63, MK_EQ), (dict(window=64), K63, MK_EQ), (dict(window=1), K63, MK_EQ),
-    (dict(window=65), GENERIC, MK_EQ), (dict(window=47, marker=1, magic=1), K63, MK_LE),
+    (dict(window=65), K63, MK_EQ), (dict(window=4096), K63, MK_EQ), (dict(window=47, marker=1, magic=1), K63, MK_LE),
     (dict(divisor=10000, magic=7), K63, MK_DIV), (dict(divisor=3 << 31, magic=7), K63, MK_DIV),
     (dict(divisor=1 << 32, magic=7), K63, MK_EQ), (dict(divisor=1 << 33, magic=7), K63, MK_REM),
     (dict(divisor=3 << 32, magic=7), K63, MK_REM), (dict(divisor=10000, magic=7, marker=1), K63, MK_REM),
-    (dict(divisor=1 << 40, magic=7, marker=1), K63, MK_REM), (dict(window=65, divisor=10000, magic=7, marker=1), GENERIC, MK_REM),
+    (dict(divisor=1 << 40, magic=7, marker=1), K63, MK_REM), (dict(window=65, divisor=10000, magic=7, marker=1), K63, MK_REM),
     (dict(poly=0x104C11DB7, divisor=1000, magic=999, marker=1), K32, MK_REM),
     (dict(poly=0x104C11DB7), K32, MK_EQ), (dict(poly=0x104C11DB7, divisor=10000, magic=3), K32, MK_DIV),
     (dict(poly=0x11D, divisor=64, magic=1), K32, MK_EQ),                         # degree 8: byte index

@@ -101,8 +101,10 @@ def test_plan_tiles_every_window_end_once(L, path):
             t_begin = p_begin + int(rng.integers(0, 200))
             sms = int(rng.choice([1, 2, 132, 148, 160]))
             small_ok = int(rng.integers(0, 2))
-            window = int(rng.choice([1, 16, 17, 47, 48, 64]))
-            zl = int(rng.integers(0, 2))
+            window = int(rng.choice([1, 16, 17, 47, 48, 64, 65, 100, 4096]))
+            zl = int(rng.integers(0, 2)) if window <= 64 else 0      # long windows: never a zero lead
+            if window > 64:
+                small_ok = 0                                          # no small shape for them
             if zl and rng.integers(0, 2):
                 t_begin = p_begin
             m = plan(L, path, small_ok, sms, addr, p_begin, t_begin, t_begin + n, window=window, zero_lead=zl)
@@ -134,4 +136,5 @@ def test_plan_rejects_inconsistent_arguments(L):
     assert L.shred_debug_plan(K63, 1, 148, 0, 100, 50, 1000, 8192, 48, 0, out) != 0   # t_begin < p_begin
     assert L.shred_debug_plan(K63, 1, 148, 0, 0, 10, 5, 8192, 48, 0, out) != 0        # t_end < t_begin
     assert L.shred_debug_plan(K63, 1, 0, 0, 0, 0, 5, 8192, 48, 0, out) != 0           # no SMs
-    assert L.shred_debug_plan(K63, 1, 148, 0, 0, 0, 5, 8192, 65, 0, out) != 0         # w > 64
+    assert L.shred_debug_plan(K63, 1, 148, 0, 0, 0, 5, 8192, 4097, 0, out) != 0       # w > 4096
+    assert L.shred_debug_plan(K63, 1, 148, 0, 0, 0, 5, 8192, 4096, 0, out) == 0       # long window
