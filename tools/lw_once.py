@@ -1,0 +1,19 @@
+"""One 1 GiB call with a long window (w = 128 by default, paper polynomial): for ncu."""
+import os
+import sys
+
+import torch
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+import paper_conf_fast_bhatotiarv12_b200 as pkg  # noqa: E402
+
+w = int(sys.argv[1]) if len(sys.argv) > 1 else 128
+x = torch.empty(1 << 30, dtype=torch.uint8, device="cuda")
+pkg.synth_fill(x, 2)
+ch = pkg.Chunker(pkg.Params(window=w))
+out = torch.empty((1 << 30) // 512, dtype=torch.int64, device="cuda")
+n = torch.zeros(1, dtype=torch.int64, device="cuda")
+for _ in range(3):
+    ch.chunk_async(x, out, n)
+torch.cuda.synchronize()
+print(int(n.item()))
