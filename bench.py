@@ -723,6 +723,16 @@ def main():
                                     "params": "P=x^63+x^11+1 (0x8000000000000801, irreducible trinomial), other params as paper",
                                     "mode": c6t.mode}
             del c6t
+            # long windows (w > 64): the hot kernel with the pops from a second TMA tile
+            lw = {}
+            for wv in (128, 1000):
+                clw = pkg.Chunker(pkg.Params(window=wv), device=local)
+                lw[f"w{wv}"] = round(timed(clw, base), 2)
+                del clw
+            line["long_window_variant"] = {"value": lw["w128"], "unit": "GB/s", "w1000": lw["w1000"],
+                                           "params": "w = 128 (and 1000), other params as paper",
+                                           "note": "windows 65-4096 on k1_bulk: pops from a second TMA tile "
+                                                   "(DESIGN.md §5 Long windows)"}
             # content sensitivity. Text-like bytes (words from a fixed
             # 1,000-word list; skewed outgoing bytes for the U lookups), 64 MiB generated on the
             # host and tiled to 256 MiB on the device; paper params on the same ctx.

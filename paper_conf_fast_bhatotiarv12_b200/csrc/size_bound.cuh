@@ -29,6 +29,10 @@
 namespace shred {
 
 #ifndef SHRED_SB_B
+// 16: a block fails to sync only if none of its candidates is accepted from both its guessed and
+// its true entry (~0.22^16 per block at min = D/4); one unsynced block sends the whole list to the
+// serial walk.  A/B (profiles/r02_ab_small_bounded.txt): 8 gained ~1 % on 1 GiB bounded but makes
+// that walk likely on GiB lists (~0.22^8 x 16 K blocks); 4 fell to 103 GB/s (the walk, every call).
 #define SHRED_SB_B 16
 #endif
 constexpr int SB_B = SHRED_SB_B;    // candidates per block (one thread; prefetched into registers)
@@ -411,8 +415,9 @@ sb_dense(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots, 
 //   emit  block b reruns from its true entry and writes its cuts; the last thread writes the
 //         forced cuts after the last candidate.
 // Larger counts run the global-memory phases above (sb_*_body); dense lists sb_dense_body.
-constexpr int SBO_THREADS = 512;
-constexpr uint32_t SBO_SMEM_N = SBO_THREADS * SB_B;       // 8192 candidates, 64 KiB
+constexpr int SBO_THREADS = 1024;
+constexpr int SBO_B = 8;      // candidates per block in sb_one_smem (its serial walk is over <= 1,024 blocks in smem)
+constexpr uint32_t SBO_SMEM_N = SBO_THREADS * SBO_B;      // 8192 candidates, 64 KiB
 constexpr size_t SBO_SMEM = (size_t)SBO_SMEM_N * 8 + (size_t)SBO_THREADS * 8 * 4;
 #ifndef SHRED_SB_ONE_MAX
 #define SHRED_SB_ONE_MAX (256ull << 20)  // A/B: 0 = always the multi-CTA chain
@@ -434,16 +439,16 @@ __device__ __forceinline__ void sb_one_smem(const SBArgs &A, uint32_t n, uint64_
     if (!loaded)
         for (uint32_t i = tid; i < n; i += SBO_THREADS) sc[i] = A.cand[i];
     __syncthreads();
-    const uint32_t nb = (n + SB_B - 1) / SB_B;
+    const uint32_t nb = (n + SBO_B - 1) / SBO_B;
     const uint32_t b = tid;
     int h0 = 0;
     uint64_t cnt = 0;
     bool synced = true;
     if (b < nb) {
-        const uint32_t first = b * SB_B, last = min(n, first + SB_B);
+        const uint32_t first = b * SBO_B, last = min(n, first + SBO_B);
         uint64_t X = 0;
         if (b) {
-            const uint32_t pf = first - SB_B;
+            const uint32_t pf = first - SBO_B;
             X = (b - 1) ? sc[pf - 1] : 0ull;
             for (uint32_t j = pf; j < first; ++j) sb_step(X, sc[j], A, h0, NoEmit{});
         }
@@ -493,7 +498,7 @@ __device__ __forceinline__ void sb_one_smem(const SBArgs &A, uint32_t n, uint64_
                 off += cn[k];
                 s = ex[k];
             } else {
-                const uint32_t first = k * SB_B, last = min(n, first + SB_B);
+                const uint32_t first = k * SBO_B, last = min(n, first + SBO_B);
                 for (uint32_t j = first; j < last; ++j) off += sb_step(s, sc[j], A, h, NoEmit{});
             }
         }
@@ -513,7 +518,7 @@ __device__ __forceinline__ void sb_one_smem(const SBArgs &A, uint32_t n, uint64_
             *n_out = o;
             if (o > cap) aux->overflow = 1;
         } else {
-            const uint32_t first = b * SB_B, last = min(n, first + SB_B);
+            const uint32_t first = b * SBO_B, last = min(n, first + SBO_B);
             int h = 0;
             for (uint32_t j = first; j < last; ++j) sb_step(s, sc[j], A, h, emit);
         }
@@ -526,7 +531,7 @@ sb_one(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots, SB
     pdl_entry();
     Aux *aux = A.aux;
     const uint64_t dense = aux->dense, n = sb_n(A);
-    if (!dense && n <= SBO_SMEM_N - SB_B) {                // nb < SBO_THREADS: thread nb writes the tail
+    if (!dense && n <= SBO_SMEM_N - SBO_B) {                // nb < SBO_THREADS: thread nb writes the tail
         sb_one_smem(A, (uint32_t)n, n_out, cap);
         return;
     }
