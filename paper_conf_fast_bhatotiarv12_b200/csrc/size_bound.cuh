@@ -29,10 +29,12 @@
 namespace shred {
 
 #ifndef SHRED_SB_B
-// 16: a block fails to sync only if none of its candidates is accepted from both its guessed and
-// its true entry (~0.22^16 per block at min = D/4); one unsynced block sends the whole list to the
-// serial walk.  A/B (profiles/r02_ab_small_bounded.txt): 8 gained ~1 % on 1 GiB bounded but makes
-// that walk likely on GiB lists (~0.22^8 x 16 K blocks); 4 fell to 103 GB/s (the walk, every call).
+// 16: a block syncs at its first candidate c >= g + min (g = its guessed entry; accepted from the
+// true entry s <= g too), so it fails only if all B candidates lie within min of g: P(Poisson(min/D)
+// >= B) for random data, and one unsynced block sends the whole list to the serial walk.  B = 16
+// keeps that negligible up to min ~ 3D on GiB lists; A/B (profiles/r02_ab_small_bounded.txt): 8
+// gained ~1 % at min = D/4 but walks on ~15 % of GiB lists at min = D; 4 walked on every call
+// at min = D/4 (103 GB/s).
 #define SHRED_SB_B 16
 #endif
 constexpr int SB_B = SHRED_SB_B;    // candidates per block (one thread; prefetched into registers)
