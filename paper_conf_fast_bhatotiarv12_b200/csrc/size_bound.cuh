@@ -222,31 +222,75 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
         }
         return;
     }
-    if (tid >= 32) return;
     // ---- sequential fallback (some block never synced with its speculation): exact.  Warp 0
     // walks the blocks in order; a block whose assumed entry holds uses its (spec + delta)
-    // count, any other block is re-walked with its 32 candidates loaded one per lane.
+    // count, any other block is re-walked by ballot: the first candidate (in order) that forces
+    // a cut or is accepted from the current state is the next one that changes it, and every
+    // candidate before it drops out with no effect -- one step per cut, not per candidate.  The
+    // other warps stage the next window of candidates and spec results in shared memory
+    // (double-buffered) while warp 0 walks the current one.  1 GiB, min >> D (blocks rarely
+    // re-sync): min = 8D 13.8 -> see profiles/r02_ab_small_bounded.txt.
+    constexpr uint32_t SBW = 2048, SBWB = SBW / SB_B;        // candidates / blocks per window
+    __shared__ uint64_t wc[2][SBW];
+    __shared__ uint64_t wx[2][SBWB + 1];                    // spec exits of blocks b0 - 1 .. b0 + SBWB - 1
+    __shared__ uint64_t wn[2][SBWB];                        // spec count + delta
+    __shared__ uint32_t wo[2][SBWB];                        // synced
+    const uint32_t nwin = (nb + SBWB - 1) / SBWB;
+    auto stage = [&](uint32_t wi, int buf, uint32_t t, uint32_t nt) {
+        const uint64_t c0 = (uint64_t)wi * SBW;
+        const uint32_t b0 = wi * SBWB;
+        for (uint32_t i = t; i < SBW; i += nt)
+            if (c0 + i < n) wc[buf][i] = A.cand[c0 + i];
+        for (uint32_t i = t; i <= SBWB; i += nt) {
+            const int64_t bb = (int64_t)b0 + (int64_t)i - 1;
+            wx[buf][i] = (bb >= 0 && bb < (int64_t)nb) ? A.spec_exit[bb] : 0ull;
+        }
+        for (uint32_t i = t; i < SBWB; i += nt)
+            if (b0 + i < nb) {
+                wn[buf][i] = (uint64_t)((int64_t)A.spec_cnt[b0 + i] + A.delta[b0 + i]);
+                wo[buf][i] = A.ok[b0 + i];
+            }
+    };
+    if (nwin) stage(0, 0, tid, blockDim.x);
+    __syncthreads();
     const uint32_t lane = tid;
     uint64_t s = aux->s, off = base0;
     int held = 0;
-    for (uint32_t b = 0; b < nb; ++b) {
-        const uint64_t first = (uint64_t)b * SB_B, last = min(n, first + SB_B);
-        if (lane == 0) { A.entry[b] = s; A.offs[b] = off; }
-        if (b == 0 || (A.ok[b] && s == A.spec_exit[b - 1])) {
-            off += (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]);
-            s = A.spec_exit[b];
-            held = (!A.fin && last == n && A.cand[n - 1] == A.end && s == A.end) ? 1 : 0;
+    for (uint32_t wi = 0; wi < nwin; ++wi) {
+        const int cur = (int)(wi & 1u);
+        if (tid >= 32) {
+            if (wi + 1 < nwin) stage(wi + 1, cur ^ 1, tid - 32, blockDim.x - 32);
         } else {
-            held = 0;
-            const uint64_t mine = (first + lane < last) ? A.cand[first + lane] : 0ull;
-            const int m = (int)(last - first);
-            for (int j = 0; j < m; ++j) {
-                const uint64_t c = __shfl_sync(0xffffffffu, mine, j);
-                off += sb_step(s, c, A, held, NoEmit{});
+            const uint32_t b0 = wi * SBWB, mb = min(SBWB, nb - b0);
+            const uint64_t c0 = (uint64_t)wi * SBW;
+            for (uint32_t j = 0; j < mb; ++j) {
+                const uint32_t b = b0 + j;
+                const uint64_t first = (uint64_t)b * SB_B, last = min(n, first + SB_B);
+                if (lane == 0) { A.entry[b] = s; A.offs[b] = off; }
+                if (b == 0 || (wo[cur][j] && s == wx[cur][j])) {
+                    off += wn[cur][j];
+                    s = wx[cur][j + 1];
+                    held = (!A.fin && last == n && A.cand[n - 1] == A.end && s == A.end) ? 1 : 0;
+                } else {
+                    held = 0;
+                    const uint32_t m = (uint32_t)(last - first);
+                    const uint64_t mine = lane < m ? wc[cur][first - c0 + lane] : 0ull;
+                    uint32_t from = 0;
+                    for (;;) {
+                        const bool ev = lane >= from && lane < m &&
+                                        ((A.maxsz && mine - s > A.maxsz) || mine - s >= A.minsz);
+                        const uint32_t bal = __ballot_sync(0xffffffffu, ev);
+                        if (!bal) break;
+                        const int jj = __ffs(bal) - 1;
+                        off += sb_step(s, __shfl_sync(0xffffffffu, mine, jj), A, held, NoEmit{});
+                        from = (uint32_t)jj + 1;
+                    }
+                }
             }
         }
+        __syncthreads();
     }
-    if (lane != 0) return;
+    if (tid != 0) return;
     aux->sb_fast = 0;
     const uint64_t mt = sb_tail_count(s, A);
     if (held_prev && aux->out_pos < A.dst_cap) A.dst[aux->out_pos] = aux->held_val;

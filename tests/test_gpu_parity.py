@@ -646,3 +646,12 @@ def test_bounded_one_shot_one_cta_paths(pkg, kind):
         assert oracle.candidates(data, oparams(p)).size > 8176
     if kind != "short":
         assert got.size > 0
+
+
+@pytest.mark.parametrize("mn,mx", [(8192, 65536), (65536, 0), (131072, 262144), (40000, 40001)])
+def test_bounded_min_above_d_serial_walk(pkg, mn, mx):
+    """min >= D: blocks of 16 candidates rarely re-sync with their speculation, so the size rule
+    takes its exact serial walk (batched block results, ballot re-walks); equal to the oracle
+    (L259-L265) on 64 MiB of random data, with and without forced cuts."""
+    data = synthgen.random_bytes(91, (64 << 20) + 333)
+    check_chunk(pkg.Chunker(pkg.Params(min_size=mn, max_size=mx)), data)
