@@ -222,6 +222,85 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
         }
         return;
     }
+    // ---- parallel repair (some block did not sync with its speculation): Jacobi passes over
+    // the blocks, block b re-run from the exit of block b-1 as currently known, until no exit
+    // changes (exact at the fixed point: every block then ran from its true entry).  A block
+    // whose speculation failed usually changes only the next block or two (min ~ D: 2-3
+    // passes); long chains of unsynced blocks (min >> D) leave it to the serial walk below.
+    {
+        uint64_t *Ea = A.entry, *Eb = A.cta_sum, *Cn = A.cta_ok, *Used = A.offs;   // scratch
+        const uint32_t T = blockDim.x, pb = (nb + T - 1) / T;
+        const uint32_t ba = min(nb, tid * pb), bb = min(nb, ba + pb);
+        for (uint32_t b = ba; b < bb; ++b) { Ea[b] = A.spec_exit[b]; Used[b] = ~0ull; }
+        __syncthreads();
+        constexpr int PASSES = 12;
+        int conv = 0, p = 0;
+        for (; p < PASSES && !conv; ++p) {
+            const uint64_t *src = (p & 1) ? Eb : Ea;
+            uint64_t *dst = (p & 1) ? Ea : Eb;
+            int changed = 0;
+            for (uint32_t b = ba; b < bb; ++b) {
+                const uint64_t e = b ? src[b - 1] : aux->s;
+                if (e != Used[b]) {
+                    const uint64_t first = (uint64_t)b * SB_B, last = min(n, first + SB_B);
+                    uint64_t x = e, cnt = 0;
+                    int h = 0;
+                    for (uint64_t j = first; j < last; ++j) cnt += sb_step(x, A.cand[j], A, h, NoEmit{});
+                    Used[b] = e;
+                    Cn[b] = cnt;
+                    changed |= (x != src[b]) ? 1 : 0;
+                    dst[b] = x;
+                } else {
+                    dst[b] = src[b];
+                }
+            }
+            conv = !__syncthreads_or(changed);
+        }
+        if (conv) {
+            const uint64_t *E = (p & 1) ? Eb : Ea;          // the last pass's output
+            const uint64_t s_last = nb ? E[nb - 1] : aux->s;  // read before entry (= Ea) is rewritten
+            // offsets: exclusive scan of the block counts (contiguous ranges per thread)
+            uint64_t rs = 0;
+            for (uint32_t b = ba; b < bb; ++b) rs += Cn[b];
+            uint64_t incl = rs;
+            for (int d = 1; d < 32; d <<= 1) {
+                const uint64_t u = __shfl_up_sync(0xffffffffu, incl, d);
+                if ((tid & 31) >= (uint32_t)d) incl += u;
+            }
+            if ((tid & 31) == 31) wsum[tid >> 5] = incl;
+            __syncthreads();
+            if (tid == 0) {
+                uint64_t r = 0;
+                for (uint32_t w = 0; w < (T >> 5); ++w) { const uint64_t x = wsum[w]; wsum[w] = r; r += x; }
+                wsum[32] = r;
+            }
+            __syncthreads();
+            uint64_t o = base0 + wsum[tid >> 5] + incl - rs;
+            for (uint32_t b = ba; b < bb; ++b) {              // entries: Used[b] (the entry of the last run)
+                const uint64_t e = Used[b];
+                A.offs[b] = o;                                 // (Used aliases offs: read first)
+                A.entry[b] = e;
+                o += Cn[b];
+            }
+            __syncthreads();
+            if (tid == 0) {
+                const uint64_t carry = wsum[32];
+                const int held_new = (!A.fin && n > 0 && A.cand[n - 1] == A.end && s_last == A.end) ? 1 : 0;
+                const uint64_t mt = sb_tail_count(s_last, A);
+                aux->sb_fast = 0;
+                if (held_prev && aux->out_pos < A.dst_cap) A.dst[aux->out_pos] = aux->held_val;
+                A.offs[nb] = base0 + carry;
+                A.entry[nb] = s_last;
+                aux->total = carry + mt;
+                aux->out_pos = base0 + carry + mt;
+                aux->s = s_last + mt * A.maxsz;
+                aux->held = (uint64_t)held_new;
+                aux->held_val = held_new ? A.end : 0;
+            }
+            return;
+        }
+        __syncthreads();
+    }
     // ---- sequential fallback (some block never synced with its speculation): exact.  Warp 0
     // walks the blocks in order; a block whose assumed entry holds uses its (spec + delta)
     // count, any other block is re-walked by ballot: the first candidate (in order) that forces
