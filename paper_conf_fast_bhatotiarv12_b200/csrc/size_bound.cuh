@@ -223,116 +223,118 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
         return;
     }
     // ---- parallel repair (some block did not sync with its speculation): Jacobi passes over
-    // the blocks, block b re-run from the exit of block b-1 as currently known, until no exit
-    // changes (exact at the fixed point: every block then ran from its true entry).  A block
-    // whose speculation failed usually changes only the next block or two (min ~ D: 2-3
-    // passes); long chains of unsynced blocks (min >> D) leave it to the serial walk below.
-    {
+    // super-blocks of G blocks, each re-run from the exit of the previous one as currently known
+    // (only when that entry changed), until no exit changes -- exact at the fixed point, where
+    // every super-block ran from its true entry.  A block whose speculation failed usually
+    // changes only the next block or two (min ~ D: converged at G = 1 in 2-3 passes).  Long
+    // chains of unsynced blocks (min >> D: a cut needs a gap >= min from the leading state) need
+    // super-blocks long enough to re-sync: G = 32 (min = 8D); beyond that the serial walk below.
+#ifndef SHRED_SB_REPAIR_LEVELS
+#define SHRED_SB_REPAIR_LEVELS 2      // G = 1, 32 (A/B: 0 = straight to the serial walk; 3 adds G = 1024,
+                                      // which cost more than the walk when it fails: min = 16D 4.1 -> 8.0 ms)
+#endif
+    for (int lvl = 0; lvl < SHRED_SB_REPAIR_LEVELS; ++lvl) {
+        const uint32_t G = lvl == 0 ? 1u : lvl == 1 ? 32u : 1024u;     // blocks per super-block
+        const uint32_t ns = (nb + G - 1) / G;                  // super-blocks
+        if (lvl > 0 && ns < 4) break;                           // no parallelism left: walk
         uint64_t *Ea = A.entry, *Eb = A.cta_sum, *Cn = A.cta_ok, *Used = A.offs;   // scratch
-        const uint32_t T = blockDim.x, pb = (nb + T - 1) / T;
-        const uint32_t ba = min(nb, tid * pb), bb = min(nb, ba + pb);
-        for (uint32_t b = ba; b < bb; ++b) { Ea[b] = A.spec_exit[b]; Used[b] = ~0ull; }
+        const uint32_t T = blockDim.x, ps = (ns + T - 1) / T;
+        const uint32_t sa = min(ns, tid * ps), se = min(ns, sa + ps);
+        for (uint32_t k = sa; k < se; ++k) { Ea[k] = A.spec_exit[min(nb, (k + 1) * G) - 1]; Used[k] = ~0ull; }
         __syncthreads();
-        constexpr int PASSES = 12;
+        const int passes = lvl == 0 ? 12 : lvl == 1 ? 6 : 3;   // a pass at G = 1024 costs ~0.35 ms
         int conv = 0, p = 0;
-        for (; p < PASSES && !conv; ++p) {
+        for (; p < passes && !conv; ++p) {
             const uint64_t *src = (p & 1) ? Eb : Ea;
             uint64_t *dst = (p & 1) ? Ea : Eb;
             int changed = 0;
-            for (uint32_t b = ba; b < bb; ++b) {
-                const uint64_t e = b ? src[b - 1] : aux->s;
-                if (e != Used[b]) {
-                    const uint64_t first = (uint64_t)b * SB_B, last = min(n, first + SB_B);
-                    uint64_t x = e, cnt = 0;
+            for (uint32_t k = sa; k < se; ++k) {
+                const uint64_t e = k ? src[k - 1] : aux->s;
+                if (e != Used[k]) {
+                    const uint64_t first = (uint64_t)k * G * SB_B, last = min(n, first + (uint64_t)G * SB_B);
+                    uint64_t x = e;
                     int h = 0;
-                    for (uint64_t j = first; j < last; ++j) cnt += sb_step(x, A.cand[j], A, h, NoEmit{});
-                    Used[b] = e;
-                    Cn[b] = cnt;
-                    changed |= (x != src[b]) ? 1 : 0;
-                    dst[b] = x;
+#pragma unroll 4
+                    for (uint64_t j = first; j < last; ++j) sb_step(x, A.cand[j], A, h, NoEmit{});
+                    Used[k] = e;
+                    changed |= (x != src[k]) ? 1 : 0;
+                    dst[k] = x;
                 } else {
-                    dst[b] = src[b];
+                    dst[k] = src[k];
                 }
             }
             conv = !__syncthreads_or(changed);
         }
-        if (conv) {
-            const uint64_t *E = (p & 1) ? Eb : Ea;          // the last pass's output
-            const uint64_t s_last = nb ? E[nb - 1] : aux->s;  // read before entry (= Ea) is rewritten
-            // offsets: exclusive scan of the block counts (contiguous ranges per thread)
-            uint64_t rs = 0;
-            for (uint32_t b = ba; b < bb; ++b) rs += Cn[b];
-            uint64_t incl = rs;
-            for (int d = 1; d < 32; d <<= 1) {
-                const uint64_t u = __shfl_up_sync(0xffffffffu, incl, d);
-                if ((tid & 31) >= (uint32_t)d) incl += u;
+        if (!conv) { __syncthreads(); continue; }
+        const uint64_t *E = (p & 1) ? Eb : Ea;                  // the last pass's output
+        const uint64_t s_last = ns ? E[ns - 1] : aux->s;
+        __syncthreads();                                        // E (= entry) is rewritten below
+        // every super-block from its true entry once more: per-block entries and counts
+        for (uint32_t k = sa; k < se; ++k) {
+            uint64_t x = Used[k];
+            int h = 0;
+            for (uint32_t b = k * G; b < min(nb, (k + 1) * G); ++b) {
+                const uint64_t first = (uint64_t)b * SB_B, last = min(n, first + SB_B);
+                A.entry[b] = x;
+                uint64_t cnt = 0;
+                for (uint64_t j = first; j < last; ++j) cnt += sb_step(x, A.cand[j], A, h, NoEmit{});
+                Cn[b] = cnt;
             }
-            if ((tid & 31) == 31) wsum[tid >> 5] = incl;
-            __syncthreads();
-            if (tid == 0) {
-                uint64_t r = 0;
-                for (uint32_t w = 0; w < (T >> 5); ++w) { const uint64_t x = wsum[w]; wsum[w] = r; r += x; }
-                wsum[32] = r;
-            }
-            __syncthreads();
-            uint64_t o = base0 + wsum[tid >> 5] + incl - rs;
-            for (uint32_t b = ba; b < bb; ++b) {              // entries: Used[b] (the entry of the last run)
-                const uint64_t e = Used[b];
-                A.offs[b] = o;                                 // (Used aliases offs: read first)
-                A.entry[b] = e;
-                o += Cn[b];
-            }
-            __syncthreads();
-            if (tid == 0) {
-                const uint64_t carry = wsum[32];
-                const int held_new = (!A.fin && n > 0 && A.cand[n - 1] == A.end && s_last == A.end) ? 1 : 0;
-                const uint64_t mt = sb_tail_count(s_last, A);
-                aux->sb_fast = 0;
-                if (held_prev && aux->out_pos < A.dst_cap) A.dst[aux->out_pos] = aux->held_val;
-                A.offs[nb] = base0 + carry;
-                A.entry[nb] = s_last;
-                aux->total = carry + mt;
-                aux->out_pos = base0 + carry + mt;
-                aux->s = s_last + mt * A.maxsz;
-                aux->held = (uint64_t)held_new;
-                aux->held_val = held_new ? A.end : 0;
-            }
-            return;
         }
         __syncthreads();
+        // offsets: exclusive scan of the block counts (contiguous ranges per thread)
+        const uint32_t pb = (nb + T - 1) / T, ba = min(nb, tid * pb), bb = min(nb, ba + pb);
+        uint64_t rs = 0;
+        for (uint32_t b = ba; b < bb; ++b) rs += Cn[b];
+        uint64_t incl = rs;
+        for (int d = 1; d < 32; d <<= 1) {
+            const uint64_t u = __shfl_up_sync(0xffffffffu, incl, d);
+            if ((tid & 31) >= (uint32_t)d) incl += u;
+        }
+        if ((tid & 31) == 31) wsum[tid >> 5] = incl;
+        __syncthreads();
+        if (tid == 0) {
+            uint64_t r = 0;
+            for (uint32_t w = 0; w < (T >> 5); ++w) { const uint64_t x = wsum[w]; wsum[w] = r; r += x; }
+            wsum[32] = r;
+        }
+        __syncthreads();
+        uint64_t o = base0 + wsum[tid >> 5] + incl - rs;
+        for (uint32_t b = ba; b < bb; ++b) { A.offs[b] = o; o += Cn[b]; }
+        if (tid == 0) {
+            const uint64_t carry = wsum[32];
+            const int held_new = (!A.fin && n > 0 && A.cand[n - 1] == A.end && s_last == A.end) ? 1 : 0;
+            const uint64_t mt = sb_tail_count(s_last, A);
+            aux->sb_fast = 0;
+            if (held_prev && aux->out_pos < A.dst_cap) A.dst[aux->out_pos] = aux->held_val;
+            A.offs[nb] = base0 + carry;
+            A.entry[nb] = s_last;
+            aux->total = carry + mt;
+            aux->out_pos = base0 + carry + mt;
+            aux->s = s_last + mt * A.maxsz;
+            aux->held = (uint64_t)held_new;
+            aux->held_val = held_new ? A.end : 0;
+        }
+        return;
     }
-    // ---- sequential fallback (some block never synced with its speculation): exact.  Warp 0
-    // walks the blocks in order; a block whose assumed entry holds uses its (spec + delta)
-    // count, any other block is re-walked by ballot: the first candidate (in order) that forces
-    // a cut or is accepted from the current state is the next one that changes it, and every
-    // candidate before it drops out with no effect -- one step per cut, not per candidate.  The
-    // other warps stage the next window of candidates and spec results in shared memory
-    // (double-buffered) while warp 0 walks the current one.  1 GiB, min >> D (blocks rarely
-    // re-sync): min = 8D 13.8 -> see profiles/r02_ab_small_bounded.txt.
-    constexpr uint32_t SBW = 2048, SBWB = SBW / SB_B;        // candidates / blocks per window
+    // ---- sequential fallback (no parallel form converged): exact.  Warp 0 runs the rule over
+    // every candidate in order, 32 at a time by ballot: the first candidate (in order) that
+    // forces a cut or is accepted from the current state is the next one that changes it, and
+    // every candidate before it drops out with no effect -- one ballot per 16 candidates plus one
+    // step per cut.  Block entries and offsets are recorded at the block boundaries.  The other
+    // warps stage the next window of candidates in shared memory (double-buffered).
+    static_assert(SB_B == 16, "the ballot walk records a block boundary every 16 candidates");
+    constexpr uint32_t SBW = 2048;                          // candidates per window
     __shared__ uint64_t wc[2][SBW];
-    __shared__ uint64_t wx[2][SBWB + 1];                    // spec exits of blocks b0 - 1 .. b0 + SBWB - 1
-    __shared__ uint64_t wn[2][SBWB];                        // spec count + delta
-    __shared__ uint32_t wo[2][SBWB];                        // synced
-    const uint32_t nwin = (nb + SBWB - 1) / SBWB;
+    const uint32_t nwin = (uint32_t)((n + SBW - 1) / SBW);
     auto stage = [&](uint32_t wi, int buf, uint32_t t, uint32_t nt) {
         const uint64_t c0 = (uint64_t)wi * SBW;
-        const uint32_t b0 = wi * SBWB;
         for (uint32_t i = t; i < SBW; i += nt)
             if (c0 + i < n) wc[buf][i] = A.cand[c0 + i];
-        for (uint32_t i = t; i <= SBWB; i += nt) {
-            const int64_t bb = (int64_t)b0 + (int64_t)i - 1;
-            wx[buf][i] = (bb >= 0 && bb < (int64_t)nb) ? A.spec_exit[bb] : 0ull;
-        }
-        for (uint32_t i = t; i < SBWB; i += nt)
-            if (b0 + i < nb) {
-                wn[buf][i] = (uint64_t)((int64_t)A.spec_cnt[b0 + i] + A.delta[b0 + i]);
-                wo[buf][i] = A.ok[b0 + i];
-            }
     };
     if (nwin) stage(0, 0, tid, blockDim.x);
     __syncthreads();
-    const uint32_t lane = tid;
+    const uint32_t lane = tid & 31;
     uint64_t s = aux->s, off = base0;
     int held = 0;
     for (uint32_t wi = 0; wi < nwin; ++wi) {
@@ -340,23 +342,19 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
         if (tid >= 32) {
             if (wi + 1 < nwin) stage(wi + 1, cur ^ 1, tid - 32, blockDim.x - 32);
         } else {
-            const uint32_t b0 = wi * SBWB, mb = min(SBWB, nb - b0);
             const uint64_t c0 = (uint64_t)wi * SBW;
-            for (uint32_t j = 0; j < mb; ++j) {
-                const uint32_t b = b0 + j;
-                const uint64_t first = (uint64_t)b * SB_B, last = min(n, first + SB_B);
-                if (lane == 0) { A.entry[b] = s; A.offs[b] = off; }
-                if (b == 0 || (wo[cur][j] && s == wx[cur][j])) {
-                    off += wn[cur][j];
-                    s = wx[cur][j + 1];
-                    held = (!A.fin && last == n && A.cand[n - 1] == A.end && s == A.end) ? 1 : 0;
-                } else {
-                    held = 0;
-                    const uint32_t m = (uint32_t)(last - first);
-                    const uint64_t mine = lane < m ? wc[cur][first - c0 + lane] : 0ull;
-                    uint32_t from = 0;
+            const uint32_t m = (uint32_t)min((uint64_t)SBW, n - c0);
+            for (uint32_t w0 = 0; w0 < m; w0 += 32) {
+                const uint64_t mine = w0 + lane < m ? wc[cur][w0 + lane] : 0ull;
+#pragma unroll
+                for (uint32_t half = 0; half < 2; ++half) {
+                    const uint32_t lo = 16u * half, hi = min(lo + 16u, m - w0);
+                    if (lo >= hi) break;
+                    const uint64_t b = (c0 + w0 + lo) / SB_B;
+                    if (lane == 0) { A.entry[b] = s; A.offs[b] = off; }
+                    uint32_t from = lo;
                     for (;;) {
-                        const bool ev = lane >= from && lane < m &&
+                        const bool ev = lane >= from && lane < hi &&
                                         ((A.maxsz && mine - s > A.maxsz) || mine - s >= A.minsz);
                         const uint32_t bal = __ballot_sync(0xffffffffu, ev);
                         if (!bal) break;
