@@ -194,7 +194,7 @@ def oracle_steps(samples, steps: int, cores: int):
     return tot, time.perf_counter() - t0, per
 
 
-def cpu_measurements(runs: int = 3) -> dict:
+def cpu_measurements(runs: int = 5) -> dict:
     """The host-core baselines, measured in a FRESH process with no CUDA context (bench.py
     --cpu-only, started before the parent touches the GPU): the oracle (R2, all cores) on the same
     bounded sample and with the same timing code as the reference arm (`oracle_samples`,
@@ -207,7 +207,7 @@ def cpu_measurements(runs: int = 3) -> dict:
     cores = sorted(os.sched_getaffinity(0))
     nc = len(cores)
     n, samples = oracle_samples(1, nc)
-    oracle_steps(samples, 1, nc)                            # warm-up step (as the reference arm's)
+    oracle_steps(samples, 3, nc)                            # warm-up steps (the reference arm: W >= 3)
     tot, dt, per = oracle_steps(samples, 2 * runs, nc)
     rate1, dt1, _ = oracle_rate(samples[0][: 8 << 20], 1)
     out = {"cpu_baseline": {
