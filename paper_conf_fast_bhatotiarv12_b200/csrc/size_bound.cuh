@@ -546,7 +546,10 @@ constexpr size_t SBO_SMEM = (size_t)SBO_SMEM_N * 8 + (size_t)SBO_THREADS * 8 * 4
 #define SHRED_SB_ONE_MAX (256ull << 20)  // A/B: 0 = always the multi-CTA chain
 #endif
 constexpr uint64_t SB_ONE_MAX_LEN = SHRED_SB_ONE_MAX;
-constexpr uint64_t SB_ONE_EXPECT = 6144;  // expected candidates (len (r+1 | 1) / D) up to which sb_one runs
+#ifndef SHRED_SB_ONE_EXPECT
+#define SHRED_SB_ONE_EXPECT 8192   // 64 MiB at D = 8 KiB (A/B: sb_one 56.6 vs chain 68.8 us; 256 MiB: 253 vs 181)
+#endif
+constexpr uint64_t SB_ONE_EXPECT = SHRED_SB_ONE_EXPECT;  // expected candidates (len (r+1 | 1) / D) up to which sb_one runs
 
 __device__ __forceinline__ void sb_one_smem(const SBArgs &A, uint32_t n, uint64_t *n_out, uint64_t cap,
                                             bool loaded = false) {
