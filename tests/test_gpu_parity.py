@@ -650,8 +650,11 @@ def test_bounded_one_shot_one_cta_paths(pkg, kind):
 
 @pytest.mark.parametrize("mn,mx", [(8192, 65536), (65536, 0), (131072, 262144), (40000, 40001)])
 def test_bounded_min_above_d_serial_walk(pkg, mn, mx):
-    """min >= D: blocks of 16 candidates rarely re-sync with their speculation, so the size rule
-    takes its exact serial walk (batched block results, ballot re-walks); equal to the oracle
-    (L259-L265) on 64 MiB of random data, with and without forced cuts."""
-    data = synthgen.random_bytes(91, (64 << 20) + 333)
-    check_chunk(pkg.Chunker(pkg.Params(min_size=mn, max_size=mx)), data)
+    """min >= D: blocks of 16 candidates often fail to re-sync with their speculation, so the size
+    rule runs its repair passes (super-blocks of 1 and 32 blocks) and, when they do not converge
+    (min >~ 16D), its ballot walk; equal to the oracle (L259-L265) on 80 MiB of random data, with
+    and without forced cuts, and on 6 MiB (the one-CTA form)."""
+    data = synthgen.random_bytes(91, (80 << 20) + 333)       # > 8,192 expected candidates: the multi-CTA rule
+    ch = pkg.Chunker(pkg.Params(min_size=mn, max_size=mx))
+    check_chunk(ch, data)
+    check_chunk(ch, data[: (6 << 20) + 5])                  # few candidates: sb_one (shared-memory form)
