@@ -104,20 +104,22 @@ __device__ __forceinline__ void sb_spec_body(const SBArgs &A, uint32_t bid, uint
     bool synced = true;
     if (b < nb) {
         const uint64_t first = b * SB_B, last = min(n, first + SB_B);
-        uint64_t v[SB_B];
+        uint64_t v[SB_B], w[SB_B];
         uint64_t X = 0;
         int hX = 0;
-        if (b) {                              // speculation of block b-1 (its guess, or exact for 0)
-            const uint64_t pf = first - SB_B;
-#pragma unroll
-            for (int j = 0; j < SB_B; ++j) v[j] = A.cand[pf + j];
-            X = (b - 1) ? A.cand[pf - 1] : A.aux->s;
-#pragma unroll
-            for (int j = 0; j < SB_B; ++j) sb_step(X, v[j], A, hX, NoEmit{});
-        }
+        // both blocks' candidates in one round trip (the previous block's for its speculation)
 #pragma unroll
         for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
-        uint64_t sg = b ? A.cand[first - 1] : A.aux->s;       // this block's guess
+        const uint64_t pf = b ? first - SB_B : 0;
+#pragma unroll
+        for (int j = 0; j < SB_B; ++j) w[j] = b ? A.cand[pf + j] : 0ull;
+        const uint64_t s0 = A.aux->s;
+        X = (b > 1) ? A.cand[pf - 1] : s0;
+        if (b) {                              // speculation of block b-1 (its guess, or exact for 0)
+#pragma unroll
+            for (int j = 0; j < SB_B; ++j) sb_step(X, w[j], A, hX, NoEmit{});
+        }
+        uint64_t sg = b ? w[SB_B - 1] : s0;   // this block's guess: the previous candidate accepted
         int hg = 0, ht = 0;
         uint64_t cg = 0;
         int64_t ct = 0, cg_sync = 0;
@@ -395,6 +397,11 @@ __device__ __forceinline__ void sb_emit_body(const SBArgs &A, uint32_t bid, uint
     for (uint64_t tile = bid; tile * T <= nb; tile += nblk) {
         const uint64_t b = tile * T + threadIdx.x;
         uint64_t s = 0, o = 0;
+        // the block's candidates first: their round trip overlaps the offset scan below
+        const uint64_t first = b * SB_B, last = b < nb ? min(n, first + SB_B) : first;
+        uint64_t v[SB_B];
+#pragma unroll
+        for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
         if (fast) {
             // entry = the previous block's spec exit; offset = tile offset + in-tile exclusive prefix
             const uint64_t v = b < nb ? (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]) : 0ull;
@@ -423,10 +430,6 @@ __device__ __forceinline__ void sb_emit_body(const SBArgs &A, uint32_t bid, uint
             for (uint64_t j = 1; j <= mt; ++j) emit(s + j * A.maxsz);
             continue;
         }
-        const uint64_t first = b * SB_B, last = min(n, first + SB_B);
-        uint64_t v[SB_B];
-#pragma unroll
-        for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
         int held = 0;
 #pragma unroll
         for (int j = 0; j < SB_B; ++j)
