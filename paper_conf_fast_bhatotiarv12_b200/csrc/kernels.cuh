@@ -28,6 +28,19 @@
 #include <cstdint>
 #include <cuda.h>
 #include <cuda_runtime.h>
+#include <cassert>
+
+// Device-side bounds checks (the pool closed compute-sanitizer in round 2): a -DSHRED_DEBUG=1
+// build (libshred_debug.so, tools/debug_build.py) asserts the index and address invariants of the
+// round-2 code paths; the GPU test suite runs against it.  Compiled out otherwise.
+#ifndef SHRED_DEBUG
+#define SHRED_DEBUG 0
+#endif
+#if SHRED_DEBUG
+#define SHRED_ASSERT(c) assert(c)
+#else
+#define SHRED_ASSERT(c) ((void)0)
+#endif
 
 #ifndef SHRED_PRODUCER_SLEEP_NS
 #define SHRED_PRODUCER_SLEEP_NS 512
@@ -973,6 +986,7 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const __grid_constant__ CUtens
         act[ch] = row < J.map.nrows;
         pos0[ch] = J.map.b0 + (uint64_t)row * J.map.S;
         o[ch].lst = J.scratch + (uint64_t)(J.map.n_head + row) * J.cap;
+        SHRED_ASSERT(!act[ch] || J.map.n_head + row < J.map.n_head + J.map.nrows);
         o[ch].cnt = 0; o[ch].cap = J.cap;
     }
     {
@@ -1038,6 +1052,8 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const __grid_constant__ CUtens
             // warm-up's first e bytes (e = 16*wa - w), i.e. the funnel of (zero, first chunk).
             uint4 first[CH], nxt[CH];
             auto wload = [&](int ch, uint32_t k) {     // warm-up chunk k of chain ch
+                SHRED_ASSERT(!act[ch] || (pos0[ch] >= J.p_begin + 16ull * K.wa &&
+                                          pos0[ch] + 16ull * k + 16u <= J.map.t_end + 16ull * K.wa));
                 return act[ch] ? __ldg(reinterpret_cast<const uint4 *>(
                                      J.src + (pos0[ch] - 16ull * K.wa + 16ull * k - J.p_begin)))
                                : Z;
@@ -1097,9 +1113,12 @@ k1_bulk(const __grid_constant__ CUtensorMap tmap, const __grid_constant__ CUtens
                     // same bytes from global memory (the row's own data, 16*wa - S + ... behind)
 #pragma unroll
                     for (int ch = 0; ch < CH; ++ch)
-                        if (act[ch])
+                        if (act[ch]) {
+                            SHRED_ASSERT(pos0[ch] + (uint64_t)nrounds * ROUND <= J.map.b0 + (uint64_t)J.map.nrows * J.map.S &&
+                                         pos0[ch] + (uint64_t)nrounds * ROUND >= J.p_begin + 16ull * K.wa);
                             PQ[ch][CPR] = __ldg(reinterpret_cast<const uint4 *>(
                                 J.src + (pos0[ch] + (uint64_t)nrounds * ROUND - 16ull * K.wa - J.p_begin)));
+                        }
                 }
             }
             __syncwarp();

@@ -241,6 +241,7 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
         if (lvl > 0 && ns < 4) break;                           // no parallelism left: walk
         uint64_t *Ea = A.entry, *Eb = A.cta_sum, *Cn = A.cta_ok, *Used = A.offs;   // scratch
         const uint32_t T = blockDim.x, ps = (ns + T - 1) / T;
+        SHRED_ASSERT(ns <= nb + 1 && nb + 1 <= A.n_cap / SB_B + 2);
         const uint32_t sa = min(ns, tid * ps), se = min(ns, sa + ps);
         for (uint32_t k = sa; k < se; ++k) { Ea[k] = A.spec_exit[min(nb, (k + 1) * G) - 1]; Used[k] = ~0ull; }
         __syncthreads();
@@ -353,6 +354,7 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
                     const uint32_t lo = 16u * half, hi = min(lo + 16u, m - w0);
                     if (lo >= hi) break;
                     const uint64_t b = (c0 + w0 + lo) / SB_B;
+                    SHRED_ASSERT(b < nb && w0 + 32 <= SBW + 32);
                     if (lane == 0) { A.entry[b] = s; A.offs[b] = off; }
                     uint32_t from = lo;
                     for (;;) {
@@ -565,6 +567,7 @@ __device__ __forceinline__ void sb_one_smem(const SBArgs &A, uint32_t n, uint64_
     __shared__ uint32_t okb[SBO_THREADS];
     __shared__ uint64_t wsum[SBO_THREADS / 32 + 1];
     const uint32_t tid = threadIdx.x;
+    SHRED_ASSERT(n <= SBO_SMEM_N - SBO_B && blockDim.x == SBO_THREADS);
     if (!loaded)
         for (uint32_t i = tid; i < n; i += SBO_THREADS) sc[i] = A.cand[i];
     __syncthreads();
