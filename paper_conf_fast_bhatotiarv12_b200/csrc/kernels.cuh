@@ -1217,7 +1217,7 @@ constexpr int MAX_GROUPS = 4096;
 __global__ void __launch_bounds__(SCATTER_THREADS)
 k_scatter(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots,
           uint64_t *__restrict__ dst, uint64_t dst_cap, Aux *aux, int streaming,
-          uint64_t *n_direct) {
+          uint64_t *n_direct, int reset) {
     pdl_entry();
     __shared__ uint64_t gbase[MAX_GROUPS];
     __shared__ uint64_t wsum[SCATTER_THREADS / 32 + 1];
@@ -1260,6 +1260,10 @@ k_scatter(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots,
     }
     const uint64_t total = carry;
     if (blockIdx.x == 0 && tid == 0) {
+        if (reset) {                          // a one-shot bounded call: its size-rule state (no
+            aux->s = 0; aux->held = 0;         // block reads it here: streaming == 0)
+            aux->held_val = 0; aux->out_pos = 0;
+        }
         aux->total = total;
         aux->ncand = total;
         aux->dense = total > dst_cap ? 1ull : 0ull;
@@ -1324,8 +1328,9 @@ __global__ void k_stream_reset(Aux *aux) {
 
 // A piece with no window ends: no candidates (the count the size rule reads, the dense flag and
 // the caller's count if given).
-__global__ void k_no_slots(Aux *aux, uint64_t *n_direct) {
+__global__ void k_no_slots(Aux *aux, uint64_t *n_direct, int reset) {
     pdl_entry();
+    if (reset) { aux->s = 0; aux->held = 0; aux->held_val = 0; aux->out_pos = 0; }
     aux->total = 0; aux->ncand = 0; aux->dense = 0;
     if (n_direct) *n_direct = 0;
 }

@@ -538,14 +538,14 @@ int launch_detect(shred_ctx *ctx, Plan &pl, cudaStream_t st) {
 
 // Ordered compaction into dst.  With no slots: total = 0 (and *n_direct = 0).
 int launch_scatter(shred_ctx *ctx, Plan &pl, uint64_t *dst, uint64_t dst_cap, Aux *aux, int streaming,
-                   uint64_t *n_direct, cudaStream_t st) {
+                   uint64_t *n_direct, cudaStream_t st, int reset = 0) {
     if (pl.nslots == 0) {
-        PDL(k_no_slots, 1, 1, 0, st, aux, n_direct);
+        PDL(k_no_slots, 1, 1, 0, st, aux, n_direct, reset);
         LAUNCHED("k_no_slots");
         return SHRED_OK;
     }
     PDL(k_scatter, (pl.nslots + SCATTER_THREADS - 1) / SCATTER_THREADS, SCATTER_THREADS, 0, st, 
-        pl.J, ctx->dp, ctx->d_gen, pl.nslots, dst, dst_cap, aux, streaming, n_direct);
+        pl.J, ctx->dp, ctx->d_gen, pl.nslots, dst, dst_cap, aux, streaming, n_direct, reset);
     LAUNCHED("k_scatter");
     return SHRED_OK;
 }
@@ -558,7 +558,7 @@ bool bounded(const shred_ctx *ctx) { return ctx->p.min_size > 0 || ctx->p.max_si
 // runs only if the ordered list could not hold every candidate.
 int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_dev, uint64_t n_host,
                       uint64_t nmax, uint64_t end, int fin, uint64_t *dst, uint64_t cap, Aux *aux,
-                      const Plan *pl, cudaStream_t st) {
+                      const Plan *pl, cudaStream_t st, uint64_t *n_out = nullptr) {
     const uint64_t nb = (nmax + SB_B - 1) / SB_B;
     int rc = grow(ctx, ctx->d_sb, ctx->sb_cap, 9 * (nb + 2), "size-rule scratch");
     if (rc) return rc;
@@ -569,7 +569,7 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
     A.spec_exit = b; A.spec_cnt = b + (nb + 2); A.entry = b + 2 * (nb + 2); A.offs = b + 3 * (nb + 2);
     A.delta = (int64_t *)(b + 4 * (nb + 2)); A.ok = (uint32_t *)(b + 5 * (nb + 2));
     A.cta_sum = b + 6 * (nb + 2); A.cta_ok = b + 7 * (nb + 2); A.cta_off = b + 8 * (nb + 2);
-    A.dst = dst; A.dst_cap = cap; A.aux = aux; A.tile = SB_THREADS;
+    A.dst = dst; A.dst_cap = cap; A.aux = aux; A.tile = SB_THREADS; A.n_out = n_out;
     // tiles of SB_THREADS blocks, at most 8 CTAs per SM (grid-stride over the true tile count)
     const uint64_t gmax = (uint64_t)ctx->sm_count * 8;
     uint64_t g = (nb + SB_THREADS - 1) / SB_THREADS;
@@ -922,12 +922,13 @@ int shred_chunk(shred_ctx *ctx, const uint8_t *d_in, uint64_t len, uint64_t *d_o
     if (SB_ONE_MAX_LEN && len <= SB_ONE_MAX_LEN &&
         (long double)len * (long double)hits_per_d(ctx->p) / (long double)ctx->p.divisor <= (long double)SB_ONE_EXPECT)
         return chunk_bounded_one(ctx, pl, len, d_out, cap, n_out, st);
-    PDL(k_stream_reset, 1, 1, 0, st, aux);
-    LAUNCHED("k_stream_reset");
-    if ((rc = run_piece(ctx, aux, d_in, 0, nullptr, 0, 0, len, len, 1, d_out, cap, st))) return rc;
-    PDL(k_call_end, 1, 1, 0, st, aux, n_out, cap, nullptr);
-    LAUNCHED("k_call_end");
-    return SHRED_OK;
+    // the multi-CTA chain: k_scatter resets the size-rule state, the rule's last kernel writes
+    // the count (no k_stream_reset / k_call_end launches)
+    if ((rc = launch_detect(ctx, pl, st))) return rc;
+    const uint64_t ccap = (uint64_t)pl.nslots * pl.J.cap + 1;
+    if ((rc = grow(ctx, ctx->d_cand, ctx->cand_cap, ccap, "candidate list"))) return rc;
+    if ((rc = launch_scatter(ctx, pl, ctx->d_cand, ccap, aux, 0, nullptr, st, 1))) return rc;
+    return launch_size_bound(ctx, ctx->d_cand, &aux->ncand, 0, ccap, len, 1, d_out, cap, aux, &pl, st, n_out);
 }
 
 int shred_candidates_range(shred_ctx *ctx, const uint8_t *d_in, uint64_t halo, uint64_t start,

@@ -55,7 +55,15 @@ struct SBArgs {
     uint64_t *dst; uint64_t dst_cap;
     Aux *aux;                       // s, held, held_val, out_pos (streaming state)
     uint32_t tile;                  // blocks per tile = the threads of the CTA running the phases
+    uint64_t *n_out;                // one-shot chain: the caller's count, written with the final state
 };
+// The call end of a one-shot chain (k_call_end's job) where the final state is written.
+__device__ __forceinline__ void sb_call_end(const SBArgs &A) {
+    if (A.n_out) {
+        *A.n_out = A.aux->out_pos;
+        if (A.aux->out_pos > A.dst_cap) A.aux->overflow = 1;
+    }
+}
 
 __device__ __forceinline__ uint64_t sb_n(const SBArgs &A) {
     if (!A.n_dev) return A.n_host;
@@ -219,6 +227,7 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
             aux->held_val = held_new ? A.end : 0;
             aux->total = carry + mt;
             aux->sb_fast = 1;
+            sb_call_end(A);
             A.offs[nb] = base0 + carry;           // the tail's forced cuts start here
             A.entry[nb] = s_last;
         }
@@ -317,6 +326,7 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
             aux->s = s_last + mt * A.maxsz;
             aux->held = (uint64_t)held_new;
             aux->held_val = held_new ? A.end : 0;
+            sb_call_end(A);
         }
         return;
     }
@@ -382,6 +392,7 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
     aux->s = s + mt * A.maxsz;
     aux->held = (uint64_t)held;
     aux->held_val = held ? A.end : 0;
+    sb_call_end(A);
 }
 __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
     pdl_entry();
@@ -517,6 +528,7 @@ __device__ __forceinline__ void sb_dense_body(const Job &J, const DevParams &P, 
         aux->s = s + mt * A.maxsz;
         aux->held = (uint64_t)held;
         aux->held_val = held ? A.end : 0;
+        sb_call_end(A);
     }
 }
 __global__ void __launch_bounds__(SBD_THREADS)
