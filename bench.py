@@ -110,12 +110,15 @@ class ClockSampler:
         nv = self.nv
         get_r = getattr(nv, "nvmlDeviceGetCurrentClocksEventReasons", None) or \
             nv.nvmlDeviceGetCurrentClocksThrottleReasons
+        k = 0
         while not self._stop.is_set():
             try:
                 self.samples.append(nv.nvmlDeviceGetClockInfo(self.h, nv.NVML_CLOCK_SM))
-                self.reasons |= int(get_r(self.h))
+                if k % 4 == 0:                 # the reasons query is the slower call on some boxes
+                    self.reasons |= int(get_r(self.h))
             except Exception:
                 pass
+            k += 1
             time.sleep(0.0005)
 
     def __enter__(self):
