@@ -86,11 +86,13 @@ enum { SHRED_MARKER_EQ = 0, SHRED_MARKER_LE = 1 };
 
 /* Kernel paths the ctx selected for its parameters (shred_path). */
 enum {
-    SHRED_PATH_K63     = 1, /* deg(P) in 33..63 (the paper's reading: 63), 1 <= w <= 64, any
-                               valid D and marker set (marker kinds below): u64 state,
-                               TMA-staged, smem LDS.64 tables                                   */
+    SHRED_PATH_K63     = 1, /* deg(P) in 33..63 (the paper's reading: 63), 1 <= w <= 4096 (w > 64:
+                               the bytes leaving the window from a second TMA tile), any valid D
+                               and marker set (marker kinds below): u64 state, TMA-staged, smem
+                               LDS.64 tables                                                    */
     SHRED_PATH_K32     = 2, /* deg(P) in 8..32, same w / D / marker conditions: u32 state, LDS.32 */
-    SHRED_PATH_GENERIC = 3  /* any other valid parameters (w > 64): byte-at-a-time             */
+    SHRED_PATH_GENERIC = 3  /* any other valid parameters: byte-at-a-time (the hot paths also use
+                               the byte loop for inputs below 4 KiB and for their edge segments) */
 };
 
 /* Fill *p with the paper defaults (readings Q1, Q5, Q6, Q15): P = 0xbfe6b8a5bf378d83, w = 48,
@@ -248,7 +250,7 @@ int shred_check_params(const shred_params *p, int *path_out, int *marker_kind_ou
 /* Test hook (no device needed): the slot map planning would use for window ends [t_begin, t_end)
    of a job whose bytes start at stream position p_begin at address src_addr, for kernel path
    `path` (SHRED_PATH_*), with (small_ok) or without the small-input launch shape, on sm_count SMs,
-   for a window of `window` bytes (1..64: the fast paths), zero_lead = 1 if the job starts at the
+   for a window of `window` bytes (1..4096; > 64 never plans a zero lead), zero_lead = 1 if the job starts at the
    stream start with no carried prefix (rows may then start at the stream start itself).
    out[16] = {bulk, small, head_start, head_seg, n_head, b0, S, nrows, tail_start, tail_seg,
    n_tail, bulk CTAs, slot groups, rows per CTA, per-slot list capacity for `divisor`, threads per
