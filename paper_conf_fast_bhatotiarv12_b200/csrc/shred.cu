@@ -559,7 +559,11 @@ bool bounded(const shred_ctx *ctx) { return ctx->p.min_size > 0 || ctx->p.max_si
 int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_dev, uint64_t n_host,
                       uint64_t nmax, uint64_t end, int fin, uint64_t *dst, uint64_t cap, Aux *aux,
                       const Plan *pl, cudaStream_t st, uint64_t *n_out = nullptr) {
-    const uint64_t nb = (nmax + SB_B - 1) / SB_B;
+    // blocks of 8 candidates when min <= half the mean candidate gap (D / h), else 16 (size_bound.cuh)
+    const bool small_b = (long double)ctx->p.min_size * 2.0L * (long double)hits_per_d(ctx->p) <=
+                         (long double)ctx->p.divisor;
+    const int B = small_b ? SB_B_SMALL : SB_B;
+    const uint64_t nb = (nmax + B - 1) / B;
     int rc = grow(ctx, ctx->d_sb, ctx->sb_cap, 9 * (nb + 2), "size-rule scratch");
     if (rc) return rc;
     SBArgs A;
@@ -575,14 +579,17 @@ int launch_size_bound(shred_ctx *ctx, const uint64_t *cand, const uint64_t *n_de
     uint64_t g = (nb + SB_THREADS - 1) / SB_THREADS;
     if (g > gmax) g = gmax;
     if (nb) {
-        PDL(sb_spec_check, (unsigned)g, SB_THREADS, 0, st, A);
+        if (small_b) { PDL(sb_spec_check<SB_B_SMALL>, (unsigned)g, SB_THREADS, 0, st, A); }
+        else         { PDL(sb_spec_check<SB_B>, (unsigned)g, SB_THREADS, 0, st, A); }
         LAUNCHED("sb_spec_check");
     }
-    PDL(sb_plan, 1, 1024, 0, st, A);
+    if (small_b) { PDL(sb_plan<SB_B_SMALL>, 1, 1024, 0, st, A); }
+    else         { PDL(sb_plan<SB_B>, 1, 1024, 0, st, A); }
     LAUNCHED("sb_plan");
     uint64_t ge = (nb + 1 + SB_THREADS - 1) / SB_THREADS;
     if (ge > gmax) ge = gmax;
-    PDL(sb_emit, (unsigned)ge, SB_THREADS, 0, st, A);
+    if (small_b) { PDL(sb_emit<SB_B_SMALL>, (unsigned)ge, SB_THREADS, 0, st, A); }
+    else         { PDL(sb_emit<SB_B>, (unsigned)ge, SB_THREADS, 0, st, A); }
     LAUNCHED("sb_emit");
     if (pl && pl->nslots) {
         uint64_t maxseg = pl->J.map.S;

@@ -28,16 +28,18 @@
 
 namespace shred {
 
+// Block size B (candidates per speculative block, one thread each).  A block syncs at its first
+// candidate c >= g + min (g = its guessed entry; accepted from the true entry s <= g too), so it
+// fails only if all B candidates lie within min of g (~P(Poisson(min/D) >= B) on random data); the
+// repair passes then fix the chain.  B = 8 (twice the threads, half the chain) is faster when
+// min <= D/2 (1 GiB at the LBFS bounds 561 -> 552 us, 256 MiB 175 -> 164 us); at min >= D its
+// repairs need more passes (min = D 0.78 -> 0.93 ms), so B = 16 there (launch_size_bound picks).
+// A/B log: profiles/r02_ab_small_bounded.txt.
 #ifndef SHRED_SB_B
-// 16: a block syncs at its first candidate c >= g + min (g = its guessed entry; accepted from the
-// true entry s <= g too), so it fails only if all B candidates lie within min of g: P(Poisson(min/D)
-// >= B) for random data, and one unsynced block sends the whole list to the serial walk.  B = 16
-// keeps that negligible up to min ~ 3D on GiB lists; A/B (profiles/r02_ab_small_bounded.txt): 8
-// gained ~1 % at min = D/4 but walks on ~15 % of GiB lists at min = D; 4 walked on every call
-// at min = D/4 (103 GB/s).
 #define SHRED_SB_B 16
 #endif
-constexpr int SB_B = SHRED_SB_B;    // candidates per block (one thread; prefetched into registers)
+constexpr int SB_B = SHRED_SB_B;      // the large-min / one-CTA block size
+constexpr int SB_B_SMALL = 8;         // min <= D/2
 constexpr int SB_THREADS = 128;
 
 struct SBArgs {
@@ -102,39 +104,40 @@ __device__ __forceinline__ uint64_t sb_tail_count(uint64_t s, const SBArgs &A) {
 // capacity bound, the tile count comes from the true count on the device).
 // The phases are device functions so that one CTA can run them back to back (sb_one): tiles of
 // A.tile = blockDim.x blocks, CTA `bid` of `nblk` takes tiles bid, bid + nblk, ...
+template <int B>
 __device__ __forceinline__ void sb_spec_body(const SBArgs &A, uint32_t bid, uint32_t nblk) {
     const uint64_t n = sb_n(A);
-    const uint64_t nb = (n + SB_B - 1) / SB_B;
+    const uint64_t nb = (n + B - 1) / B;
     const uint32_t T = blockDim.x;
     for (uint64_t tile = bid; tile * T < nb; tile += nblk) {
     const uint64_t b = tile * T + threadIdx.x;
     uint64_t cnt = 0;
     bool synced = true;
     if (b < nb) {
-        const uint64_t first = b * SB_B, last = min(n, first + SB_B);
-        uint64_t v[SB_B], w[SB_B];
+        const uint64_t first = b * B, last = min(n, first + B);
+        uint64_t v[B], w[B];
         uint64_t X = 0;
         int hX = 0;
         // both blocks' candidates in one round trip (the previous block's for its speculation)
 #pragma unroll
-        for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
-        const uint64_t pf = b ? first - SB_B : 0;
+        for (int j = 0; j < B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
+        const uint64_t pf = b ? first - B : 0;
 #pragma unroll
-        for (int j = 0; j < SB_B; ++j) w[j] = b ? A.cand[pf + j] : 0ull;
+        for (int j = 0; j < B; ++j) w[j] = b ? A.cand[pf + j] : 0ull;
         const uint64_t s0 = A.aux->s;
         X = (b > 1) ? A.cand[pf - 1] : s0;
         if (b) {                              // speculation of block b-1 (its guess, or exact for 0)
 #pragma unroll
-            for (int j = 0; j < SB_B; ++j) sb_step(X, w[j], A, hX, NoEmit{});
+            for (int j = 0; j < B; ++j) sb_step(X, w[j], A, hX, NoEmit{});
         }
-        uint64_t sg = b ? w[SB_B - 1] : s0;   // this block's guess: the previous candidate accepted
+        uint64_t sg = b ? w[B - 1] : s0;   // this block's guess: the previous candidate accepted
         int hg = 0, ht = 0;
         uint64_t cg = 0;
         int64_t ct = 0, cg_sync = 0;
         synced = (b == 0) || (X == sg && hX == 0);
         uint64_t st = X;
 #pragma unroll
-        for (int j = 0; j < SB_B; ++j) {
+        for (int j = 0; j < B; ++j) {
             if (first + j < last) {
                 const uint64_t k = sb_step(sg, v[j], A, hg, NoEmit{});
                 cg += k;
@@ -167,18 +170,20 @@ __device__ __forceinline__ void sb_spec_body(const SBArgs &A, uint32_t bid, uint
     __syncthreads();                          // red reused by the next tile
     }
 }
+template <int B>
 __global__ void __launch_bounds__(SB_THREADS) sb_spec_check(SBArgs A) {
     pdl_entry();
     if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
-    sb_spec_body(A, blockIdx.x, gridDim.x);
+    sb_spec_body<B>(A, blockIdx.x, gridDim.x);
 }
 
 // One CTA: entries, offsets, totals and the streaming state.  Each thread owns a contiguous
 // range of blocks; one block scan of the range sums gives every block's offset.
+template <int B>
 __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
     __shared__ uint64_t wsum[33];
     const uint64_t n = sb_n(A);
-    const uint32_t nb = (uint32_t)((n + SB_B - 1) / SB_B);
+    const uint32_t nb = (uint32_t)((n + B - 1) / B);
     const uint32_t tid = threadIdx.x;
     const uint32_t nc = (nb + A.tile - 1) / A.tile;                 // tiles with blocks
     const uint32_t per = (nc + blockDim.x - 1) / blockDim.x;
@@ -250,7 +255,7 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
         if (lvl > 0 && ns < 4) break;                           // no parallelism left: walk
         uint64_t *Ea = A.entry, *Eb = A.cta_sum, *Cn = A.cta_ok, *Used = A.offs;   // scratch
         const uint32_t T = blockDim.x, ps = (ns + T - 1) / T;
-        SHRED_ASSERT(ns <= nb + 1 && nb + 1 <= A.n_cap / SB_B + 2);
+        SHRED_ASSERT(ns <= nb + 1 && nb + 1 <= A.n_cap / B + 2);
         const uint32_t sa = min(ns, tid * ps), se = min(ns, sa + ps);
         for (uint32_t k = sa; k < se; ++k) { Ea[k] = A.spec_exit[min(nb, (k + 1) * G) - 1]; Used[k] = ~0ull; }
         __syncthreads();
@@ -263,7 +268,7 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
             for (uint32_t k = sa; k < se; ++k) {
                 const uint64_t e = k ? src[k - 1] : aux->s;
                 if (e != Used[k]) {
-                    const uint64_t first = (uint64_t)k * G * SB_B, last = min(n, first + (uint64_t)G * SB_B);
+                    const uint64_t first = (uint64_t)k * G * B, last = min(n, first + (uint64_t)G * B);
                     uint64_t x = e;
                     int h = 0;
 #pragma unroll 4
@@ -286,7 +291,7 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
             uint64_t x = Used[k];
             int h = 0;
             for (uint32_t b = k * G; b < min(nb, (k + 1) * G); ++b) {
-                const uint64_t first = (uint64_t)b * SB_B, last = min(n, first + SB_B);
+                const uint64_t first = (uint64_t)b * B, last = min(n, first + B);
                 A.entry[b] = x;
                 uint64_t cnt = 0;
                 for (uint64_t j = first; j < last; ++j) cnt += sb_step(x, A.cand[j], A, h, NoEmit{});
@@ -333,10 +338,10 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
     // ---- sequential fallback (no parallel form converged): exact.  Warp 0 runs the rule over
     // every candidate in order, 32 at a time by ballot: the first candidate (in order) that
     // forces a cut or is accepted from the current state is the next one that changes it, and
-    // every candidate before it drops out with no effect -- one ballot per 16 candidates plus one
-    // step per cut.  Block entries and offsets are recorded at the block boundaries.  The other
+    // every candidate before it drops out with no effect -- one ballot per block of B
+    // candidates plus one step per cut.  Block entries and offsets are recorded at the block boundaries.  The other
     // warps stage the next window of candidates in shared memory (double-buffered).
-    static_assert(SB_B == 16, "the ballot walk records a block boundary every 16 candidates");
+    static_assert(32 % B == 0, "the ballot walk records a block boundary every B candidates");
     constexpr uint32_t SBW = 2048;                          // candidates per window
     __shared__ uint64_t wc[2][SBW];
     const uint32_t nwin = (uint32_t)((n + SBW - 1) / SBW);
@@ -360,10 +365,10 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
             for (uint32_t w0 = 0; w0 < m; w0 += 32) {
                 const uint64_t mine = w0 + lane < m ? wc[cur][w0 + lane] : 0ull;
 #pragma unroll
-                for (uint32_t half = 0; half < 2; ++half) {
-                    const uint32_t lo = 16u * half, hi = min(lo + 16u, m - w0);
+                for (uint32_t part = 0; part < 32u / B; ++part) {
+                    const uint32_t lo = B * part, hi = min(lo + (uint32_t)B, m - w0);
                     if (lo >= hi) break;
-                    const uint64_t b = (c0 + w0 + lo) / SB_B;
+                    const uint64_t b = (c0 + w0 + lo) / B;
                     SHRED_ASSERT(b < nb && w0 + 32 <= SBW + 32);
                     if (lane == 0) { A.entry[b] = s; A.offs[b] = off; }
                     uint32_t from = lo;
@@ -394,16 +399,18 @@ __device__ __forceinline__ void sb_plan_body(const SBArgs &A) {
     aux->held_val = held ? A.end : 0;
     sb_call_end(A);
 }
+template <int B>
 __global__ void __launch_bounds__(1024) sb_plan(SBArgs A) {
     pdl_entry();
     if (A.aux->dense) return;
-    sb_plan_body(A);
+    sb_plan_body<B>(A);
 }
 
 // Every block writes its cuts; thread nb writes the forced cuts after the last candidate.
+template <int B>
 __device__ __forceinline__ void sb_emit_body(const SBArgs &A, uint32_t bid, uint32_t nblk) {
     const uint64_t n = sb_n(A);
-    const uint64_t nb = (n + SB_B - 1) / SB_B;
+    const uint64_t nb = (n + B - 1) / B;
     const bool fast = A.aux->sb_fast != 0;
     const uint32_t T = blockDim.x;
     __shared__ uint64_t ws[33];
@@ -411,10 +418,10 @@ __device__ __forceinline__ void sb_emit_body(const SBArgs &A, uint32_t bid, uint
         const uint64_t b = tile * T + threadIdx.x;
         uint64_t s = 0, o = 0;
         // the block's candidates first: their round trip overlaps the offset scan below
-        const uint64_t first = b * SB_B, last = b < nb ? min(n, first + SB_B) : first;
-        uint64_t v[SB_B];
+        const uint64_t first = b * B, last = b < nb ? min(n, first + B) : first;
+        uint64_t v[B];
 #pragma unroll
-        for (int j = 0; j < SB_B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
+        for (int j = 0; j < B; ++j) v[j] = (first + j < last) ? A.cand[first + j] : 0ull;
         if (fast) {
             // entry = the previous block's spec exit; offset = tile offset + in-tile exclusive prefix
             const uint64_t v = b < nb ? (uint64_t)((int64_t)A.spec_cnt[b] + A.delta[b]) : 0ull;
@@ -445,14 +452,15 @@ __device__ __forceinline__ void sb_emit_body(const SBArgs &A, uint32_t bid, uint
         }
         int held = 0;
 #pragma unroll
-        for (int j = 0; j < SB_B; ++j)
+        for (int j = 0; j < B; ++j)
             if (first + j < last) sb_step(s, v[j], A, held, emit);
     }
 }
+template <int B>
 __global__ void __launch_bounds__(SB_THREADS) sb_emit(SBArgs A) {
     pdl_entry();
     if (A.aux->dense) return;                 // the candidates did not fit: sb_dense runs
-    sb_emit_body(A, blockIdx.x, gridDim.x);
+    sb_emit_body<B>(A, blockIdx.x, gridDim.x);
 }
 
 // ------------------------------------------------------------------------------ sb_dense
@@ -685,11 +693,11 @@ sb_one(Job J, DevParams P, const GenTables *__restrict__ gt, uint32_t nslots, SB
     if (dense) {
         sb_dense_body(J, P, gt, nslots, A);
     } else {
-        sb_spec_body(A, 0, 1);
+        sb_spec_body<SB_B>(A, 0, 1);
         __syncthreads();
-        sb_plan_body(A);
+        sb_plan_body<SB_B>(A);
         __syncthreads();
-        sb_emit_body(A, 0, 1);
+        sb_emit_body<SB_B>(A, 0, 1);
     }
     __syncthreads();
     if (threadIdx.x == 0) {
