@@ -166,15 +166,18 @@ def test_virtual_shards_concatenate_to_chunk(pkg, G):
     assert np.array_equal(cuts.astype(np.uint64), oracle.size_bound(exp, n, 256, 8192))
 
 
-def test_size_bound_state_chains_over_virtual_shards(pkg):
+@pytest.mark.parametrize("mn,mx", [(256, 8192), (4096, 65536), (16384, 0)])
+def test_size_bound_state_chains_over_virtual_shards(pkg, mn, mx):
     """shred_size_bound_state: chaining the rule over shard ranges through the exit states equals
-    the whole-stream rule (the per-rank step of the distributed size rule, f1)."""
+    the whole-stream rule (the per-rank step of the distributed size rule, f1); min < D (blocks
+    of 8), min = 4D (repair passes) and min = 16D (the serial walk), with held cuts at the
+    shard ends."""
     n = (9 << 20) + 321
     data = synthgen.random_bytes(17, n)
-    p = pkg.Params(divisor=1024, min_size=256, max_size=8192)
+    p = pkg.Params(divisor=1024, min_size=mn, max_size=mx)
     ch = pkg.Chunker(p)
     cand = oracle.candidates(data, oracle.Params(divisor=1024)).astype(np.int64)
-    exp = oracle.size_bound(cand.astype(np.uint64), n, 256, 8192)
+    exp = oracle.size_bound(cand.astype(np.uint64), n, mn, mx)
     for G in (1, 3, 8):
         bounds = [n * g // G for g in range(G + 1)]
         s, held, got = 0, False, []
